@@ -1,0 +1,267 @@
+/*
+ * skl.h — C ABI of libskl.so, a B200-native (sm_100a) implementation of the
+ * data-parallel hot path of SkelCL (Steuwer & Gorlatch, "SkelCL: Enhancing
+ * OpenCL for High-Level Programming of Multi-GPU Systems", PaCT 2013;
+ * /root/reference/PAPER.md, cited as P:Lx-y).  Readings of passages the paper
+ * leaves open are numbered A<n> and listed in DESIGN.md §3.
+ *
+ * Conventions:
+ *  - Every call returns skl_status: SKL_OK (0) or a negative SKL_ERR_* code.
+ *    skl_last_error() returns a thread-local message (with the NVRTC log for
+ *    SKL_ERR_COMPILE).  Nothing here aborts the process.
+ *  - Handles are opaque and owned by the library.  The caller destroys
+ *    containers and skeletons; skl_finalize() frees everything still alive.
+ *  - A context is driven by one host thread, matching the paper's sequential
+ *    host program.
+ *  - Calls enqueue asynchronously on one stream per device.  Only calls that
+ *    hand data to the host (skl_copy_out, skl_host_data, skl_scalar_get,
+ *    skl_sync) wait.
+ *  - Pointers named `host` are host memory (pinned memory gives DMA speed);
+ *    pointers returned by skl_local_part are device memory, borrowed.
+ *  - There is no CPU fallback: every skeleton runs as CUDA kernels for
+ *    sm_100a, JIT-compiled with NVRTC from the user's source string.  Without a
+ *    usable GPU, skl_init returns SKL_ERR_CUDA.
+ */
+#ifndef SKL_H
+#define SKL_H
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef int skl_status;
+#define SKL_OK 0
+#define SKL_ERR_INVALID_ARG -1   /* bad handle, NULL pointer, bad enum value      */
+#define SKL_ERR_TYPE -2          /* element types do not fit the skeleton         */
+#define SKL_ERR_SIZE_MISMATCH -3 /* Zip inputs of different sizes    */
+#define SKL_ERR_EMPTY -4         /* Reduce / Scan of an empty vector (A11)        */
+#define SKL_ERR_COMPILE -5       /* NVRTC rejected the source; log in last_error  */
+#define SKL_ERR_OUT_OF_RANGE -6  /* debug bounds: get() beyond d (A21) */
+#define SKL_ERR_DISTRIBUTION -7  /* distribution request that cannot be honoured  */
+#define SKL_ERR_OOM -8           /* device or pinned-host allocation failed       */
+#define SKL_ERR_CUDA -9          /* CUDA runtime error (message in last_error)    */
+#define SKL_ERR_NCCL -10         /* NCCL error in multi-process mode              */
+#define SKL_ERR_UNSUPPORTED -11  /* feature not available (e.g. NCCL library)    */
+
+typedef struct skl_ctx skl_ctx;
+typedef struct skl_cont skl_cont;
+typedef struct skl_skel skl_skel;
+
+/* ------------------------------------------------------------------ types
+ * Element types of containers and of customising-function parameters.  The
+ * paper's examples use int, float, char and complex numbers (P:L156, P:L254,
+ * P:L468).  Struct element types (A27, LM OSEM events) are registered
+ * with skl_type_struct.  OR-ing SKL_PTR into an *extra-argument* type declares a
+ * container argument (the customising function receives `T*`).               */
+typedef int skl_type;
+#define SKL_VOID 0
+#define SKL_U8 1   /* uchar / unsigned char                                   */
+#define SKL_I8 2
+#define SKL_I32 3  /* int                                                     */
+#define SKL_U32 4  /* uint                                                    */
+#define SKL_F32 5  /* float                                                   */
+#define SKL_F64 6  /* double                                                  */
+#define SKL_F32X2 7 /* float2 (complex numbers, Mandelbrot P:L468)            */
+#define SKL_I64 8
+#define SKL_U64 9
+#define SKL_I16 10
+#define SKL_U16 11
+#define SKL_PTR 0x1000
+/* Register a struct type.  `name` is the C identifier used in sources,
+ * `decl_src` its definition (e.g. "struct Event { float x0,y0,z0,x1,y1,z1; };"),
+ * size/align as the C compiler lays it out.  The declaration is prepended to
+ * every program that uses the type.  Returns the new type id in *out.          */
+skl_status skl_type_struct(skl_ctx* ctx, const char* name, const char* decl_src, size_t size,
+                           size_t align, skl_type* out);
+skl_status skl_type_size(skl_ctx* ctx, skl_type t, size_t* size);
+
+/* ------------------------------------------------------------------ context
+ * SkelCL::init(): "the calculation specified by a skeleton is
+ * performed automatically on all GPUs available".
+ *
+ * skl_init: one process drives `ndev` devices.  devices[g] is the CUDA ordinal
+ * of logical device g; NULL means all visible GPUs (ndev = 0) or devices
+ * g % visible (ndev > 0).  Several logical devices may share one physical GPU
+ * ("logical-device mode"): each gets its own stream and its own
+ * memory, and data moves between them by device-to-device copies, so the whole
+ * distribution machinery runs on a 1-GPU box.
+ *
+ * skl_init_dist: one process per GPU (torchrun).  Global device g is rank g;
+ * `nccl_id` is the 128-byte ncclUniqueId from skl_nccl_unique_id() on rank 0,
+ * broadcast by the caller.  Exchanges between ranks use NCCL send/recv over
+ * NVLink (libnccl.so.2 is loaded on first use).  Every rank must issue the same
+ * sequence of calls (SPMD): host-visible results and redistributions are
+ * collective.                                                                  */
+skl_status skl_init(int ndev, const int* devices, skl_ctx** out);
+skl_status skl_init_dist(int rank, int world, int cuda_device, const void* nccl_id, skl_ctx** out);
+skl_status skl_nccl_unique_id(void* out128);
+skl_status skl_finalize(skl_ctx* ctx);
+skl_status skl_num_devices(skl_ctx* ctx, int* ndev, int* first_local, int* nlocal);
+/* Use the caller's stream (e.g. torch's current stream) for device g; NULL
+ * restores the library's own stream.  Only local devices.                      */
+skl_status skl_set_stream(skl_ctx* ctx, int g, void* cuda_stream);
+skl_status skl_get_stream(skl_ctx* ctx, int g, void** cuda_stream);
+skl_status skl_sync(skl_ctx* ctx);
+/* Options: "block_threads" (work-group size; default 256),
+ * "debug_bounds" (1 = get() range-checked, A21), "map_unroll" (chunks per
+ * thread, default 4).                                                          */
+skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
+/* Counters: "launches" (kernels this library launched), "compiles" (NVRTC runs),
+ * "cache_hits", "h2d_bytes", "d2h_bytes", "p2p_bytes" (device-to-device bytes). */
+skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value);
+const char* skl_last_error(void);
+
+/* ------------------------------------------------------------------ containers
+ * Vector<T> / Matrix<T>: "when a container is created on the CPU,
+ * memory is allocated on the GPUs automatically; when a container ... is
+ * deleted, the memory allocated on the GPUs is freed automatically".  A matrix
+ * is row-major (index j*width+i) and is distributed by rows (A2).     */
+skl_status skl_vector_create(skl_ctx* ctx, skl_type t, size_t n, skl_cont** out);
+skl_status skl_matrix_create(skl_ctx* ctx, skl_type t, size_t rows, size_t cols, skl_cont** out);
+skl_status skl_cont_destroy(skl_cont* c);
+/* rows = n and cols = 1 for a vector.                                          */
+skl_status skl_cont_info(skl_cont* c, skl_type* t, size_t* rows, size_t* cols, int* is_matrix);
+
+/* Implicit transfers.  skl_copy_in writes the whole container
+ * from `host` (bytes must equal the container size): if a distribution is set
+ * the data goes straight to the devices that need it (no host mirror), else it
+ * lands in the host mirror and is uploaded by the first skeleton that reads it.
+ * skl_copy_out downloads the whole container into `host` (collective in
+ * multi-process mode).  skl_copy_out_part downloads only the part that local
+ * device g owns (its block rows/elements); first_unit / nunits say which.     */
+skl_status skl_copy_in(skl_cont* c, const void* host, size_t bytes);
+skl_status skl_copy_out(skl_cont* c, void* host, size_t bytes);
+skl_status skl_copy_out_part(skl_cont* c, int g, void* host, size_t bytes, size_t* first_unit,
+                             size_t* nunits);
+/* Host view ("vec[i] = i"): a pinned mirror of the whole container.
+ * SKL_READ downloads it if devices are newer; SKL_WRITE / SKL_RW mark the device
+ * copies stale.  Valid until the next call that writes c, or its destruction.  */
+#define SKL_READ 1
+#define SKL_WRITE 2
+#define SKL_RW 3
+skl_status skl_host_data(skl_cont* c, int mode, void** host);
+/* Fill every element with *value (on the devices of the current distribution;
+ * a container with no distribution is filled in the host mirror).             */
+skl_status skl_fill(skl_cont* c, const void* value);
+
+/* ------------------------------------------------------------------ distributions
+ * P:L205-222 (Figs. 1, 2): single (whole container on one GPU, the first by
+ * default), copy (full replica on every GPU), block (contiguous disjoint chunk
+ * per GPU; chunk = ceil(units/G), A1), overlap (block plus `arg` border units of
+ * each neighbour; rows for a matrix).  P:L223-231: changing the distribution at
+ * run time moves the data implicitly, device to device.
+ *
+ * `combine` (copy only; A25, BASELINE north_star): a Reduce skeleton whose
+ * binary function (+) folds diverged replicas when the container leaves the copy
+ * distribution: block g = r_0[g] (+) r_1[g] (+) ... (+) r_{G-1}[g], GPU order.
+ * Replicas diverge when a skeleton writes the container as an extra argument
+ * (SKL_WRITE) on several devices.  NULL = replicas are assumed identical.      */
+#define SKL_DIST_NONE 0
+#define SKL_SINGLE 1
+#define SKL_COPY 2
+#define SKL_BLOCK 3
+#define SKL_OVERLAP 4
+skl_status skl_set_distribution(skl_cont* c, int kind, int arg, skl_skel* combine);
+skl_status skl_get_distribution(skl_cont* c, int* kind, int* arg);
+/* Borrowed device view of device g's part: *dptr addresses unit *first_unit;
+ * *nunits units are valid (including valid halo units for overlap).  For
+ * tests and interop; NULL dptr if g holds nothing or is not local.            */
+skl_status skl_local_part(skl_cont* c, int g, void** dptr, size_t* first_unit, size_t* nunits);
+
+/* ------------------------------------------------------------------ skeletons
+ * Customising functions are source strings (P:L252-254, P:L279-282,
+ * P:L626-633), compiled at skeleton creation with NVRTC for sm_100a
+ * (-fmad=false, IEEE div/sqrt, no FTZ: the GPU twin of the oracle's
+ * -ffp-contract=off) and spliced into the skeleton's kernel.  The language is
+ * CUDA C++ device code plus a compatibility prelude: uchar, uint, ushort,
+ * `__global` (ignored), get(p,dx,dy) / get(p,dx) and SCL_NEUTRAL / SCL_NEAREST
+ * (A14).  Functions need no __device__ qualifier.  `entry` names the function
+ * to apply; NULL = the last top-level function defined in `src` (A13).
+ *
+ *  Map        P:L249-256   out[i] = f(in[i]);  out type SKL_VOID allowed (A27)
+ *  Zip        P:L257-263   out[i] = l[i] (+) r[i]
+ *  Reduce     P:L264-270   v1 (+) v2 (+) ... (+) vn, (+) associative only
+ *  Scan       P:L271-278   inclusive prefix, (+) associative only (A9)
+ *  MapOverlap P:L311-384   out[i,j] = f(&in[i,j]) with get(p,dx,dy), |dx|,|dy| <= d;
+ *                          outside the matrix: `neutral` (SKL_NEUTRAL) or the
+ *                          nearest valid element (SKL_NEAREST, A20)
+ *
+ * Extra arguments (A27, not in the paper): `extra[k]` types are appended to the
+ * customising function's parameters; SKL_PTR-flagged ones are containers (the
+ * function receives the local device's `T*`; a copy-distributed container is
+ * the device's replica), others are passed by value.                          */
+#define SKL_NEUTRAL 0
+#define SKL_NEAREST 1
+skl_status skl_map_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in,
+                          skl_type out, const skl_type* extra, int nextra, skl_skel** sk);
+skl_status skl_zip_create(skl_ctx* ctx, const char* src, const char* entry, skl_type left,
+                          skl_type right, skl_type out, const skl_type* extra, int nextra,
+                          skl_skel** sk);
+skl_status skl_reduce_create(skl_ctx* ctx, const char* src, const char* entry, skl_type t,
+                             skl_skel** sk);
+skl_status skl_scan_create(skl_ctx* ctx, const char* src, const char* entry, skl_type t,
+                           skl_skel** sk);
+skl_status skl_mapoverlap_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in,
+                                 skl_type out, int d, int boundary, const void* neutral,
+                                 skl_skel** sk);
+skl_status skl_skel_destroy(skl_skel* sk);
+
+/* One extra argument at run time.                                             */
+#define SKL_ARG_SCALAR 1
+#define SKL_ARG_CONT 2
+typedef struct skl_arg {
+  int kind;          /* SKL_ARG_SCALAR or SKL_ARG_CONT                        */
+  int mode;          /* containers: SKL_READ, SKL_WRITE or SKL_RW             */
+  const void* value; /* scalars: pointer to the value (host)                  */
+  size_t bytes;      /* scalars: size of the value                            */
+  skl_cont* cont;    /* containers                                            */
+} skl_arg;
+
+/* Execution: `*out` NULL = allocate a new output container; otherwise it is
+ * reused (must have the right type and size).  Distributions (A6-A8): inputs
+ * without one default to block (MapOverlap: overlap(d)); Zip redistributes its
+ * right input to the left one's; outputs take the input's distribution, except
+ * MapOverlap (block) and Reduce (a 1-element scalar: single(0) with one process,
+ * copy across processes).  A copy input is computed whole on every device.     */
+skl_status skl_map_run(skl_skel* sk, skl_cont* in, skl_cont** out, const skl_arg* extra, int nextra);
+skl_status skl_zip_run(skl_skel* sk, skl_cont* left, skl_cont* right, skl_cont** out,
+                       const skl_arg* extra, int nextra);
+skl_status skl_reduce_run(skl_skel* sk, skl_cont* in, skl_cont** scalar);
+skl_status skl_scan_run(skl_skel* sk, skl_cont* in, skl_cont** out);
+skl_status skl_mapoverlap_run(skl_skel* sk, skl_cont* in, skl_cont** out);
+/* Scalar<T>::getValue(): download the 1-element result.           */
+skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes);
+
+/* ------------------------------------------------------------------ offline compilation
+ * skl_init_offline: a context without devices (no GPU needed) in which
+ * skeleton creation runs the full NVRTC compilation for sm_100a but loads
+ * nothing; containers and skeleton calls fail with SKL_ERR_CUDA.  Used for
+ * compile tests and for SASS inspection of the generated
+ * kernels.  skl_skel_cubin copies the skeleton's sm_100a cubin (main program)
+ * into buf (if cap suffices) and returns its size; skl_skel_source does the same
+ * for the generated CUDA source.                                               */
+skl_status skl_init_offline(skl_ctx** out);
+skl_status skl_skel_cubin(skl_skel* sk, void* buf, size_t cap, size_t* size);
+skl_status skl_skel_source(skl_skel* sk, char* buf, size_t cap, size_t* size);
+
+/* ------------------------------------------------------------------ host-only planning
+ * Pure host logic (no GPU needed), exported for tests of the multi-device path.
+ * skl_plan_range: the unit range [lo,hi) device g must hold for a distribution
+ * over `units` units and G devices (kind/arg as in skl_set_distribution;
+ * `with_halo` = include overlap halos).
+ * skl_plan_transfers: the device-to-device transfers that turn distribution
+ * (from_kind, from_arg) into (to_kind, to_arg); written as 5-tuples
+ * (src_device, src_unit, dst_device, dst_unit, nunits) in canonical order (the
+ * order both sides of an NCCL send/recv pair issue them).  Returns the count in
+ * *ntransfers (at most cap are written).                                       */
+skl_status skl_plan_range(size_t units, int G, int kind, int arg, int g, int with_halo,
+                          size_t* lo, size_t* hi);
+skl_status skl_plan_transfers(size_t units, int G, int from_kind, int from_arg, int to_kind,
+                              int to_arg, int64_t* tuples, size_t cap, size_t* ntransfers);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* SKL_H */

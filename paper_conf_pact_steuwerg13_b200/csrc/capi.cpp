@@ -1,0 +1,492 @@
+// capi.cpp — the C ABI (include/skl.h).  Argument checking and error mapping
+// only: every call converts exceptions to skl_status + skl_last_error().
+#include <functional>
+
+#include "skl_internal.h"
+
+namespace skl {
+Ctx* ctx_create_local(int ndev, const int* devices);
+Ctx* ctx_create_dist(int rank, int world, int cuda_device, const void* nccl_id);
+Ctx* ctx_create_offline();
+void ctx_destroy(Ctx* c);
+const char* last_error_cstr();
+void set_last_error(const std::string& s);
+}  // namespace skl
+
+using namespace skl;
+
+
+namespace {
+template <class F>
+skl_status guard(F&& f) {
+  try {
+    f();
+    return SKL_OK;
+  } catch (const Error& e) {
+    set_last_error(e.what());
+    return e.code;
+  } catch (const std::bad_alloc&) {
+    set_last_error("host allocation failed");
+    return SKL_ERR_OOM;
+  } catch (const std::exception& e) {
+    set_last_error(e.what());
+    return SKL_ERR_INVALID_ARG;
+  }
+}
+// Handles map 1:1 onto internal objects; the wrapper structs are owned by them.
+std::map<Ctx*, skl_ctx*> g_ctx;
+std::map<Cont*, skl_cont*> g_cont;
+std::map<Skel*, skl_skel*> g_skel;
+
+Ctx* C(skl_ctx* x) {
+  if (!x || !x->c) fail(SKL_ERR_INVALID_ARG, "NULL context");
+  return x->c;
+}
+Cont* K(skl_cont* x) {
+  if (!x || !x->c) fail(SKL_ERR_INVALID_ARG, "NULL container");
+  return x->c;
+}
+Skel* S(skl_skel* x) {
+  if (!x || !x->s) fail(SKL_ERR_INVALID_ARG, "NULL skeleton");
+  return x->s;
+}
+skl_cont* wrap(Cont* c) {
+  auto it = g_cont.find(c);
+  if (it != g_cont.end()) return it->second;
+  auto* w = new skl_cont{c};
+  g_cont[c] = w;
+  return w;
+}
+skl_skel* wrap(Skel* s) {
+  auto* w = new skl_skel{s};
+  g_skel[s] = w;
+  return w;
+}
+void forget_ctx_objects(Ctx* c) {
+  for (auto it = g_cont.begin(); it != g_cont.end();)
+    if (it->first->ctx == c) { it->second->c = nullptr; it = g_cont.erase(it); } else ++it;
+  for (auto it = g_skel.begin(); it != g_skel.end();)
+    if (it->first->ctx == c) { it->second->s = nullptr; it = g_skel.erase(it); } else ++it;
+}
+// output container handles: NULL -> new container
+skl_status run_out(skl_cont** out, const std::function<void(Cont**)>& f) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL output handle pointer");
+    Cont* o = *out ? K(*out) : nullptr;
+    f(&o);
+    *out = wrap(o);
+  });
+}
+}  // namespace
+
+extern "C" {
+
+const char* skl_last_error(void) { return last_error_cstr(); }
+
+skl_status skl_init(int ndev, const int* devices, skl_ctx** out) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    Ctx* c = ctx_create_local(ndev, devices);
+    *out = new skl_ctx{c};
+    g_ctx[c] = *out;
+  });
+}
+skl_status skl_init_dist(int rank, int world, int cuda_device, const void* nccl_id, skl_ctx** out) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    Ctx* c = ctx_create_dist(rank, world, cuda_device, nccl_id);
+    *out = new skl_ctx{c};
+    g_ctx[c] = *out;
+  });
+}
+skl_status skl_nccl_unique_id(void* out128) {
+  return guard([&] {
+    if (!out128) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    nccl_get_unique_id(out128);
+  });
+}
+skl_status skl_finalize(skl_ctx* ctx) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    forget_ctx_objects(c);
+    ctx_destroy(c);
+    g_ctx.erase(c);
+    ctx->c = nullptr;
+    delete ctx;
+  });
+}
+skl_status skl_num_devices(skl_ctx* ctx, int* ndev, int* first_local, int* nlocal) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (ndev) *ndev = c->G;
+    if (first_local) *first_local = c->first_local;
+    if (nlocal) *nlocal = c->nlocal;
+  });
+}
+skl_status skl_set_stream(skl_ctx* ctx, int g, void* stream) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (!c->is_local(g)) fail(SKL_ERR_INVALID_ARG, "device is not local");
+    Device& d = c->D(g);
+    cudaStream_t ns = stream ? (cudaStream_t)stream : d.own;
+    if (ns == d.stream) return;
+    // order the new stream after everything queued on the old one
+    c->set_device(g);
+    SKL_CUDA(cudaEventRecord(d.ev, d.stream));
+    SKL_CUDA(cudaStreamWaitEvent(ns, d.ev, 0));
+    d.stream = ns;
+  });
+}
+skl_status skl_get_stream(skl_ctx* ctx, int g, void** stream) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (!c->is_local(g) || !stream) fail(SKL_ERR_INVALID_ARG, "bad device or NULL out");
+    *stream = (void*)c->D(g).stream;
+  });
+}
+skl_status skl_sync(skl_ctx* ctx) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    for (auto& d : c->dev) {
+      SKL_CUDA(cudaSetDevice(d.phys));
+      SKL_CUDA(cudaStreamSynchronize(d.stream));
+    }
+    SKL_CUDA(cudaGetLastError());
+  });
+}
+skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    const std::string k = key ? key : "";
+    if (k == "block_threads") {
+      if (value < 64 || value > 1024 || value % 32) fail(SKL_ERR_INVALID_ARG, "block_threads must be a multiple of 32 in [64,1024]");
+      c->block_threads = (int)value;
+    } else if (k == "debug_bounds") {
+      c->debug_bounds = value ? 1 : 0;
+    } else if (k == "map_unroll") {
+      if (value < 1 || value > 16) fail(SKL_ERR_INVALID_ARG, "map_unroll in [1,16]");
+      c->map_unroll = (int)value;
+    } else {
+      fail(SKL_ERR_INVALID_ARG, "unknown option " + k);
+    }
+  });
+}
+skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    const std::string k = key ? key : "";
+    if (!value) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    if (k == "launches") *value = c->n_launch;
+    else if (k == "compiles") *value = c->n_compile;
+    else if (k == "cache_hits") *value = c->n_cache_hit;
+    else if (k == "h2d_bytes") *value = c->h2d;
+    else if (k == "d2h_bytes") *value = c->d2h;
+    else if (k == "p2p_bytes") *value = c->p2p;
+    else fail(SKL_ERR_INVALID_ARG, "unknown counter " + k);
+  });
+}
+
+skl_status skl_type_struct(skl_ctx* ctx, const char* name, const char* decl_src, size_t size,
+                           size_t align, skl_type* out) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (!name || !decl_src || !out || size == 0) fail(SKL_ERR_INVALID_ARG, "bad struct type");
+    for (size_t i = 0; i < c->types.size(); ++i)
+      if (c->types[i].name == name) {
+        if (c->types[i].decl != decl_src || c->types[i].size != size)
+          fail(SKL_ERR_TYPE, std::string("struct type ") + name + " already registered differently");
+        *out = (skl_type)i;  // idempotent
+        return;
+      }
+    TypeInfo t;
+    t.name = name;
+    t.decl = decl_src;
+    t.size = size;
+    t.align = align ? align : 1;
+    c->types.push_back(t);
+    *out = (skl_type)(c->types.size() - 1);
+  });
+}
+skl_status skl_type_size(skl_ctx* ctx, skl_type t, size_t* size) {
+  return guard([&] {
+    if (!size) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *size = C(ctx)->type(t & ~SKL_PTR).size;
+  });
+}
+
+// ---- containers
+skl_status skl_vector_create(skl_ctx* ctx, skl_type t, size_t n, skl_cont** out) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *out = wrap(cont_create(C(ctx), t, n, 1, false));
+  });
+}
+skl_status skl_matrix_create(skl_ctx* ctx, skl_type t, size_t rows, size_t cols, skl_cont** out) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *out = wrap(cont_create(C(ctx), t, rows, cols, true));
+  });
+}
+skl_status skl_cont_destroy(skl_cont* c) {
+  return guard([&] {
+    Cont* k = K(c);
+    g_cont.erase(k);
+    cont_destroy(k);
+    c->c = nullptr;
+    delete c;
+  });
+}
+skl_status skl_cont_info(skl_cont* c, skl_type* t, size_t* rows, size_t* cols, int* is_matrix) {
+  return guard([&] {
+    Cont* k = K(c);
+    if (t) *t = k->type;
+    if (rows) *rows = k->rows;
+    if (cols) *cols = k->cols;
+    if (is_matrix) *is_matrix = k->matrix;
+  });
+}
+skl_status skl_copy_in(skl_cont* c, const void* host, size_t bytes) {
+  return guard([&] {
+    Cont* k = K(c);
+    if (!host || bytes != k->bytes()) fail(SKL_ERR_SIZE_MISMATCH, "copy_in: byte count must equal the container size");
+    if (k->dist.kind == DNONE) {
+      void* m = host_mirror(k, SKL_WRITE);
+      std::memcpy(m, host, bytes);
+    } else {
+      host_upload(k, host);
+      k->host_valid = false;
+    }
+  });
+}
+skl_status skl_copy_out(skl_cont* c, void* host, size_t bytes) {
+  return guard([&] {
+    Cont* k = K(c);
+    if (!host || bytes != k->bytes()) fail(SKL_ERR_SIZE_MISMATCH, "copy_out: byte count must equal the container size");
+    if (k->host_valid && k->host) std::memcpy(host, k->host, bytes);
+    else host_download(k, host);
+  });
+}
+skl_status skl_copy_out_part(skl_cont* c, int g, void* host, size_t bytes, size_t* first_unit,
+                             size_t* nunits) {
+  return guard([&] {
+    Cont* k = K(c);
+    size_t f = 0, n = 0;
+    const Range r = core_range(k->units(), k->ctx->G, k->dist, g);
+    if (!host || bytes < r.size() * k->unit_bytes()) fail(SKL_ERR_SIZE_MISMATCH, "copy_out_part: buffer too small");
+    download_part(k, g, host, &f, &n);
+    if (first_unit) *first_unit = f;
+    if (nunits) *nunits = n;
+  });
+}
+skl_status skl_host_data(skl_cont* c, int mode, void** host) {
+  return guard([&] {
+    if (!host || mode < 1 || mode > 3) fail(SKL_ERR_INVALID_ARG, "bad mode or NULL out");
+    *host = host_mirror(K(c), mode);
+  });
+}
+skl_status skl_fill(skl_cont* c, const void* value) {
+  return guard([&] {
+    if (!value) fail(SKL_ERR_INVALID_ARG, "NULL value");
+    fill(K(c), value);
+  });
+}
+skl_status skl_set_distribution(skl_cont* c, int kind, int arg, skl_skel* combine) {
+  return guard([&] {
+    Cont* k = K(c);
+    Ctx* ctx = k->ctx;
+    Dist d{kind, 0};
+    switch (kind) {
+      case SKL_SINGLE:
+        if (arg < 0 || arg >= ctx->G) fail(SKL_ERR_INVALID_ARG, "single: device out of range");
+        d.arg = arg;
+        break;
+      case SKL_COPY:
+      case SKL_BLOCK:
+        break;
+      case SKL_OVERLAP:
+        if (arg < 0) fail(SKL_ERR_INVALID_ARG, "overlap size must be >= 0");
+        d.arg = arg;
+        break;
+      default:
+        fail(SKL_ERR_INVALID_ARG, "unknown distribution");
+    }
+    if (combine) {
+      if (kind != SKL_COPY) fail(SKL_ERR_DISTRIBUTION, "a combine function needs the copy distribution (A25)");
+      Skel* s = S(combine);
+      if (s->kind != K_REDUCE || ctx->type(s->tin).size != k->elt)
+        fail(SKL_ERR_TYPE, "combine must be a Reduce skeleton over the container's element type");
+    }
+    if (!k->dev_valid) {
+      k->dist = d;  // data moves lazily (upload at first use)
+    } else {
+      ensure(k, d, kind == SKL_OVERLAP);
+    }
+    if (kind == SKL_COPY) k->combine = combine ? S(combine) : nullptr;
+  });
+}
+skl_status skl_get_distribution(skl_cont* c, int* kind, int* arg) {
+  return guard([&] {
+    Cont* k = K(c);
+    if (kind) *kind = k->dist.kind;
+    if (arg) *arg = k->dist.arg;
+  });
+}
+skl_status skl_local_part(skl_cont* c, int g, void** dptr, size_t* first_unit, size_t* nunits) {
+  return guard([&] {
+    Cont* k = K(c);
+    if (!dptr) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *dptr = nullptr;
+    if (first_unit) *first_unit = 0;
+    if (nunits) *nunits = 0;
+    if (g < 0 || g >= k->ctx->G || !k->ctx->is_local(g)) return;
+    Part& p = k->parts[(size_t)g];
+    if (!p.ptr || p.valid.empty() || !k->dev_valid) return;
+    *dptr = part_ptr(k, g, p.valid.lo);
+    if (first_unit) *first_unit = p.valid.lo;
+    if (nunits) *nunits = p.valid.size();
+  });
+}
+
+// ---- skeletons
+skl_status skl_map_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in, skl_type out,
+                          const skl_type* extra, int nextra, skl_skel** sk) {
+  return guard([&] {
+    if (!sk || nextra < 0 || (nextra && !extra)) fail(SKL_ERR_INVALID_ARG, "bad arguments");
+    *sk = wrap(skel_create(C(ctx), K_MAP, src, entry, in, 0, out, extra, nextra, 0, 0, nullptr));
+  });
+}
+skl_status skl_zip_create(skl_ctx* ctx, const char* src, const char* entry, skl_type left,
+                          skl_type right, skl_type out, const skl_type* extra, int nextra,
+                          skl_skel** sk) {
+  return guard([&] {
+    if (!sk || nextra < 0 || (nextra && !extra)) fail(SKL_ERR_INVALID_ARG, "bad arguments");
+    *sk = wrap(skel_create(C(ctx), K_ZIP, src, entry, left, right, out, extra, nextra, 0, 0, nullptr));
+  });
+}
+skl_status skl_reduce_create(skl_ctx* ctx, const char* src, const char* entry, skl_type t, skl_skel** sk) {
+  return guard([&] {
+    if (!sk) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *sk = wrap(skel_create(C(ctx), K_REDUCE, src, entry, t, 0, t, nullptr, 0, 0, 0, nullptr));
+  });
+}
+skl_status skl_scan_create(skl_ctx* ctx, const char* src, const char* entry, skl_type t, skl_skel** sk) {
+  return guard([&] {
+    if (!sk) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *sk = wrap(skel_create(C(ctx), K_SCAN, src, entry, t, 0, t, nullptr, 0, 0, 0, nullptr));
+  });
+}
+skl_status skl_mapoverlap_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in,
+                                 skl_type out, int d, int boundary, const void* neutral, skl_skel** sk) {
+  return guard([&] {
+    if (!sk) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *sk = wrap(skel_create(C(ctx), K_MAPOVERLAP, src, entry, in, 0, out, nullptr, 0, d, boundary, neutral));
+  });
+}
+skl_status skl_skel_destroy(skl_skel* sk) {
+  return guard([&] {
+    Skel* s = S(sk);
+    g_skel.erase(s);
+    skel_destroy(s);
+    sk->s = nullptr;
+    delete sk;
+  });
+}
+skl_status skl_map_run(skl_skel* sk, skl_cont* in, skl_cont** out, const skl_arg* extra, int nextra) {
+  Skel* s = nullptr;
+  skl_status st = guard([&] { s = S(sk); K(in); });
+  if (st) return st;
+  if (s->tout == SKL_VOID) {
+    return guard([&] {
+      Cont* none = nullptr;
+      run_map(s, K(in), &none, extra, nextra);
+      if (out) *out = nullptr;
+    });
+  }
+  return run_out(out, [&](Cont** o) { run_map(s, K(in), o, extra, nextra); });
+}
+skl_status skl_zip_run(skl_skel* sk, skl_cont* left, skl_cont* right, skl_cont** out,
+                       const skl_arg* extra, int nextra) {
+  Skel* s = nullptr;
+  skl_status st = guard([&] { s = S(sk); K(left); K(right); });
+  if (st) return st;
+  if (s->tout == SKL_VOID) {
+    return guard([&] {
+      Cont* none = nullptr;
+      run_zip(s, K(left), K(right), &none, extra, nextra);
+      if (out) *out = nullptr;
+    });
+  }
+  return run_out(out, [&](Cont** o) { run_zip(s, K(left), K(right), o, extra, nextra); });
+}
+skl_status skl_reduce_run(skl_skel* sk, skl_cont* in, skl_cont** scalar) {
+  return run_out(scalar, [&](Cont** o) { run_reduce(S(sk), K(in), o); });
+}
+skl_status skl_scan_run(skl_skel* sk, skl_cont* in, skl_cont** out) {
+  return run_out(out, [&](Cont** o) { run_scan(S(sk), K(in), o); });
+}
+skl_status skl_mapoverlap_run(skl_skel* sk, skl_cont* in, skl_cont** out) {
+  return run_out(out, [&](Cont** o) { run_mapoverlap(S(sk), K(in), o); });
+}
+skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes) {
+  return guard([&] {
+    Cont* k = K(scalar);
+    if (!value || bytes != k->bytes()) fail(SKL_ERR_SIZE_MISMATCH, "scalar_get: byte count must equal the element size");
+    host_download(k, value);
+  });
+}
+
+// ---- offline compilation / introspection
+skl_status skl_init_offline(skl_ctx** out) {
+  return guard([&] {
+    if (!out) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    Ctx* c = ctx_create_offline();
+    *out = new skl_ctx{c};
+    g_ctx[c] = *out;
+  });
+}
+skl_status skl_skel_cubin(skl_skel* sk, void* buf, size_t cap, size_t* size) {
+  return guard([&] {
+    Skel* s = S(sk);
+    if (!size) fail(SKL_ERR_INVALID_ARG, "NULL size");
+    *size = s->prog->cubin.size();
+    if (buf && cap >= *size) std::memcpy(buf, s->prog->cubin.data(), *size);
+  });
+}
+skl_status skl_skel_source(skl_skel* sk, char* buf, size_t cap, size_t* size) {
+  return guard([&] {
+    Skel* s = S(sk);
+    if (!size) fail(SKL_ERR_INVALID_ARG, "NULL size");
+    *size = s->prog->source.size() + 1;
+    if (buf && cap >= *size) std::memcpy(buf, s->prog->source.c_str(), *size);
+  });
+}
+
+// ---- host-only planning
+skl_status skl_plan_range(size_t units, int G, int kind, int arg, int g, int with_halo, size_t* lo,
+                          size_t* hi) {
+  return guard([&] {
+    if (G < 1 || g < 0 || g >= G || !lo || !hi) fail(SKL_ERR_INVALID_ARG, "bad arguments");
+    const Dist d{kind, arg};
+    const Range r = with_halo ? need_range(units, G, d, g) : core_range(units, G, d, g);
+    *lo = r.lo;
+    *hi = r.hi;
+  });
+}
+skl_status skl_plan_transfers(size_t units, int G, int from_kind, int from_arg, int to_kind, int to_arg,
+                              int64_t* tuples, size_t cap, size_t* ntransfers) {
+  return guard([&] {
+    if (G < 1 || !ntransfers) fail(SKL_ERR_INVALID_ARG, "bad arguments");
+    const std::vector<Transfer> tr = plan_transfers(units, G, Dist{from_kind, from_arg}, from_kind == SKL_OVERLAP,
+                                                    Dist{to_kind, to_arg}, to_kind == SKL_OVERLAP);
+    *ntransfers = tr.size();
+    for (size_t i = 0; i < tr.size() && i < cap && tuples; ++i) {
+      tuples[5 * i + 0] = tr[i].src;
+      tuples[5 * i + 1] = (int64_t)tr[i].src_unit;
+      tuples[5 * i + 2] = tr[i].dst;
+      tuples[5 * i + 3] = (int64_t)tr[i].dst_unit;
+      tuples[5 * i + 4] = (int64_t)tr[i].n;
+    }
+  });
+}
+
+}  // extern "C"

@@ -1,0 +1,427 @@
+// container.cpp — containers, implicit transfers and the redistribution engine
+// (SURVEY §1 layers B2/B3).
+//
+// Vector / Matrix containers; "when a container is created on the
+// CPU, memory is allocated on the GPUs automatically".  P:L158-168: transfers
+// CPU<->GPU happen implicitly: before a skeleton reads a container and before
+// the host reads it.  P:L223-231: a container's distribution can change at run
+// time and SkelCL moves the data.  Reading A25: leaving a copy distribution whose
+// replicas diverged folds them with the combine function, in GPU order.
+//
+// Storage model: device g's part is one buffer covering a unit range `buf`
+// (units = elements of a vector, rows of a matrix); `valid` is the sub-range
+// holding data.  A part may keep spare halo room so that block -> overlap(d)
+// (the halo refresh of iterated stencils) moves only the 2d border units.
+#include <algorithm>
+
+#include "skl_internal.h"
+
+namespace skl {
+
+void launch_fill(Ctx* ctx, int g, void* dst, size_t bytes, const void* pattern, size_t elt);
+
+Cont* cont_create(Ctx* ctx, int type, size_t rows, size_t cols, bool matrix) {
+  const TypeInfo& ti = ctx->type(type);
+  if (ti.size == 0) fail(SKL_ERR_TYPE, "containers cannot hold void");
+  auto* c = new Cont();
+  c->ctx = ctx;
+  c->type = type;
+  c->elt = ti.size;
+  c->matrix = matrix;
+  c->rows = rows;
+  c->cols = matrix ? cols : 1;
+  c->parts.resize((size_t)ctx->G);
+  ctx->conts.insert(c);
+  return c;
+}
+
+static void free_part(Cont* c, int g) {
+  Part& p = c->parts[(size_t)g];
+  if (p.ptr) device_free(c->ctx, g, p.ptr);
+  p = Part();
+}
+
+void cont_destroy(Cont* c) {
+  Ctx* ctx = c->ctx;
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) free_part(c, g);
+  if (c->host) cudaFreeHost(c->host);
+  ctx->conts.erase(c);
+  delete c;
+}
+
+void* part_ptr(Cont* c, int g, size_t unit) {
+  Part& p = c->parts[(size_t)g];
+  if (!p.ptr || unit < p.buf.lo || unit > p.buf.hi)
+    fail(SKL_ERR_DISTRIBUTION, "internal: unit " + std::to_string(unit) + " not stored on device " +
+                                   std::to_string(g));
+  return (char*)p.ptr + (unit - p.buf.lo) * c->unit_bytes();
+}
+
+static Range alloc_range(Cont* c, const Dist& d, int g) {
+  Range need = need_range(c->units(), c->ctx->G, d, g);
+  if (need.empty()) return need;
+  if ((d.kind == DBLOCK || d.kind == DOVERLAP) && c->spare_halo) {
+    const Range core = core_range(c->units(), c->ctx->G, d, g);
+    const size_t s = c->spare_halo;
+    need.lo = std::min(need.lo, core.lo >= s ? core.lo - s : 0);
+    need.hi = std::max(need.hi, std::min(c->units(), core.hi + s));
+  }
+  return need;
+}
+
+// (Re)allocate device parts for layout d; data in reused buffers is kept.
+static void set_layout(Cont* c, const Dist& d) {
+  Ctx* ctx = c->ctx;
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range ar = alloc_range(c, d, g);
+    Part& p = c->parts[(size_t)g];
+    if (ar.empty()) {
+      free_part(c, g);
+      continue;
+    }
+    if (p.ptr && p.buf.contains(ar)) continue;
+    free_part(c, g);
+    p.ptr = device_alloc(ctx, g, ar.size() * c->unit_bytes());
+    p.buf = ar;
+    p.cap_bytes = ar.size() * c->unit_bytes();
+  }
+}
+
+static void set_valid(Cont* c, const Dist& d, bool halo) {
+  Ctx* ctx = c->ctx;
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    c->parts[(size_t)g].valid =
+        halo ? need_range(c->units(), ctx->G, d, g) : core_range(c->units(), ctx->G, d, g);
+  }
+}
+
+void mark_written(Cont* c) {
+  c->dev_valid = true;
+  c->host_valid = false;
+  c->halo_valid = false;
+  set_valid(c, c->dist, false);
+}
+
+void prepare_output(Cont* c, const Dist& d, size_t spare) {
+  if (spare > c->spare_halo) c->spare_halo = spare;
+  // buffers that must move would lose data; outputs are overwritten anyway
+  set_layout(c, d);
+  c->dist = d;
+  c->diverged = false;
+  c->dev_valid = false;
+  c->halo_valid = false;
+}
+
+// ------------------------------------------------------------------ host <-> device
+void host_upload(Cont* c, const void* host) {
+  Ctx* ctx = c->ctx;
+  const size_t ub = c->unit_bytes();
+  Dist d = c->dist;
+  if (d.kind == DCOPY && ctx->G > 1) {
+    // one PCIe upload, then replicate device-to-device over NVLink: upload the
+    // block slices (each device its own) and all-gather them.
+    Dist b{DBLOCK, 0};
+    c->dist = b;
+    host_upload(c, host);
+    c->diverged = false;
+    ensure(c, d, false);
+    return;
+  }
+  set_layout(c, d);
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range r = need_range(c->units(), ctx->G, d, g);
+    if (r.empty()) continue;
+    ctx->set_device(g);
+    SKL_CUDA(cudaMemcpyAsync(part_ptr(c, g, r.lo), (const char*)host + r.lo * ub, r.size() * ub,
+                             cudaMemcpyHostToDevice, ctx->D(g).stream));
+    ctx->h2d += (long long)(r.size() * ub);
+  }
+  set_valid(c, d, true);
+  c->dev_valid = true;
+  c->halo_valid = true;
+  c->diverged = false;
+}
+
+static void sync_local(Ctx* ctx) {
+  for (auto& d : ctx->dev) {
+    SKL_CUDA(cudaSetDevice(d.phys));
+    SKL_CUDA(cudaStreamSynchronize(d.stream));
+  }
+}
+
+namespace {
+struct ContPtrs : PtrFn {
+  Cont* src_c;
+  std::vector<Part>* src_parts;  // old parts (may differ from src_c->parts)
+  Cont* dst_c;
+  void* src(const Transfer& t) override {
+    Part& p = (*src_parts)[(size_t)t.src];
+    return (char*)p.ptr + (t.src_unit - p.buf.lo) * src_c->unit_bytes();
+  }
+  void* dst(const Transfer& t) override { return part_ptr(dst_c, t.dst, t.dst_unit); }
+};
+// gather everything into one full-size buffer on the local device (dist mode)
+struct GatherPtrs : PtrFn {
+  Cont* c;
+  void* buf;
+  void* src(const Transfer& t) override { return part_ptr(c, t.src, t.src_unit); }
+  void* dst(const Transfer& t) override { return (char*)buf + t.dst_unit * c->unit_bytes(); }
+};
+}  // namespace
+
+void host_download(Cont* c, void* host) {
+  Ctx* ctx = c->ctx;
+  const size_t ub = c->unit_bytes();
+  if (!c->dev_valid) {
+    if (c->host_valid && c->host && host != c->host) std::memcpy(host, c->host, c->bytes());
+    else if (!c->host_valid) std::memset(host, 0, c->bytes());
+    return;
+  }
+  if (c->dist.kind == DCOPY && c->diverged && c->combine) copy_combine_to_copy(c);
+  if (!ctx->dist_mode) {
+    for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+      // each unit from its owner (copy: device g's block slice, parallel D2H)
+      Range r = c->dist.kind == DCOPY ? block_range(c->units(), ctx->G, g)
+                                      : core_range(c->units(), ctx->G, c->dist, g);
+      if (r.empty()) continue;
+      ctx->set_device(g);
+      SKL_CUDA(cudaMemcpyAsync((char*)host + r.lo * ub, part_ptr(c, g, r.lo), r.size() * ub,
+                               cudaMemcpyDeviceToHost, ctx->D(g).stream));
+      ctx->d2h += (long long)(r.size() * ub);
+    }
+    sync_local(ctx);
+    return;
+  }
+  // one process per GPU: every rank assembles the whole container (collective)
+  const int g = ctx->first_local;
+  const Range have = core_range(c->units(), ctx->G, c->dist, g);
+  if (c->dist.kind == DCOPY) {
+    ctx->set_device(g);
+    SKL_CUDA(cudaMemcpyAsync(host, part_ptr(c, g, 0), c->bytes(), cudaMemcpyDeviceToHost, ctx->D(g).stream));
+    ctx->d2h += (long long)c->bytes();
+    sync_local(ctx);
+    return;
+  }
+  void* buf = device_alloc(ctx, g, c->bytes());
+  if (!have.empty()) {
+    ctx->set_device(g);
+    SKL_CUDA(cudaMemcpyAsync((char*)buf + have.lo * ub, part_ptr(c, g, have.lo), have.size() * ub,
+                             cudaMemcpyDeviceToDevice, ctx->D(g).stream));
+  }
+  const std::vector<Transfer> tr =
+      plan_transfers(c->units(), ctx->G, c->dist, false, Dist{DCOPY, 0}, false);
+  GatherPtrs gp;
+  gp.c = c;
+  gp.buf = buf;
+  run_transfers(ctx, tr, ub, gp);
+  ctx->set_device(g);
+  SKL_CUDA(cudaMemcpyAsync(host, buf, c->bytes(), cudaMemcpyDeviceToHost, ctx->D(g).stream));
+  ctx->d2h += (long long)c->bytes();
+  device_free(ctx, g, buf);
+  sync_local(ctx);
+}
+
+void download_part(Cont* c, int g, void* host, size_t* first, size_t* n) {
+  Ctx* ctx = c->ctx;
+  if (!ctx->is_local(g)) fail(SKL_ERR_INVALID_ARG, "device is not local to this process");
+  if (!c->dev_valid) fail(SKL_ERR_DISTRIBUTION, "container has no device data");
+  if (c->dist.kind == DCOPY && c->diverged && c->combine) copy_combine_to_copy(c);
+  const Range r = core_range(c->units(), ctx->G, c->dist, g);
+  *first = r.lo;
+  *n = r.size();
+  if (r.empty()) return;
+  ctx->set_device(g);
+  SKL_CUDA(cudaMemcpyAsync(host, part_ptr(c, g, r.lo), r.size() * c->unit_bytes(),
+                           cudaMemcpyDeviceToHost, ctx->D(g).stream));
+  ctx->d2h += (long long)(r.size() * c->unit_bytes());
+  SKL_CUDA(cudaStreamSynchronize(ctx->D(g).stream));
+}
+
+void* host_mirror(Cont* c, int mode) {
+  if (!c->host) SKL_CUDA(cudaHostAlloc(&c->host, std::max<size_t>(c->bytes(), 1), cudaHostAllocPortable));
+  if ((mode & SKL_READ) && !c->host_valid) {
+    host_download(c, c->host);
+    c->host_valid = true;
+  }
+  if (mode & SKL_WRITE) {
+    c->host_valid = true;
+    c->dev_valid = false;  // devices become stale
+    c->diverged = false;
+  }
+  return c->host;
+}
+
+void fill(Cont* c, const void* value) {
+  Ctx* ctx = c->ctx;
+  if (c->dist.kind == DNONE) {
+    char* h = (char*)host_mirror(c, SKL_WRITE);
+    for (size_t i = 0; i < c->rows * c->cols; ++i) std::memcpy(h + i * c->elt, value, c->elt);
+    return;
+  }
+  set_layout(c, c->dist);
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    Part& p = c->parts[(size_t)g];
+    if (!p.ptr) continue;
+    launch_fill(ctx, g, p.ptr, p.buf.size() * c->unit_bytes(), value, c->elt);
+  }
+  set_valid(c, c->dist, true);
+  c->dev_valid = true;
+  c->halo_valid = true;
+  c->host_valid = false;
+  c->diverged = false;
+}
+
+// ------------------------------------------------------------------ redistribution
+// copy(+) -> block (reading A25): block g = r_0[g] (+) ... (+) r_{G-1}[g].
+// Every device gathers the G replica slices of its block into staging (one
+// canonical all-to-all), then the ordered-combine kernel folds them.
+static void combine_to_block(Cont* c) {
+  Ctx* ctx = c->ctx;
+  const int G = ctx->G;
+  const size_t U = c->units(), ub = c->unit_bytes();
+  const Dist blk{DBLOCK, 0};
+  std::vector<void*> staging((size_t)G, nullptr);
+  std::vector<Transfer> tr;
+  for (int g = 0; g < G; ++g) {
+    const Range r = block_range(U, G, g);
+    if (r.empty()) continue;
+    for (int h = 0; h < G; ++h) tr.push_back(Transfer{h, g, r.lo, r.lo, r.size(), h});
+  }
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range r = block_range(U, G, g);
+    if (!r.empty()) staging[(size_t)g] = device_alloc(ctx, g, (size_t)G * r.size() * ub);
+  }
+  struct StagePtrs : PtrFn {
+    Cont* c;
+    std::vector<void*>* st;
+    size_t U;
+    int G;
+    void* src(const Transfer& t) override { return part_ptr(c, t.src, t.src_unit); }
+    void* dst(const Transfer& t) override {
+      const Range r = block_range(U, G, t.dst);
+      return (char*)(*st)[(size_t)t.dst] + ((size_t)t.slot * r.size() + (t.dst_unit - r.lo)) * c->unit_bytes();
+    }
+  } sp;
+  sp.c = c;
+  sp.st = &staging;
+  sp.U = U;
+  sp.G = G;
+  run_transfers(ctx, tr, ub, sp);
+  // replace the replicas by the folded blocks
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range r = block_range(U, G, g);
+    free_part(c, g);
+    if (r.empty()) continue;
+    Part& p = c->parts[(size_t)g];
+    const Range ar = alloc_range(c, blk, g);
+    p.ptr = device_alloc(ctx, g, ar.size() * ub);
+    p.buf = ar;
+    p.cap_bytes = ar.size() * ub;
+    run_combine(c->combine, g, staging[(size_t)g], r.size() * c->cols, G, part_ptr(c, g, r.lo),
+                r.size() * c->cols);
+    device_free(ctx, g, staging[(size_t)g]);
+  }
+  c->dist = blk;
+  c->diverged = false;
+  c->dev_valid = true;
+  c->halo_valid = false;
+  set_valid(c, blk, false);
+}
+
+static void redistribute(Cont* c, const Dist& to) {
+  Ctx* ctx = c->ctx;
+  const size_t U = c->units(), ub = c->unit_bytes();
+  const Dist from = c->dist;
+  const bool from_halo = from.kind == DOVERLAP && c->halo_valid;
+  const bool to_halo = to.kind == DOVERLAP;
+  const std::vector<Transfer> tr = plan_transfers(U, ctx->G, from, from_halo, to, to_halo);
+  std::vector<Part> old = c->parts;
+  std::vector<bool> moved((size_t)ctx->G, false);
+  // new layout; keep buffers that already cover the target
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range ar = alloc_range(c, to, g);
+    Part& p = c->parts[(size_t)g];
+    if (ar.empty()) {
+      if (p.ptr) moved[(size_t)g] = true;  // freed after the exchange
+      p = Part();
+      continue;
+    }
+    if (p.ptr && p.buf.contains(ar)) continue;
+    moved[(size_t)g] = p.ptr != nullptr;
+    p = Part();
+    p.ptr = device_alloc(ctx, g, ar.size() * ub);
+    p.buf = ar;
+    p.cap_bytes = ar.size() * ub;
+    // units this device already holds move locally into the new buffer
+    const Range have = from_halo ? need_range(U, ctx->G, from, g) : core_range(U, ctx->G, from, g);
+    const Range want = to_halo ? need_range(U, ctx->G, to, g) : core_range(U, ctx->G, to, g);
+    const Range keep{std::max(have.lo, want.lo), std::min(have.hi, want.hi)};
+    const Part& o = old[(size_t)g];
+    if (!keep.empty() && o.ptr) {
+      ctx->set_device(g);
+      SKL_CUDA(cudaMemcpyAsync((char*)p.ptr + (keep.lo - p.buf.lo) * ub,
+                               (const char*)o.ptr + (keep.lo - o.buf.lo) * ub, keep.size() * ub,
+                               cudaMemcpyDeviceToDevice, ctx->D(g).stream));
+    }
+  }
+  ContPtrs cp;
+  cp.src_c = c;
+  cp.src_parts = &old;
+  cp.dst_c = c;
+  run_transfers(ctx, tr, ub, cp);
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g)
+    if (moved[(size_t)g] && old[(size_t)g].ptr) device_free(ctx, g, old[(size_t)g].ptr);
+  c->dist = to;
+  c->dev_valid = true;
+  c->halo_valid = to_halo;
+  set_valid(c, to, to_halo);
+}
+
+void ensure(Cont* c, const Dist& d, bool halo) {
+  if (d.kind == DNONE) fail(SKL_ERR_DISTRIBUTION, "no distribution");
+  if (c->dev_valid && c->dist.kind == DCOPY && c->diverged && c->combine && !(d == c->dist)) {
+    combine_to_block(c);
+  }
+  if (c->dev_valid && c->dist.kind == DCOPY && c->diverged && d.kind == DCOPY && c->combine) {
+    copy_combine_to_copy(c);
+    return;
+  }
+  if (c->dist == d && c->dev_valid) {
+    if (d.kind == DOVERLAP && halo && !c->halo_valid) {
+      // halo refresh: only the border units move
+      const std::vector<Transfer> tr = plan_transfers(c->units(), c->ctx->G, d, false, d, true);
+      set_layout(c, d);  // buffers already cover the halo (need_range)
+      std::vector<Part> cur = c->parts;
+      ContPtrs cp;
+      cp.src_c = c;
+      cp.src_parts = &cur;
+      cp.dst_c = c;
+      run_transfers(c->ctx, tr, c->unit_bytes(), cp);
+      c->halo_valid = true;
+      set_valid(c, d, true);
+    }
+    return;
+  }
+  if (!c->dev_valid) {
+    c->dist = d;
+    if (c->host_valid && c->host) {
+      host_upload(c, c->host);
+    } else {
+      // never written: allocate only (contents undefined, A-none)
+      set_layout(c, d);
+      set_valid(c, d, true);
+      c->dev_valid = true;
+      c->halo_valid = true;
+    }
+    return;
+  }
+  if (c->dist.kind == DCOPY && c->diverged && !c->combine) c->diverged = false;  // A26
+  redistribute(c, d);
+}
+
+void copy_combine_to_copy(Cont* c) {
+  combine_to_block(c);
+  redistribute(c, Dist{DCOPY, 0});
+}
+
+}  // namespace skl

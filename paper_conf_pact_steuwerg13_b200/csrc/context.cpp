@@ -1,0 +1,200 @@
+// context.cpp — device context and communication (SURVEY §1 layers B1, comm).
+//
+// SkelCL::init() makes every GPU available; skeletons then run "on all
+// GPUs available in the system".  B200-native plumbing:
+//  * one CUDA stream per (logical) device; stream-ordered memory pools
+//    (cudaMallocAsync) with the release threshold raised so steady-state
+//    allocations are free;
+//  * single process, several devices: device-to-device copies
+//    (cudaMemcpyPeerAsync over NVLink when the physical GPUs differ);
+//  * one process per GPU (torchrun): NCCL grouped send/recv of the same
+//    canonical transfer list on every rank (libnccl.so.2 via dlopen).
+// The paper moves data between GPUs "via the CPU" in plain OpenCL (P:L119-121,
+// P:L228-231); nothing here stages through the host.
+#include <dlfcn.h>
+
+#include <cstdio>
+
+#include "skl_internal.h"
+
+namespace skl {
+
+static thread_local std::string g_last_error;
+const char* last_error_cstr() { return g_last_error.c_str(); }
+void set_last_error(const std::string& s) { g_last_error = s; }
+
+void fail(int code, const std::string& msg) { throw Error(code, msg); }
+
+void cuda_check(cudaError_t e, const char* what) {
+  if (e == cudaSuccess) return;
+  const int code = (e == cudaErrorMemoryAllocation) ? SKL_ERR_OOM : SKL_ERR_CUDA;
+  fail(code, std::string(what) + ": " + cudaGetErrorName(e) + " (" + cudaGetErrorString(e) + ")");
+}
+
+const TypeInfo& Ctx::type(int t) const {
+  if (t < 0 || (size_t)t >= types.size() || types[(size_t)t].size == 0)
+    fail(SKL_ERR_TYPE, "unknown element type " + std::to_string(t));
+  return types[(size_t)t];
+}
+
+void Ctx::set_device(int g) {
+  if (offline) fail(SKL_ERR_CUDA, "offline context (skl_init_offline) has no devices");
+  SKL_CUDA(cudaSetDevice(D(g).phys));
+}
+
+static void init_types(Ctx* c) {
+  c->types.resize(12);
+  c->types[SKL_VOID] = {"void", 0, 1, ""};
+  c->types[SKL_U8] = {"unsigned char", 1, 1, ""};
+  c->types[SKL_I8] = {"signed char", 1, 1, ""};
+  c->types[SKL_I32] = {"int", 4, 4, ""};
+  c->types[SKL_U32] = {"unsigned int", 4, 4, ""};
+  c->types[SKL_F32] = {"float", 4, 4, ""};
+  c->types[SKL_F64] = {"double", 8, 8, ""};
+  c->types[SKL_F32X2] = {"float2", 8, 8, ""};
+  c->types[SKL_I64] = {"long long", 8, 8, ""};
+  c->types[SKL_U64] = {"unsigned long long", 8, 8, ""};
+  c->types[SKL_I16] = {"short", 2, 2, ""};
+  c->types[SKL_U16] = {"unsigned short", 2, 2, ""};
+}
+
+static void init_device(Ctx* c, Device& d) {
+  SKL_CUDA(cudaSetDevice(d.phys));
+  SKL_CUDA(cudaStreamCreateWithFlags(&d.own, cudaStreamNonBlocking));
+  d.stream = d.own;
+  SKL_CUDA(cudaEventCreateWithFlags(&d.ev, cudaEventDisableTiming));
+  SKL_CUDA(cudaDeviceGetAttribute(&d.sm_count, cudaDevAttrMultiProcessorCount, d.phys));
+  cudaMemPool_t pool;
+  SKL_CUDA(cudaDeviceGetDefaultMemPool(&pool, d.phys));
+  uint64_t thr = UINT64_MAX;
+  SKL_CUDA(cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr));
+  (void)c;
+}
+
+Ctx* ctx_create_local(int ndev, const int* devices) {
+  int nvis = 0;
+  cudaError_t e = cudaGetDeviceCount(&nvis);
+  if (e != cudaSuccess || nvis <= 0)
+    fail(SKL_ERR_CUDA, std::string("no CUDA device available: ") + cudaGetErrorString(e));
+  auto* c = new Ctx();
+  init_types(c);
+  c->G = ndev > 0 ? ndev : nvis;
+  c->first_local = 0;
+  c->nlocal = c->G;
+  c->dev.resize((size_t)c->G);
+  try {
+    for (int g = 0; g < c->G; ++g) {
+      c->dev[(size_t)g].global = g;
+      c->dev[(size_t)g].phys = devices ? devices[g] : g % nvis;
+      if (c->dev[(size_t)g].phys < 0 || c->dev[(size_t)g].phys >= nvis)
+        fail(SKL_ERR_INVALID_ARG, "device ordinal out of range");
+      init_device(c, c->dev[(size_t)g]);
+    }
+    // peer access between distinct physical GPUs (NVLink / NVSwitch)
+    for (auto& a : c->dev)
+      for (auto& b : c->dev)
+        if (a.phys != b.phys) {
+          int can = 0;
+          cudaDeviceCanAccessPeer(&can, a.phys, b.phys);
+          if (can) {
+            cudaSetDevice(a.phys);
+            cudaError_t pe = cudaDeviceEnablePeerAccess(b.phys, 0);
+            if (pe != cudaSuccess) cudaGetLastError();  // already enabled is fine
+          }
+        }
+  } catch (...) {
+    delete c;
+    throw;
+  }
+  return c;
+}
+
+Ctx* ctx_create_dist(int rank, int world, int cuda_device, const void* nccl_id) {
+  int nvis = 0;
+  cudaError_t e = cudaGetDeviceCount(&nvis);
+  if (e != cudaSuccess || nvis <= 0)
+    fail(SKL_ERR_CUDA, std::string("no CUDA device available: ") + cudaGetErrorString(e));
+  if (world < 1 || rank < 0 || rank >= world) fail(SKL_ERR_INVALID_ARG, "bad rank/world");
+  auto* c = new Ctx();
+  init_types(c);
+  c->G = world;
+  c->dist_mode = world > 1;
+  c->rank = rank;
+  c->world = world;
+  c->first_local = rank;
+  c->nlocal = 1;
+  c->dev.resize(1);
+  c->dev[0].global = rank;
+  c->dev[0].phys = cuda_device;
+  try {
+    init_device(c, c->dev[0]);
+    if (world > 1) nccl_init(c, nccl_id);
+  } catch (...) {
+    delete c;
+    throw;
+  }
+  return c;
+}
+
+Ctx* ctx_create_offline() {
+  auto* c = new Ctx();
+  init_types(c);
+  c->offline = true;
+  c->G = 1;
+  c->nlocal = 0;
+  return c;
+}
+
+void ctx_destroy(Ctx* c) {
+  for (auto& d : c->dev) {
+    cudaSetDevice(d.phys);
+    cudaStreamSynchronize(d.stream);
+    cudaStreamSynchronize(d.own);
+  }
+  while (!c->skels.empty()) skel_destroy(*c->skels.begin());
+  while (!c->conts.empty()) cont_destroy(*c->conts.begin());
+  for (auto& kv : c->programs)
+    if (kv.second) {
+      // cudaLibraryUnload is safe after the streams drained
+      extern void program_unload(Program*);
+      program_unload(kv.second.get());
+    }
+  if (c->nccl_comm) nccl_destroy(c);
+  for (auto& d : c->dev) {
+    cudaSetDevice(d.phys);
+    if (d.ev) cudaEventDestroy(d.ev);
+    if (d.own) cudaStreamDestroy(d.own);
+  }
+  delete c;
+}
+
+void* device_alloc(Ctx* ctx, int g, size_t bytes) {
+  if (bytes == 0) bytes = 16;
+  ctx->set_device(g);
+  void* p = nullptr;
+  SKL_CUDA(cudaMallocAsync(&p, bytes, ctx->D(g).stream));
+  return p;
+}
+void device_free(Ctx* ctx, int g, void* p) {
+  if (!p) return;
+  ctx->set_device(g);
+  SKL_CUDA(cudaFreeAsync(p, ctx->D(g).stream));
+}
+
+// Every local stream waits for the work already queued on every other local
+// stream: orders a multi-device exchange after its producers and before its
+// consumers (G <= 8, so at most 64 event waits).
+void barrier_streams(Ctx* ctx) {
+  if (ctx->nlocal <= 1) return;
+  for (auto& d : ctx->dev) {
+    SKL_CUDA(cudaSetDevice(d.phys));
+    SKL_CUDA(cudaEventRecord(d.ev, d.stream));
+  }
+  for (auto& a : ctx->dev) {
+    SKL_CUDA(cudaSetDevice(a.phys));
+    for (auto& b : ctx->dev)
+      if (&a != &b) SKL_CUDA(cudaStreamWaitEvent(a.stream, b.ev, 0));
+  }
+}
+
+}  // namespace skl

@@ -1,0 +1,154 @@
+// mapoverlap.cuh — MapOverlap skeleton, matrix and vector forms.
+//
+//   mout[i,j] = f( min[i-d .. i+d, j-d .. j+d] )
+// f receives a pointer to the centre element and reads neighbours with
+// get(p, dx, dy), dx = column offset, dy = row offset (A15).
+// Out-of-bounds neighbours read a neutral value or the nearest valid element
+// (A20: each coordinate clamped independently).
+//
+// B200 design: the paper's kernel "uses the fast local memory";
+// here each block stages an output tile plus its halo in shared memory with
+// coalesced 16-byte loads, resolving the boundary mode while loading (no
+// per-access branch in f), then every thread applies f to a SKL_RH x SKL_CW
+// register block of outputs so neighbouring calls share shared-memory reads.
+// get() is a constant-offset load from the tile (SKL_PITCH is a compile-time
+// row pitch).  The input part holds rows [in_row0, in_row0 + in_rows) of the
+// global matrix (block rows + halo rows under the overlap distribution).
+// Configuration: SKL_TIN, SKL_TOUT, SKL_FUNC, SKL_D, SKL_BOUNDARY, SKL_TH,
+// SKL_TW, SKL_RH, SKL_CW, SKL_A (halo columns staged, >= d, 16-byte multiple),
+// SKL_PITCH, SKL_BLOCK, SKL_MO1D.
+#if SKL_DEBUG_BOUNDS
+extern "C" __device__ unsigned int skl_bounds_flag = 0u;
+#endif
+
+template <int B> struct SklRaw { typedef unsigned char type; };  // unused width
+template <> struct SklRaw<1> { typedef unsigned char type; };
+template <> struct SklRaw<2> { typedef unsigned short type; };
+template <> struct SklRaw<4> { typedef unsigned int type; };
+template <> struct SklRaw<8> { typedef uint2 type; };
+template <> struct SklRaw<16> { typedef uint4 type; };
+
+#define SKL_EPC (16 / (int)sizeof(SKL_TIN))
+// SKL_OUTB = SKL_CW * sizeof(SKL_TOUT), written by the host (used in #if)
+#define SKL_OUT_PACK (SKL_OUTB == 1 || SKL_OUTB == 2 || SKL_OUTB == 4 || SKL_OUTB == 8 || SKL_OUTB == 16)
+
+__device__ __forceinline__ long skl_clampl(long v, long lo, long hi) {
+  return v < lo ? lo : (v > hi ? hi : v);
+}
+
+#if !SKL_MO1D
+// ------------------------------------------------------------------ 2-D
+#define SKL_SROWS (SKL_TH + 2 * SKL_D)
+#define SKL_CPR (SKL_PITCH / SKL_EPC)  // 16-byte chunks per smem row
+
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
+         long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok) {
+  __shared__ __align__(16) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
+  const long r0 = r_begin + (long)blockIdx.y * SKL_TH;
+  const long c0 = (long)blockIdx.x * SKL_TW;
+  // ---- stage rows r0-d .. r0+TH+d-1, columns c0-A .. c0+TW+A-1
+  for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
+    const int i = q / SKL_CPR, jc = q - i * SKL_CPR;
+    long gr = r0 - SKL_D + i;
+    const long gc0 = c0 - SKL_A + (long)jc * SKL_EPC;
+    const bool row_in = gr >= 0 && gr < R;
+#if SKL_BOUNDARY == 1
+    gr = skl_clampl(gr, 0, R - 1);
+#endif
+    SKL_TIN* dst = tile + i * SKL_PITCH + jc * SKL_EPC;
+    if (r0 - SKL_D + i >= r_end + SKL_D) {  // below the last output row's window: unused
+#pragma unroll
+      for (int e = 0; e < SKL_EPC; ++e) dst[e] = neutral;
+      continue;
+    }
+    if (vec_ok && (SKL_BOUNDARY == 1 || row_in) && gc0 >= 0 && gc0 + SKL_EPC <= C) {
+      *(uint4*)dst = skl_ld16(in + (gr - in_row0) * C + gc0);
+    } else {
+#pragma unroll
+      for (int e = 0; e < SKL_EPC; ++e) {
+        long gc = gc0 + e;
+        SKL_TIN v;
+#if SKL_BOUNDARY == 1
+        gc = skl_clampl(gc, 0, C - 1);
+        v = in[(gr - in_row0) * C + gc];
+#else
+        if (row_in && gc >= 0 && gc < C) v = in[(gr - in_row0) * C + gc];
+        else v = neutral;
+#endif
+        dst[e] = v;
+      }
+    }
+  }
+  __syncthreads();
+  // ---- apply f to a SKL_RH x SKL_CW block per thread
+  const int ty = threadIdx.x / (SKL_TW / SKL_CW), tx = threadIdx.x % (SKL_TW / SKL_CW);
+  const long cc = c0 + (long)tx * SKL_CW;
+#pragma unroll
+  for (int i = 0; i < SKL_RH; ++i) {
+    const long r = r0 + (long)ty * SKL_RH + i;
+    const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
+    union {
+      SKL_TOUT e[SKL_CW];
+      typename SklRaw<SKL_OUTB>::type raw;
+    } res;
+#pragma unroll
+    // f may declare a non-const pointer (Listing 1.2: "float func(float* m_in)")
+    for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
+    if (r < r_end) {
+      SKL_TOUT* o = out + (r - out_row0) * C + cc;
+#if SKL_OUT_PACK
+      if (cc + SKL_CW <= C && vec_ok) {
+        *(typename SklRaw<SKL_OUTB>::type*)o = res.raw;
+        continue;
+      }
+#endif
+#pragma unroll
+      for (int j = 0; j < SKL_CW; ++j)
+        if (cc + j < C) o[j] = res.e[j];
+    }
+  }
+  (void)in_rows;
+}
+#else
+// ------------------------------------------------------------------ 1-D (vector)
+#define SKL_SLEN (SKL_TW + 2 * SKL_A)
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_mo1d(const SKL_TIN* __restrict__ in, long in_lo, long in_n, SKL_TOUT* __restrict__ out,
+         long out_lo, long N, long unused, long i_begin, long i_end, SKL_TIN neutral, int vec_ok) {
+  __shared__ __align__(16) SKL_TIN tile[SKL_SLEN];
+  const long e0 = i_begin + (long)blockIdx.x * SKL_TW;
+  for (int q = threadIdx.x; q < SKL_SLEN / SKL_EPC; q += SKL_BLOCK) {
+    const long g0 = e0 - SKL_A + (long)q * SKL_EPC;
+    SKL_TIN* dst = tile + q * SKL_EPC;
+    if (vec_ok && g0 >= in_lo && g0 + SKL_EPC <= in_lo + in_n && g0 >= 0 && g0 + SKL_EPC <= N &&
+        ((g0 - in_lo) % SKL_EPC) == 0) {
+      *(uint4*)dst = skl_ld16(in + (g0 - in_lo));
+    } else {
+#pragma unroll
+      for (int e = 0; e < SKL_EPC; ++e) {
+        long g = g0 + e;
+        SKL_TIN v;
+#if SKL_BOUNDARY == 1
+        g = skl_clampl(g, 0, N - 1);
+        if (g >= in_lo && g < in_lo + in_n) v = in[g - in_lo];
+        else v = neutral;  // outside every needed window
+#else
+        if (g >= 0 && g < N && g >= in_lo && g < in_lo + in_n) v = in[g - in_lo];
+        else v = neutral;
+#endif
+        dst[e] = v;
+      }
+    }
+  }
+  __syncthreads();
+  const long i0 = e0 + (long)threadIdx.x * SKL_CW;
+  const SKL_TIN* p = tile + SKL_A + threadIdx.x * SKL_CW;
+#pragma unroll
+  for (int j = 0; j < SKL_CW; ++j) {
+    const long i = i0 + j;
+    if (i < i_end) out[i - out_lo] = SKL_FUNC((SKL_TIN*)(p + j));
+  }
+  (void)unused;
+}
+#endif

@@ -1,0 +1,599 @@
+// skeletons.cpp — skeleton objects and their executors (SURVEY §1 layer B5).
+//
+// A skeleton is "a higher-order function that executes one or more
+// user-defined (so-called customizing) functions in a pre-defined parallel
+// manner".  Creation compiles the customising source into the
+// skeleton's sm_100a kernel template (NVRTC, compiler.cpp); a call
+// ("resultVector = neg(inputVector)") makes the inputs resident in
+// the distribution the skeleton needs (implicit transfers / redistribution,
+// container.cpp), launches one kernel per device on that device's part, and
+// performs the one cross-device step the skeleton has, if any:
+//   Map, Zip      none                       (block: independent parts)
+//   Reduce        ordered fold of the G device partials
+//   Scan          device totals -> carry-in of the later devices
+//   MapOverlap    overlap halo refresh before the stencil
+#include <algorithm>
+#include <cstdio>
+#include <numeric>
+
+#include "skl_internal.h"
+
+namespace skl {
+
+extern void set_last_error(const std::string& s);
+
+namespace {
+
+size_t gcd_sz(size_t a, size_t b) { return b ? gcd_sz(b, a % b) : a; }
+size_t lcm_sz(size_t a, size_t b) { return a / gcd_sz(a, b) * b; }
+// elements per chunk so that VEC * size is a multiple of 16 bytes for every size
+size_t vec_for(std::initializer_list<size_t> sizes) {
+  size_t v = 1;
+  for (size_t s : sizes)
+    if (s) v = lcm_sz(v, 16 / gcd_sz(16, s));
+  return v;
+}
+bool aligned16(const void* p) { return ((uintptr_t)p & 15u) == 0; }
+size_t ceil_div(size_t a, size_t b) { return (a + b - 1) / b; }
+
+std::string defs_common(Ctx* ctx, const std::string& entry) {
+  std::string s;
+  s += "#define SKL_BLOCK " + std::to_string(ctx->block_threads) + "\n";
+  s += "#define SKL_DEBUG_BOUNDS " + std::to_string(ctx->debug_bounds ? 1 : 0) + "\n";
+  s += "#define SKL_FUNC " + entry + "\n";
+  return s;
+}
+
+std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
+
+// Scratch buffer per (skeleton, device), grown on demand.
+void* scratch(Skel* s, std::map<int, Scratch>& m, int g, size_t bytes, bool zero) {
+  Scratch& sc = m[g];
+  if (sc.bytes < bytes) {
+    if (sc.ptr) device_free(s->ctx, g, sc.ptr);
+    sc.ptr = device_alloc(s->ctx, g, bytes);
+    sc.bytes = bytes;
+    if (zero) {
+      s->ctx->set_device(g);
+      SKL_CUDA(cudaMemsetAsync(sc.ptr, 0, bytes, s->ctx->D(g).stream));
+    }
+  }
+  return sc.ptr;
+}
+
+}  // namespace
+
+// ------------------------------------------------------------------ creation
+Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int tin, int tin2,
+                  int tout, const int* extra, int nextra, int d, int boundary, const void* neutral) {
+  if (!src) fail(SKL_ERR_INVALID_ARG, "customising function source is NULL");
+  auto s = std::make_unique<Skel>();
+  s->ctx = ctx;
+  s->kind = kind;
+  s->user_src = src;
+  s->entry = (entry && *entry) ? std::string(entry) : detect_entry(s->user_src);
+  s->tin = tin;
+  s->tin2 = tin2;
+  s->tout = tout;
+  for (int i = 0; i < nextra; ++i) s->extra.push_back(extra[i]);
+  s->d = d;
+  s->boundary = boundary;
+  const std::string user = "\n// ---- customising function (user source)\n#line 1 \"user_source\"\n" +
+                           s->user_src + "\n#line 1 \"skeleton_template\"\n";
+  std::string defs = defs_common(ctx, s->entry);
+  std::string body;
+  switch (kind) {
+    case K_MAP:
+    case K_ZIP: {
+      const size_t si = ctx->type(tin).size;
+      const size_t si2 = kind == K_ZIP ? ctx->type(tin2).size : 0;
+      const size_t so = tout == SKL_VOID ? 0 : ctx->type(tout).size;
+      if (si == 0 || (kind == K_ZIP && si2 == 0)) fail(SKL_ERR_TYPE, "void input type");
+      const size_t vec = std::min<size_t>(vec_for({si, si2, so}), 64);
+      defs += "#define SKL_TIN " + tname(ctx, tin) + "\n";
+      if (kind == K_ZIP) defs += "#define SKL_TIN2 " + tname(ctx, tin2) + "\n#define SKL_ZIP 1\n";
+      else defs += "#define SKL_ZIP 0\n";
+      if (tout == SKL_VOID) defs += "#define SKL_TOUT void\n#define SKL_OUT_VOID 1\n";
+      else defs += "#define SKL_TOUT " + tname(ctx, tout) + "\n#define SKL_OUT_VOID 0\n";
+      defs += "#define SKL_VEC " + std::to_string(vec) + "\n";
+      defs += "#define SKL_UNROLL " + std::to_string(ctx->map_unroll) + "\n";
+      std::string xp, xa;
+      for (size_t k = 0; k < s->extra.size(); ++k) {
+        const int t = s->extra[k];
+        const bool ptr = (t & SKL_PTR) != 0;
+        const int base = t & ~SKL_PTR;
+        if (ctx->type(base).size == 0) fail(SKL_ERR_TYPE, "void extra argument");
+        xp += ", " + tname(ctx, base) + (ptr ? "* " : " ") + "skl_x" + std::to_string(k);
+        xa += ", skl_x" + std::to_string(k);
+      }
+      defs += "#define SKL_XPARAMS " + xp + "\n#define SKL_XARGS " + xa + "\n";
+      body = user + kernel_template("common.cuh") + kernel_template("map.cuh");
+      break;
+    }
+    case K_REDUCE:
+    case K_SCAN: {
+      const size_t st = ctx->type(tin).size;
+      if (st == 0) fail(SKL_ERR_TYPE, "void element type");
+      defs += "#define SKL_T " + tname(ctx, tin) + "\n";
+      const int rvec = (16 % st == 0) ? (int)(16 / st) : 1;
+      defs += "#define SKL_RVEC " + std::to_string(rvec) + "\n#define SKL_RU 4\n";
+      if (kind == K_SCAN) {
+        // 8 chunks (128 B) per thread: 8192 fp32 elements per tile (SURVEY §7 hard part 2)
+        const int ch = (16 % st == 0) ? 8 : 0;
+        const int items = ch ? (int)(ch * 16 / st) : 8;
+        defs += "#define SKL_CH " + std::to_string(ch) + "\n#define SKL_ITEMS " + std::to_string(items) + "\n";
+      }
+      body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +
+             kernel_template("reduce.cuh") + (kind == K_SCAN ? kernel_template("scan.cuh") : "");
+      break;
+    }
+    case K_MAPOVERLAP: {
+      const size_t si = ctx->type(tin).size, so = ctx->type(tout).size;
+      if (si == 0 || so == 0) fail(SKL_ERR_TYPE, "MapOverlap needs non-void types");
+      if (16 % si != 0) fail(SKL_ERR_TYPE, "MapOverlap element size must divide 16 bytes");
+      if (d < 0) fail(SKL_ERR_INVALID_ARG, "negative overlap size");
+      if (boundary != SKL_NEUTRAL && boundary != SKL_NEAREST) fail(SKL_ERR_INVALID_ARG, "bad boundary mode");
+      s->neutral.assign(si, 0);
+      if (neutral) std::memcpy(s->neutral.data(), neutral, si);
+      const int epc = (int)(16 / si);
+      const int A = (int)ceil_div((size_t)d, (size_t)epc) * epc;
+      int cw, rh, tw, th;
+      if (si == 1 || si == 2) { cw = 4; rh = 8; }
+      else if (si == 4) { cw = 2; rh = 8; }
+      else { cw = 1; rh = 4; }
+      const int nthr = ctx->block_threads;
+      tw = 32 * cw;
+      const int rows_thr = nthr / 32;
+      th = rows_thr * rh;
+      while (rh > 1 && (size_t)(th + 2 * d) * (size_t)(tw + 2 * A) * si > 44 * 1024) {
+        rh /= 2;
+        th = rows_thr * rh;
+      }
+      s->mo_tw = tw;
+      s->mo_th = th;
+      s->mo_a = A;
+      s->mo_pitch = tw + 2 * A;
+      defs += "#define SKL_TIN " + tname(ctx, tin) + "\n#define SKL_TOUT " + tname(ctx, tout) + "\n";
+      defs += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(boundary) + "\n";
+      defs += "#define SKL_A " + std::to_string(A) + "\n";
+      defs += "#define SKL_PITCH " + std::to_string(tw + 2 * A) + "\n";
+      defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_TH " + std::to_string(th) + "\n";
+      defs += "#define SKL_CW " + std::to_string(cw) + "\n#define SKL_RH " + std::to_string(rh) + "\n";
+      defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n";
+      defs += "#define SKL_MO1D 0\n";
+      body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
+      // 1-D variant (vector containers), compiled lazily in run_mapoverlap
+      break;
+    }
+    default:
+      fail(SKL_ERR_INVALID_ARG, "unknown skeleton kind");
+  }
+  std::string log;
+  s->prog = compile(ctx, defs + program_source(ctx, body), &log);
+  Skel* raw = s.release();
+  ctx->skels.insert(raw);
+  return raw;
+}
+
+void skel_destroy(Skel* s) {
+  Ctx* ctx = s->ctx;
+  for (auto* m : {&s->scratch_red, &s->scratch_scan, &s->scratch_stage})
+    for (auto& kv : *m)
+      if (kv.second.ptr && ctx->is_local(kv.first)) device_free(ctx, kv.first, kv.second.ptr);
+  for (Cont* c : ctx->conts)
+    if (c->combine == s) c->combine = nullptr;
+  ctx->skels.erase(s);
+  delete s;
+}
+
+// ------------------------------------------------------------------ helpers
+namespace {
+
+Dist default_dist(Cont* c, Dist def) { return c->dist.kind == DNONE ? def : c->dist; }
+// elementwise skeletons compute a container's core: overlap behaves as block
+Dist elementwise(Dist d) { return d.kind == DOVERLAP ? Dist{DBLOCK, 0} : d; }
+
+Cont* output_for(Ctx* ctx, Cont** out, int type, size_t rows, size_t cols, bool matrix) {
+  if (*out) {
+    Cont* o = *out;
+    if (o->type != type) fail(SKL_ERR_TYPE, "output container has the wrong element type");
+    if (o->rows != rows || o->cols != cols) fail(SKL_ERR_SIZE_MISMATCH, "output container has the wrong size");
+    return o;
+  }
+  *out = cont_create(ctx, type, rows, cols, matrix);
+  return *out;
+}
+
+struct ExtraArgs {
+  std::vector<std::vector<unsigned char>> scalars;
+  std::vector<Cont*> conts;
+  std::vector<int> modes;
+};
+
+ExtraArgs prepare_extras(Skel* s, const skl_arg* extra, int nextra) {
+  if (nextra != (int)s->extra.size())
+    fail(SKL_ERR_INVALID_ARG, "skeleton expects " + std::to_string(s->extra.size()) + " extra arguments");
+  ExtraArgs ea;
+  ea.scalars.resize((size_t)nextra);
+  ea.conts.assign((size_t)nextra, nullptr);
+  ea.modes.assign((size_t)nextra, 0);
+  for (int k = 0; k < nextra; ++k) {
+    const int t = s->extra[(size_t)k];
+    const bool ptr = (t & SKL_PTR) != 0;
+    const size_t sz = s->ctx->type(t & ~SKL_PTR).size;
+    if (ptr) {
+      if (extra[k].kind != SKL_ARG_CONT || !extra[k].cont || !extra[k].cont->c)
+        fail(SKL_ERR_INVALID_ARG, "extra argument " + std::to_string(k) + " must be a container");
+      Cont* c = extra[k].cont->c;
+      if (c->elt != sz) fail(SKL_ERR_TYPE, "extra container argument has the wrong element type");
+      // A27: a container argument is read at arbitrary indices: every device needs
+      // the whole container, i.e. the copy distribution.
+      ensure(c, Dist{DCOPY, 0}, false);
+      ea.conts[(size_t)k] = c;
+      ea.modes[(size_t)k] = extra[k].mode ? extra[k].mode : SKL_READ;
+    } else {
+      if (extra[k].kind != SKL_ARG_SCALAR || !extra[k].value || extra[k].bytes != sz)
+        fail(SKL_ERR_INVALID_ARG, "extra argument " + std::to_string(k) + " must be a scalar of " +
+                                      std::to_string(sz) + " bytes");
+      ea.scalars[(size_t)k].assign((const unsigned char*)extra[k].value,
+                                   (const unsigned char*)extra[k].value + sz);
+    }
+  }
+  return ea;
+}
+
+void finish_extras(Ctx* ctx, ExtraArgs& ea, int ndev_exec) {
+  for (size_t k = 0; k < ea.conts.size(); ++k) {
+    Cont* c = ea.conts[k];
+    if (!c || !(ea.modes[k] & SKL_WRITE)) continue;
+    c->host_valid = false;
+    if (ndev_exec > 1 || ctx->G > 1) c->diverged = true;  // replicas written independently (A25)
+  }
+}
+
+}  // namespace
+
+// ------------------------------------------------------------------ Map / Zip
+static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_arg* extra,
+                            int nextra) {
+  Ctx* ctx = s->ctx;
+  if (in->type != s->tin && in->elt != ctx->type(s->tin).size)
+    fail(SKL_ERR_TYPE, "input container type does not match the skeleton");
+  if (in2) {
+    if (in2->elt != ctx->type(s->tin2).size) fail(SKL_ERR_TYPE, "right input type mismatch");
+    if (in2->rows * in2->cols != in->rows * in->cols || in2->rows != in->rows)
+      fail(SKL_ERR_SIZE_MISMATCH, "zip inputs differ in size (P:L257-259)");
+  }
+  const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));  // A6
+  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  if (in2) {
+    // A7: the right input follows the left input's distribution
+    if (!(elementwise(in2->dist) == din && in2->dev_valid)) ensure(in2, din, false);
+    else ensure(in2, in2->dist, false);
+  }
+  ExtraArgs ea = prepare_extras(s, extra, nextra);
+  Cont* o = nullptr;
+  if (s->tout != SKL_VOID) {
+    o = output_for(ctx, out, s->tout, in->rows, in->cols, in->matrix);
+    if (o == in && !(in->dist == din)) fail(SKL_ERR_INVALID_ARG, "in-place call needs a block/copy/single input");
+    prepare_output(o, din, 0);
+  }
+  const size_t vec = std::min<size_t>(
+      vec_for({ctx->type(s->tin).size, in2 ? ctx->type(s->tin2).size : 0,
+               s->tout == SKL_VOID ? 0 : ctx->type(s->tout).size}), 64);
+  const size_t per_block = (size_t)ctx->block_threads * (size_t)ctx->map_unroll;
+  int ndev = 0;
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range r = core_range(in->units(), ctx->G, din, g);
+    if (r.empty()) continue;
+    ++ndev;
+    const void* pin = part_ptr(in, g, r.lo);
+    const void* pin2 = in2 ? part_ptr(in2, g, r.lo) : nullptr;
+    void* pout = o ? part_ptr(o, g, r.lo) : nullptr;
+    unsigned long long n = (unsigned long long)(r.size() * in->cols);
+    const bool vec_ok = aligned16(pin) && (!in2 || aligned16(pin2)) && (!o || aligned16(pout));
+    std::vector<void*> args;
+    args.push_back(&pin);
+    if (in2) args.push_back(&pin2);
+    args.push_back(&pout);
+    args.push_back(&n);
+    std::vector<void*> xptr(ea.conts.size(), nullptr);
+    for (size_t k = 0; k < ea.conts.size(); ++k) {
+      if (ea.conts[k]) {
+        xptr[k] = part_ptr(ea.conts[k], g, 0);
+        args.push_back(&xptr[k]);
+      } else {
+        args.push_back(ea.scalars[k].data());
+      }
+    }
+    size_t grid;
+    const char* kname;
+    if (vec_ok) {
+      grid = std::max<size_t>(1, ceil_div(n / vec, per_block));
+      kname = "skl_map_vec";
+    } else {
+      grid = ceil_div(n, per_block);
+      kname = "skl_map_sc";
+    }
+    launch(ctx, g, s->prog, kname, dim3((unsigned)grid), dim3(ctx->block_threads), 0, args.data());
+  }
+  if (o) mark_written(o);
+  finish_extras(ctx, ea, ndev);
+}
+
+void run_map(Skel* s, Cont* in, Cont** out, const skl_arg* extra, int nextra) {
+  if (s->kind != K_MAP) fail(SKL_ERR_INVALID_ARG, "not a Map skeleton");
+  run_elementwise(s, in, nullptr, out, extra, nextra);
+}
+void run_zip(Skel* s, Cont* l, Cont* r, Cont** out, const skl_arg* extra, int nextra) {
+  if (s->kind != K_ZIP) fail(SKL_ERR_INVALID_ARG, "not a Zip skeleton");
+  if (!r) fail(SKL_ERR_INVALID_ARG, "zip needs two inputs");
+  run_elementwise(s, l, r, out, extra, nextra);
+}
+
+// ------------------------------------------------------------------ Reduce
+// One device's fold of n elements at `in` into `result` (device pointer).
+static void reduce_on_device(Skel* s, int g, const void* in, size_t n, void* result) {
+  Ctx* ctx = s->ctx;
+  const size_t st = ctx->type(s->tin).size;
+  const int nw = ctx->block_threads / 32;
+  const bool vec = (16 % st == 0) && aligned16(in);
+  const size_t rtile = 32 * (vec ? 16 / st : 1);
+  const size_t ru = 4;
+  const size_t max_blocks = (size_t)ctx->D(g).sm_count * (2048 / (size_t)ctx->block_threads);
+  size_t nblocks = std::min(max_blocks, std::max<size_t>(1, ceil_div(n, (size_t)nw * rtile * ru)));
+  size_t wseg = ceil_div(ceil_div(n, nblocks * (size_t)nw), rtile) * rtile;
+  nblocks = ceil_div(n, (size_t)nw * wseg);
+  // scratch: [counter (16 B)] [partials]
+  char* sc = (char*)scratch(s, s->scratch_red, g, 16 + max_blocks * std::max<size_t>(st, 8), true);
+  void* counter = sc;
+  void* partials = sc + 16;
+  unsigned long long nn = n, ws = wseg;
+  void* args[] = {(void*)&in, &nn, &ws, &partials, &counter, &result};
+  launch(ctx, g, s->prog, vec ? "skl_reduce_vec" : "skl_reduce_sc", dim3((unsigned)nblocks),
+         dim3(ctx->block_threads), 0, args);
+}
+
+void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
+                 size_t nelem) {
+  if (!s || (s->kind != K_REDUCE && s->kind != K_SCAN)) fail(SKL_ERR_INVALID_ARG, "combine needs a Reduce skeleton");
+  Ctx* ctx = s->ctx;
+  unsigned long long stride = stride_elems, n = nelem;
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(nelem, (size_t)ctx->block_threads),
+                                                           (size_t)ctx->D(g).sm_count * 8));
+  void* args[] = {(void*)&staging, &stride, &nrep, &dst, &n};
+  launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(ctx->block_threads), 0, args);
+}
+
+void run_reduce(Skel* s, Cont* in, Cont** out) {
+  if (s->kind != K_REDUCE) fail(SKL_ERR_INVALID_ARG, "not a Reduce skeleton");
+  Ctx* ctx = s->ctx;
+  if (in->elt != ctx->type(s->tin).size) fail(SKL_ERR_TYPE, "input type does not match the skeleton");
+  if (in->rows * in->cols == 0) fail(SKL_ERR_EMPTY, "reduce of an empty container (A11)");
+  if (in->dist.kind == DCOPY && in->diverged && in->combine) ensure(in, Dist{DCOPY, 0}, false);
+  const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));
+  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  Cont* o = output_for(ctx, out, s->tin, 1, 1, false);
+  // participants, in device order: devices whose core holds elements.  A copy
+  // input is reduced once per process (replicas are identical).
+  std::vector<int> parts;
+  for (int g = 0; g < ctx->G; ++g) {
+    if (din.kind == DCOPY) {
+      if (ctx->dist_mode ? g == ctx->first_local : g == 0) parts.push_back(g);
+      continue;
+    }
+    if (!core_range(in->units(), ctx->G, din, g).empty()) parts.push_back(g);
+  }
+  // result distribution: single(first participant) in one process; copy across
+  // processes so every rank's getValue() works (SPMD).
+  const bool cross = parts.size() > 1;
+  Dist dout = ctx->dist_mode ? Dist{DCOPY, 0} : Dist{DSINGLE, parts[0]};
+  if (!ctx->dist_mode && cross) dout = Dist{DSINGLE, 0};
+  prepare_output(o, dout, 0);
+  const size_t st = in->elt;
+  if (!cross) {
+    // one device computes everything
+    for (int g : parts) {
+      if (!ctx->is_local(g)) continue;
+      const Range r = core_range(in->units(), ctx->G, din, g);
+      reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, part_ptr(o, g, 0));
+    }
+    mark_written(o);
+    return;
+  }
+  // per-device partials (into slot p of a staging row), then gather + ordered fold
+  const int P = (int)parts.size();
+  std::map<int, void*> stage;  // device -> [P] staging
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g)
+    stage[g] = scratch(s, s->scratch_stage, g, (size_t)P * std::max<size_t>(st, 8) + 64, false);
+  std::vector<int> dsts;
+  if (dout.kind == DSINGLE) dsts.push_back(dout.arg);
+  else for (int g = 0; g < ctx->G; ++g) dsts.push_back(g);
+  for (int i = 0; i < P; ++i) {
+    const int g = parts[(size_t)i];
+    if (!ctx->is_local(g)) continue;
+    const Range r = core_range(in->units(), ctx->G, din, g);
+    // partial lands in its own slot i on its own device
+    reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, (char*)stage[g] + (size_t)i * st);
+  }
+  std::vector<Transfer> tr;
+  for (int dg : dsts)
+    for (int i = 0; i < P; ++i)
+      if (parts[(size_t)i] != dg) tr.push_back(Transfer{parts[(size_t)i], dg, 0, 0, 1, i});
+  struct SPtr : PtrFn {
+    std::map<int, void*>* stage;
+    size_t st;
+    void* src(const Transfer& t) override { return (char*)(*stage)[t.src] + (size_t)t.slot * st; }
+    void* dst(const Transfer& t) override { return (char*)(*stage)[t.dst] + (size_t)t.slot * st; }
+  } sp;
+  sp.stage = &stage;
+  sp.st = st;
+  run_transfers(ctx, tr, st, sp);
+  for (int dg : dsts)
+    if (ctx->is_local(dg)) run_combine(s, dg, stage[dg], 1, P, part_ptr(o, dg, 0), 1);
+  mark_written(o);
+}
+
+// ------------------------------------------------------------------ Scan
+void run_scan(Skel* s, Cont* in, Cont** out) {
+  if (s->kind != K_SCAN) fail(SKL_ERR_INVALID_ARG, "not a Scan skeleton");
+  Ctx* ctx = s->ctx;
+  if (in->elt != ctx->type(s->tin).size) fail(SKL_ERR_TYPE, "input type does not match the skeleton");
+  if (in->rows * in->cols == 0) fail(SKL_ERR_EMPTY, "scan of an empty container");
+  if (in->dist.kind == DCOPY && in->diverged && in->combine) ensure(in, Dist{DCOPY, 0}, false);
+  const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));
+  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  Cont* o = output_for(ctx, out, s->tin, in->rows, in->cols, in->matrix);
+  if (o == in) fail(SKL_ERR_INVALID_ARG, "scan cannot run in place");
+  prepare_output(o, din, 0);
+  const size_t st = in->elt;
+  const bool chunked = (16 % st == 0);
+  const int items = chunked ? (int)(8 * 16 / st) : 8;
+  const size_t tile = (size_t)ctx->block_threads * (size_t)items;
+  // participants with distinct data (block / single); copy scans whole on each device
+  std::vector<int> parts;
+  for (int g = 0; g < ctx->G; ++g)
+    if (!core_range(in->units(), ctx->G, din, g).empty()) parts.push_back(g);
+  const bool carry = din.kind == DBLOCK && parts.size() > 1;
+  const int P = (int)parts.size();
+  std::map<int, void*> totals;
+  if (carry) {
+    // pass 1: device totals (order-preserving reduce), all-gathered so device g
+    // folds t_0 .. t_{g-1} as its carry-in
+    for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g)
+      totals[g] = scratch(s, s->scratch_stage, g, (size_t)P * std::max<size_t>(st, 8) + 64, false);
+    for (int i = 0; i < P; ++i) {
+      const int g = parts[(size_t)i];
+      if (!ctx->is_local(g)) continue;
+      const Range r = core_range(in->units(), ctx->G, din, g);
+      reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, (char*)totals[g] + (size_t)i * st);
+    }
+    std::vector<Transfer> tr;
+    for (int j = 0; j < P; ++j)
+      for (int i = 0; i < j; ++i) tr.push_back(Transfer{parts[(size_t)i], parts[(size_t)j], 0, 0, 1, i});
+    struct TPtr : PtrFn {
+      std::map<int, void*>* t;
+      size_t st;
+      void* src(const Transfer& x) override { return (char*)(*t)[x.src] + (size_t)x.slot * st; }
+      void* dst(const Transfer& x) override { return (char*)(*t)[x.dst] + (size_t)x.slot * st; }
+    } tp;
+    tp.t = &totals;
+    tp.st = st;
+    run_transfers(ctx, tr, st, tp);
+  }
+  for (int i = 0; i < P; ++i) {
+    const int g = parts[(size_t)i];
+    if (!ctx->is_local(g)) continue;
+    const Range r = core_range(in->units(), ctx->G, din, g);
+    const size_t n = r.size() * in->cols;
+    const size_t ntiles = ceil_div(n, tile);
+    // status: [flags u32 x ntiles] [aggs T x ntiles] [incls T x ntiles], 16-B aligned
+    const size_t fbytes = ceil_div(ntiles * 4, 16) * 16, tbytes = ceil_div(ntiles * st, 16) * 16;
+    Scratch& sc = s->scratch_scan[g];
+    const bool fresh = sc.bytes < fbytes + 2 * tbytes;
+    char* base = (char*)scratch(s, s->scratch_scan, g, fbytes + 2 * tbytes, true);
+    if (fresh) s->epoch[g] = 0;  // zeroed flags: every epoch >= 1 is new
+    unsigned ep = ++s->epoch[g];
+    if (ep >= (1u << 30)) {
+      ctx->set_device(g);
+      SKL_CUDA(cudaMemsetAsync(base, 0, fbytes, ctx->D(g).stream));
+      ep = s->epoch[g] = 1;
+    }
+    void* flags = base;
+    void* aggs = base + fbytes;
+    void* incls = base + fbytes + tbytes;
+    const void* pin = part_ptr(in, g, r.lo);
+    void* pout = part_ptr(o, g, r.lo);
+    unsigned long long nn = n;
+    const void* cptr = carry ? totals[g] : nullptr;
+    int ncarry = carry ? i : 0;
+    void* args[] = {(void*)&pin, &pout, &nn, &flags, &aggs, &incls, &ep, (void*)&cptr, &ncarry};
+    const bool vec = chunked && aligned16(pin) && aligned16(pout);
+    launch(ctx, g, s->prog, vec ? "skl_scan_vec" : "skl_scan_sc", dim3((unsigned)ntiles),
+           dim3(ctx->block_threads), 0, args);
+  }
+  mark_written(o);
+}
+
+// ------------------------------------------------------------------ MapOverlap
+void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
+  if (s->kind != K_MAPOVERLAP) fail(SKL_ERR_INVALID_ARG, "not a MapOverlap skeleton");
+  Ctx* ctx = s->ctx;
+  if (in->elt != ctx->type(s->tin).size) fail(SKL_ERR_TYPE, "input type does not match the skeleton");
+  const int d = s->d;
+  // A4/A6: the input must be overlap(d' >= d) (or copy / single, computed whole)
+  Dist din = in->dist;
+  if (din.kind == DNONE || din.kind == DBLOCK || (din.kind == DOVERLAP && din.arg < d))
+    din = Dist{DOVERLAP, d};
+  ensure(in, din, true);
+  const Dist dout = (din.kind == DOVERLAP) ? Dist{DBLOCK, 0} : din;
+  Cont* o = output_for(ctx, out, s->tout, in->rows, in->cols, in->matrix);
+  if (o == in) fail(SKL_ERR_INVALID_ARG, "MapOverlap cannot run in place");
+  prepare_output(o, dout, dout.kind == DBLOCK ? (size_t)d : 0);
+  const size_t si = in->elt, so = o->elt;
+  if (in->matrix) {
+    for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+      const Range r = core_range(in->units(), ctx->G, dout, g);
+      if (r.empty()) continue;
+      Part& pi = in->parts[(size_t)g];
+      Part& po = o->parts[(size_t)g];
+      const void* pin = pi.ptr;
+      void* pout = po.ptr;
+      long in_row0 = (long)pi.buf.lo, in_rows = (long)pi.buf.size(), out_row0 = (long)po.buf.lo;
+      long R = (long)in->rows, C = (long)in->cols, rb = (long)r.lo, re = (long)r.hi;
+      const int cw = s->mo_tw / 32;
+      int vec_ok = ((size_t)C * si) % 16 == 0 && aligned16(pin) && ((size_t)C * so) % ((size_t)cw * so) == 0 &&
+                   ((uintptr_t)pout % ((size_t)cw * so) == 0);
+      void* args[] = {(void*)&pin, &in_row0, &in_rows, &pout, &out_row0, &R, &C, &rb, &re,
+                      s->neutral.data(), &vec_ok};
+      const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
+                      (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
+      launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(ctx->block_threads), 0, args);
+    }
+  } else {
+    // vector form: compile the 1-D variant once
+    if (!s->prog1d) {
+      const size_t epc = 16 / si;
+      const int A = (int)(ceil_div((size_t)d, epc) * epc);
+      const int cw = 4, tw = ctx->block_threads * cw;
+      std::string defs = defs_common(ctx, s->entry);
+      defs += "#define SKL_TIN " + tname(ctx, s->tin) + "\n#define SKL_TOUT " + tname(ctx, s->tout) + "\n";
+      defs += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(s->boundary) + "\n";
+      defs += "#define SKL_A " + std::to_string(A) + "\n#define SKL_PITCH 0\n";
+      defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_TH 1\n#define SKL_CW " +
+              std::to_string(cw) + "\n#define SKL_RH 1\n#define SKL_MO1D 1\n#define SKL_OUTB " +
+              std::to_string((size_t)cw * ctx->type(s->tout).size) + "\n";
+      const std::string user = "\n#line 1 \"user_source\"\n" + s->user_src + "\n#line 1 \"skeleton_template\"\n";
+      s->prog1d = compile(ctx, defs + program_source(ctx, user + kernel_template("common.cuh") +
+                                                                   kernel_template("mapoverlap.cuh")),
+                                nullptr);
+      s->mo_1d = true;
+    }
+    const int tw = ctx->block_threads * 4;
+    for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+      const Range r = core_range(in->units(), ctx->G, dout, g);
+      if (r.empty()) continue;
+      Part& pi = in->parts[(size_t)g];
+      Part& po = o->parts[(size_t)g];
+      const void* pin = pi.ptr;
+      void* pout = po.ptr;
+      long in_lo = (long)pi.buf.lo, in_n = (long)pi.buf.size(), out_lo = (long)po.buf.lo;
+      long N = (long)in->rows, unused = 0, rb = (long)r.lo, re = (long)r.hi;
+      int vec_ok = aligned16(pin);
+      void* args[] = {(void*)&pin, &in_lo, &in_n, &pout, &out_lo, &N, &unused, &rb, &re,
+                      s->neutral.data(), &vec_ok};
+      launch(ctx, g, s->prog1d, "skl_mo1d", dim3((unsigned)ceil_div(r.size(), (size_t)tw)),
+             dim3(ctx->block_threads), 0, args);
+    }
+  }
+  mark_written(o);
+  if (ctx->debug_bounds) check_debug_flag(ctx);
+}
+
+void check_debug_flag(Ctx* ctx) {
+  extern bool read_and_clear_bounds_flags(Ctx*);
+  if (read_and_clear_bounds_flags(ctx))
+    fail(SKL_ERR_OUT_OF_RANGE, "get() accessed an element beyond the overlap range d (P:L362-368)");
+}
+
+}  // namespace skl

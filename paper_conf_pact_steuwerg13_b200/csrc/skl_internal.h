@@ -1,0 +1,236 @@
+// skl_internal.h — internal data model of libskl.so (not installed).
+//
+// Layers (SURVEY.md §1 "New build"): B1 device context (Ctx), B2 containers +
+// coherence (Cont, Part), B3 distribution planner + redistribution (plan.cpp,
+// container.cpp), B4 NVRTC customisation compiler (compiler.cpp), B5 skeleton
+// executors (skeletons.cpp, kernels/*.cuh), B6 C ABI (capi.cpp, include/skl.h).
+#pragma once
+
+#include <cuda_runtime.h>
+
+#include <atomic>
+#include <cstdint>
+#include <cstring>
+#include <map>
+#include <memory>
+#include <mutex>
+#include <set>
+#include <stdexcept>
+#include <string>
+#include <vector>
+
+#include "../../include/skl.h"
+
+namespace skl {
+
+// ------------------------------------------------------------------ errors
+struct Error : std::runtime_error {
+  int code;
+  Error(int c, const std::string& m) : std::runtime_error(m), code(c) {}
+};
+[[noreturn]] void fail(int code, const std::string& msg);
+void cuda_check(cudaError_t e, const char* what);
+#define SKL_CUDA(x) ::skl::cuda_check((x), #x)
+
+// ------------------------------------------------------------------ types
+struct TypeInfo {
+  std::string name;  // C spelling used in generated source
+  size_t size = 0, align = 1;
+  std::string decl;  // struct declaration ("" for builtins)
+};
+
+// ------------------------------------------------------------------ distributions
+enum DistKind { DNONE = SKL_DIST_NONE, DSINGLE = SKL_SINGLE, DCOPY = SKL_COPY,
+                DBLOCK = SKL_BLOCK, DOVERLAP = SKL_OVERLAP };
+struct Dist {
+  int kind = DNONE;
+  int arg = 0;  // device (single) or overlap size d (overlap)
+  bool operator==(const Dist& o) const { return kind == o.kind && arg == o.arg; }
+};
+struct Range {
+  size_t lo = 0, hi = 0;
+  size_t size() const { return hi > lo ? hi - lo : 0; }
+  bool empty() const { return hi <= lo; }
+  bool contains(const Range& r) const { return r.empty() || (lo <= r.lo && r.hi <= hi); }
+};
+// plan.cpp — pure host arithmetic (readings A1-A3)
+Range block_range(size_t units, int G, int g);
+Range core_range(size_t units, int G, const Dist& d, int g);  // units device g owns/computes
+Range need_range(size_t units, int G, const Dist& d, int g);   // units g stores (with halo)
+struct Transfer {
+  int src, dst;      // global devices
+  size_t src_unit;   // first unit (global index) read from src's part
+  size_t dst_unit;   // first unit (global index) written into dst's part
+  size_t n;          // units
+  int slot = 0;      // staging slot (combine gathers), else 0
+};
+// Transfers turning distribution `from` (all of its need ranges valid, or only
+// core ranges when from_core_only) into `to` (need ranges incl. halo when
+// to_halo).  Units already present on the destination device are not moved.
+std::vector<Transfer> plan_transfers(size_t units, int G, const Dist& from, bool from_halo_valid,
+                                     const Dist& to, bool to_halo);
+
+// ------------------------------------------------------------------ compiler
+// One NVRTC-compiled module per distinct source text.  A cudaLibrary is context
+// independent, so one load serves every device.
+struct Program {
+  std::string source;
+  std::vector<char> cubin;
+  cudaLibrary_t lib = nullptr;
+  std::map<std::string, cudaKernel_t> kernels;
+  std::map<std::string, size_t> smem_set;  // dynamic smem attribute already raised
+};
+
+// ------------------------------------------------------------------ devices
+struct Device {
+  int global = 0;      // global device index g
+  int phys = 0;        // CUDA ordinal
+  cudaStream_t own = nullptr, stream = nullptr;  // library stream, current stream
+  cudaEvent_t ev = nullptr;                      // scratch event for cross-stream sync
+  int sm_count = 148;
+};
+
+struct Cont;
+struct Skel;
+
+struct Ctx {
+  int G = 1;                   // global devices
+  int first_local = 0, nlocal = 1;
+  bool dist_mode = false;      // one process per GPU, NCCL between ranks
+  bool offline = false;        // no devices: compile only (skl_init_offline)
+  int rank = 0, world = 1;
+  void* nccl_comm = nullptr;   // ncclComm_t
+  std::vector<Device> dev;     // local devices, index g - first_local
+  std::vector<TypeInfo> types; // index = skl_type (builtins first)
+  std::set<Cont*> conts;
+  std::set<Skel*> skels;
+  // options
+  int block_threads = 256;
+  int debug_bounds = 0;
+  int map_unroll = 4;
+  // counters
+  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0};
+  // NVRTC cache: source hash -> program
+  std::map<std::string, std::unique_ptr<Program>> programs;
+  // builtin kernels (fill) per element size
+  bool is_local(int g) const { return g >= first_local && g < first_local + nlocal; }
+  Device& D(int g) { return dev.at((size_t)(g - first_local)); }
+  const TypeInfo& type(int t) const;
+  void set_device(int g);
+};
+
+// ------------------------------------------------------------------ containers
+struct Part {
+  void* ptr = nullptr;  // device buffer; addresses unit buf.lo
+  Range buf;            // units the buffer covers
+  Range valid;          // units holding valid data (subset of buf)
+  size_t cap_bytes = 0;
+};
+
+struct Cont {
+  Ctx* ctx = nullptr;
+  int type = 0;
+  size_t elt = 0;          // element bytes
+  bool matrix = false;
+  size_t rows = 0, cols = 1;  // vector: rows = n, cols = 1
+  size_t units() const { return rows; }
+  size_t unit_bytes() const { return cols * elt; }
+  size_t bytes() const { return rows * cols * elt; }
+  Dist dist;
+  bool dev_valid = false;    // core ranges of `dist` valid on every device
+  bool halo_valid = false;   // overlap halos valid too
+  bool diverged = false;     // copy replicas written independently
+  Skel* combine = nullptr;   // copy(+) combine function (A25)
+  std::vector<Part> parts;   // indexed by global device; only local ones used
+  void* host = nullptr;      // pinned host mirror (lazily allocated)
+  bool host_valid = false;
+  size_t spare_halo = 0;     // allocate parts with this many extra halo units
+};
+
+// container.cpp
+Cont* cont_create(Ctx* ctx, int type, size_t rows, size_t cols, bool matrix);
+void cont_destroy(Cont* c);
+// Make `c` hold valid data in distribution `d` on the devices (upload from the
+// host mirror or redistribute device-to-device as needed).  `halo` = overlap
+// halos must be valid too.
+void ensure(Cont* c, const Dist& d, bool halo);
+// Prepare `c` as an output in distribution `d` (contents will be overwritten on
+// the core ranges); allocates parts with `spare` halo units of room.
+void prepare_output(Cont* c, const Dist& d, size_t spare);
+void mark_written(Cont* c);  // devices valid, host stale, halos stale
+void* part_ptr(Cont* c, int g, size_t unit);  // device pointer to global unit on device g
+void host_upload(Cont* c, const void* host);  // into current distribution
+void host_download(Cont* c, void* host);      // whole container (collective)
+void download_part(Cont* c, int g, void* host, size_t* first, size_t* n);
+void fill(Cont* c, const void* value);
+void* host_mirror(Cont* c, int mode);
+void copy_combine_to_copy(Cont* c);  // fold diverged replicas, keep copy
+
+// comm.cpp — execute transfers between per-device buffers.  srcp/dstp resolve
+// (device, unit) to a device pointer for LOCAL devices.
+struct PtrFn {
+  virtual void* src(const Transfer& t) = 0;  // local t.src only
+  virtual void* dst(const Transfer& t) = 0;  // local t.dst only
+  virtual ~PtrFn() = default;
+};
+void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes, PtrFn& p);
+void barrier_streams(Ctx* ctx);  // every local stream waits for every other
+// NCCL (dlopen)
+void nccl_get_unique_id(void* out128);
+void nccl_init(Ctx* ctx, const void* id);
+void nccl_destroy(Ctx* ctx);
+
+// ------------------------------------------------------------------ compiler.cpp
+std::string program_source(Ctx* ctx, const std::string& body);
+Program* compile(Ctx* ctx, const std::string& source, std::string* log_out);
+void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 block,
+            size_t smem, void** args);
+int max_smem_optin(Ctx* ctx, int g);
+std::string detect_entry(const std::string& src);
+std::string kernel_template(const char* name);  // embedded kernels/*.cuh
+
+// ------------------------------------------------------------------ skeletons
+enum SkelKind { K_MAP = 1, K_ZIP, K_REDUCE, K_SCAN, K_MAPOVERLAP };
+struct Scratch {  // per-device persistent scratch (reduce partials, scan status)
+  void* ptr = nullptr;
+  size_t bytes = 0;
+};
+struct Skel {
+  Ctx* ctx = nullptr;
+  int kind = 0;
+  std::string user_src, entry;
+  int tin = 0, tin2 = 0, tout = 0;
+  std::vector<int> extra;  // extra arg types (with SKL_PTR flag)
+  int d = 0, boundary = 0;
+  std::vector<unsigned char> neutral;
+  Program* prog = nullptr;
+  Program* prog1d = nullptr;        // MapOverlap on vectors (compiled lazily)
+  std::map<int, Scratch> scratch_red;    // per device: reduce ticket counter + block partials
+  std::map<int, Scratch> scratch_scan;   // per device: decoupled look-back status
+  std::map<int, Scratch> scratch_stage;  // per device: cross-device partials / totals
+  std::map<int, uint32_t> epoch;    // scan lookback epochs per device
+  // MapOverlap tile geometry (compile-time constants of prog)
+  int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0;
+  bool mo_1d = false;
+};
+Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int tin, int tin2,
+                  int tout, const int* extra, int nextra, int d, int boundary, const void* neutral);
+void skel_destroy(Skel* s);
+void run_map(Skel* s, Cont* in, Cont** out, const skl_arg* extra, int nextra);
+void run_zip(Skel* s, Cont* l, Cont* r, Cont** out, const skl_arg* extra, int nextra);
+void run_reduce(Skel* s, Cont* in, Cont** out);
+void run_scan(Skel* s, Cont* in, Cont** out);
+void run_mapoverlap(Skel* s, Cont* in, Cont** out);
+// ordered combine of G staged replica slices into dst (A25), on device g
+void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
+                 size_t nelem);
+void* device_alloc(Ctx* ctx, int g, size_t bytes);
+void device_free(Ctx* ctx, int g, void* p);
+void check_debug_flag(Ctx* ctx);
+
+}  // namespace skl
+
+// C handles (include/skl.h) wrap the internal objects.
+struct skl_ctx { skl::Ctx* c; };
+struct skl_cont { skl::Cont* c; };
+struct skl_skel { skl::Skel* s; };
