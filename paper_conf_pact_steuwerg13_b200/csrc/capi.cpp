@@ -339,6 +339,8 @@ skl_status skl_local_part(skl_cont* c, int g, void** dptr, size_t* first_unit, s
     if (first_unit) *first_unit = 0;
     if (nunits) *nunits = 0;
     if (g < 0 || g >= k->ctx->G || !k->ctx->is_local(g)) return;
+    // a distribution set on host data becomes resident here (implicit upload)
+    if (k->dist.kind != DNONE && !k->dev_valid && k->host_valid) ensure(k, k->dist, k->dist.kind == DOVERLAP);
     Part& p = k->parts[(size_t)g];
     if (!p.ptr || p.valid.empty() || !k->dev_valid) return;
     *dptr = part_ptr(k, g, p.valid.lo);

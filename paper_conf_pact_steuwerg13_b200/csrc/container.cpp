@@ -280,6 +280,12 @@ static void combine_to_block(Cont* c) {
   const int G = ctx->G;
   const size_t U = c->units(), ub = c->unit_bytes();
   const Dist blk{DBLOCK, 0};
+  if (G == 1) {  // the fold of a single replica is the replica itself
+    c->dist = blk;
+    c->diverged = false;
+    set_valid(c, blk, false);
+    return;
+  }
   std::vector<void*> staging((size_t)G, nullptr);
   std::vector<Transfer> tr;
   for (int g = 0; g < G; ++g) {

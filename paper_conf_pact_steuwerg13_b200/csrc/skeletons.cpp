@@ -247,7 +247,8 @@ void finish_extras(Ctx* ctx, ExtraArgs& ea, int ndev_exec) {
     Cont* c = ea.conts[k];
     if (!c || !(ea.modes[k] & SKL_WRITE)) continue;
     c->host_valid = false;
-    if (ndev_exec > 1 || ctx->G > 1) c->diverged = true;  // replicas written independently (A25)
+    // replicas written independently (A25); one device: its replica is the fold
+    if (ctx->G > 1 && ndev_exec >= 1) c->diverged = true;
   }
 }
 
