@@ -163,6 +163,25 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->block_threads = (int)value;
     } else if (k == "debug_bounds") {
       c->debug_bounds = value ? 1 : 0;
+    } else if (k == "scan_chunks") {
+      if (value != 2 && value != 4 && value != 8) fail(SKL_ERR_INVALID_ARG, "scan_chunks in {2,4,8}");
+      c->scan_chunks = (int)value;
+    } else if (k == "scan_sub") {
+      if (value < 1 || value > 64) fail(SKL_ERR_INVALID_ARG, "scan_sub in [1,64]");
+      c->scan_sub = (int)value;
+    } else if (k == "scan_fstride") {
+      if (value < 1 || value > 64) fail(SKL_ERR_INVALID_ARG, "scan_fstride in [1,64]");
+      c->scan_fstride = (int)value;
+    } else if (k == "scan_spin_ns") {
+      if (value < 0 || value > 100000) fail(SKL_ERR_INVALID_ARG, "scan_spin_ns in [0,100000]");
+      c->scan_spin_ns = (int)value;
+    } else if (k == "scan_minb") {
+      if (value < 1 || value > 32) fail(SKL_ERR_INVALID_ARG, "scan_minb in [1,32]");
+      c->scan_minb = (int)value;
+    } else if (k == "scan_variant") {
+      c->scan_variant = (int)value;
+    } else if (k == "scan_persistent") {
+      c->scan_persistent = value ? 1 : 0;
     } else if (k == "map_unroll") {
       if (value < 1 || value > 16) fail(SKL_ERR_INVALID_ARG, "map_unroll in [1,16]");
       c->map_unroll = (int)value;

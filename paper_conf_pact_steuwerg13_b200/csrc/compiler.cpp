@@ -119,11 +119,7 @@ Program* compile(Ctx* ctx, const std::string& source, std::string* log_out) {
   return raw;
 }
 
-void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 block, size_t smem,
-            void** args) {
-  if (grid.x == 0 || grid.y == 0 || grid.z == 0) return;
-  Device& D = ctx->D(g);
-  ctx->set_device(g);
+static cudaKernel_t get_kernel(Program* prog, const char* kernel, size_t smem) {
   auto it = prog->kernels.find(kernel);
   cudaKernel_t k;
   if (it == prog->kernels.end()) {
@@ -132,13 +128,31 @@ void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 
   } else {
     k = it->second;
   }
-  if (smem > 48 * 1024) {
+  if (smem > 16 * 1024) {  // static + dynamic may exceed the 48 KB default: raise the limit
     auto s = prog->smem_set.find(kernel);
     if (s == prog->smem_set.end() || s->second < smem) {
       SKL_CUDA(cudaFuncSetAttribute((const void*)k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
       prog->smem_set[kernel] = smem;
     }
   }
+  return k;
+}
+
+// Resident blocks per SM for a kernel at a block size / dynamic smem (persistent grids).
+int occupancy(Ctx* ctx, int g, Program* prog, const char* kernel, int block, size_t smem) {
+  ctx->set_device(g);
+  cudaKernel_t k = get_kernel(prog, kernel, smem);
+  int nb = 0;
+  SKL_CUDA(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, (const void*)k, block, smem));
+  return nb;
+}
+
+void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 block, size_t smem,
+            void** args) {
+  if (grid.x == 0 || grid.y == 0 || grid.z == 0) return;
+  Device& D = ctx->D(g);
+  ctx->set_device(g);
+  cudaKernel_t k = get_kernel(prog, kernel, smem);
   SKL_CUDA(cudaLaunchKernel((const void*)k, grid, block, args, smem, D.stream));
   ctx->n_launch++;
 }

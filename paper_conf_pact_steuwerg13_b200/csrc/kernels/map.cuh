@@ -78,6 +78,11 @@ skl_map_vec(const SKL_TIN* __restrict__ in SKL_IN2_PARAM SKL_OUT_PARAM, skl_u64 
 #pragma unroll
   for (int u = 0; u < SKL_UNROLL; ++u) {
     const skl_u64 c = base + (skl_u64)u * SKL_BLOCK;
+    // Lanes running this chunk reconverge after every element: a customising
+    // function with a data-dependent loop (LM OSEM ray walks, Mandelbrot) would
+    // otherwise leave the warp split into drifting one-lane groups (independent
+    // thread scheduling does not force reconvergence between unrolled calls).
+    const unsigned act = __ballot_sync(SKL_FULL, c < nch);
     if (c < nch) {
 #if SKL_OUT_VOID
 #pragma unroll
@@ -87,6 +92,7 @@ skl_map_vec(const SKL_TIN* __restrict__ in SKL_IN2_PARAM SKL_OUT_PARAM, skl_u64 
 #else
         SKL_FUNC(a[u].e[k] SKL_XARGS);
 #endif
+        __syncwarp(act);
       }
 #else
       SklChunk<SKL_TOUT, SKL_VEC> r;
@@ -97,6 +103,7 @@ skl_map_vec(const SKL_TIN* __restrict__ in SKL_IN2_PARAM SKL_OUT_PARAM, skl_u64 
 #else
         r.e[k] = SKL_FUNC(a[u].e[k] SKL_XARGS);
 #endif
+        __syncwarp(act);
       }
       char* o = (char*)out + c * (SKL_VEC * sizeof(SKL_TOUT));
 #pragma unroll

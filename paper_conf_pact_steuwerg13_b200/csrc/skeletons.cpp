@@ -36,9 +36,9 @@ size_t vec_for(std::initializer_list<size_t> sizes) {
 bool aligned16(const void* p) { return ((uintptr_t)p & 15u) == 0; }
 size_t ceil_div(size_t a, size_t b) { return (a + b - 1) / b; }
 
-std::string defs_common(Ctx* ctx, const std::string& entry) {
+std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
   std::string s;
-  s += "#define SKL_BLOCK " + std::to_string(ctx->block_threads) + "\n";
+  s += "#define SKL_BLOCK " + std::to_string(block) + "\n";
   s += "#define SKL_DEBUG_BOUNDS " + std::to_string(ctx->debug_bounds ? 1 : 0) + "\n";
   s += "#define SKL_FUNC " + entry + "\n";
   return s;
@@ -80,7 +80,10 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
   s->boundary = boundary;
   const std::string user = "\n// ---- customising function (user source)\n#line 1 \"user_source\"\n" +
                            s->user_src + "\n#line 1 \"skeleton_template\"\n";
-  std::string defs = defs_common(ctx, s->entry);
+  // launch geometry is fixed at creation (compiled into the program)
+  s->block = ctx->block_threads;
+  s->unroll = ctx->map_unroll;
+  std::string defs = defs_common(ctx, s->entry, s->block);
   std::string body;
   switch (kind) {
     case K_MAP:
@@ -119,9 +122,19 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       defs += "#define SKL_RVEC " + std::to_string(rvec) + "\n#define SKL_RU 4\n";
       if (kind == K_SCAN) {
         // 8 chunks (128 B) per thread: 8192 fp32 elements per tile (SURVEY §7 hard part 2)
-        const int ch = (16 % st == 0) ? 8 : 0;
+        const int ch = (16 % st == 0) ? ctx->scan_chunks : 0;
+        s->scan_ch = ch;
         const int items = ch ? (int)(ch * 16 / st) : 8;
         defs += "#define SKL_CH " + std::to_string(ch) + "\n#define SKL_ITEMS " + std::to_string(items) + "\n";
+        defs += std::string("#define SKL_PACKED ") + (st <= 4 ? "1" : "0") + "\n";
+        defs += "#define SKL_SCAN_VARIANT " + std::to_string(ctx->scan_variant) + "\n";
+        s->scan_sub = ctx->scan_sub;
+        s->scan_variant = ctx->scan_variant;
+        s->scan_fstride = ctx->scan_fstride;
+        defs += "#define SKL_FSTRIDE " + std::to_string(s->scan_fstride) + "\n";
+        defs += "#define SKL_SPIN_NS " + std::to_string(ctx->scan_spin_ns) + "\n";
+        defs += "#define SKL_MINB " + std::to_string(ctx->scan_minb) + "\n";
+        defs += "#define SKL_SUB " + std::to_string(s->scan_sub) + "\n";
       }
       body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +
              kernel_template("reduce.cuh") + (kind == K_SCAN ? kernel_template("scan.cuh") : "");
@@ -282,7 +295,7 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
   const size_t vec = std::min<size_t>(
       vec_for({ctx->type(s->tin).size, in2 ? ctx->type(s->tin2).size : 0,
                s->tout == SKL_VOID ? 0 : ctx->type(s->tout).size}), 64);
-  const size_t per_block = (size_t)ctx->block_threads * (size_t)ctx->map_unroll;
+  const size_t per_block = (size_t)s->block * (size_t)s->unroll;
   int ndev = 0;
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
     const Range r = core_range(in->units(), ctx->G, din, g);
@@ -316,7 +329,7 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
       grid = ceil_div(n, per_block);
       kname = "skl_map_sc";
     }
-    launch(ctx, g, s->prog, kname, dim3((unsigned)grid), dim3(ctx->block_threads), 0, args.data());
+    launch(ctx, g, s->prog, kname, dim3((unsigned)grid), dim3(s->block), 0, args.data());
   }
   if (o) mark_written(o);
   finish_extras(ctx, ea, ndev);
@@ -337,11 +350,11 @@ void run_zip(Skel* s, Cont* l, Cont* r, Cont** out, const skl_arg* extra, int ne
 static void reduce_on_device(Skel* s, int g, const void* in, size_t n, void* result) {
   Ctx* ctx = s->ctx;
   const size_t st = ctx->type(s->tin).size;
-  const int nw = ctx->block_threads / 32;
+  const int nw = s->block / 32;
   const bool vec = (16 % st == 0) && aligned16(in);
   const size_t rtile = 32 * (vec ? 16 / st : 1);
   const size_t ru = 4;
-  const size_t max_blocks = (size_t)ctx->D(g).sm_count * (2048 / (size_t)ctx->block_threads);
+  const size_t max_blocks = (size_t)ctx->D(g).sm_count * (2048 / (size_t)s->block);
   size_t nblocks = std::min(max_blocks, std::max<size_t>(1, ceil_div(n, (size_t)nw * rtile * ru)));
   size_t wseg = ceil_div(ceil_div(n, nblocks * (size_t)nw), rtile) * rtile;
   nblocks = ceil_div(n, (size_t)nw * wseg);
@@ -352,7 +365,7 @@ static void reduce_on_device(Skel* s, int g, const void* in, size_t n, void* res
   unsigned long long nn = n, ws = wseg;
   void* args[] = {(void*)&in, &nn, &ws, &partials, &counter, &result};
   launch(ctx, g, s->prog, vec ? "skl_reduce_vec" : "skl_reduce_sc", dim3((unsigned)nblocks),
-         dim3(ctx->block_threads), 0, args);
+         dim3(s->block), 0, args);
 }
 
 void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
@@ -360,10 +373,10 @@ void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int n
   if (!s || (s->kind != K_REDUCE && s->kind != K_SCAN)) fail(SKL_ERR_INVALID_ARG, "combine needs a Reduce skeleton");
   Ctx* ctx = s->ctx;
   unsigned long long stride = stride_elems, n = nelem;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(nelem, (size_t)ctx->block_threads),
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(nelem, (size_t)s->block),
                                                            (size_t)ctx->D(g).sm_count * 8));
   void* args[] = {(void*)&staging, &stride, &nrep, &dst, &n};
-  launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(ctx->block_threads), 0, args);
+  launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(s->block), 0, args);
 }
 
 void run_reduce(Skel* s, Cont* in, Cont** out) {
@@ -448,9 +461,8 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
   if (o == in) fail(SKL_ERR_INVALID_ARG, "scan cannot run in place");
   prepare_output(o, din, 0);
   const size_t st = in->elt;
-  const bool chunked = (16 % st == 0);
-  const int items = chunked ? (int)(8 * 16 / st) : 8;
-  const size_t tile = (size_t)ctx->block_threads * (size_t)items;
+  const bool chunked = s->scan_ch > 0;
+  const int items = chunked ? (int)((size_t)s->scan_ch * 16 / st) : 8;
   // participants with distinct data (block / single); copy scans whole on each device
   std::vector<int> parts;
   for (int g = 0; g < ctx->G; ++g)
@@ -487,9 +499,19 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
     if (!ctx->is_local(g)) continue;
     const Range r = core_range(in->units(), ctx->G, din, g);
     const size_t n = r.size() * in->cols;
-    const size_t ntiles = ceil_div(n, tile);
-    // status: [flags u32 x ntiles] [aggs T x ntiles] [incls T x ntiles], 16-B aligned
-    const size_t fbytes = ceil_div(ntiles * 4, 16) * 16, tbytes = ceil_div(ntiles * st, 16) * 16;
+    const void* pin = part_ptr(in, g, r.lo);
+    void* pout = part_ptr(o, g, r.lo);
+    const bool vec = chunked && aligned16(pin) && aligned16(pout);
+    // look-back unit: a chunk of scan_sub tiles (vector kernel) or one tile of 8 items
+    // per thread (generic kernel)
+    const size_t tile = (size_t)s->block * (size_t)(vec ? items : 8);
+    const bool per_tile = s->scan_variant >= 2;  // one block per tile, tile look-back
+    const size_t ntiles = ceil_div(n, vec && !per_tile ? tile * (size_t)s->scan_sub : tile);
+    // status: [flags u32 x units] [aggs T x units] [incls T x units], 16-B aligned
+    // packed status (elements <= 4 bytes): one u64 per tile holds value and flag
+    // (status words are s->scan_fstride x 8 bytes apart: one L2 line per unit by default)
+    const size_t fbytes = ceil_div(ntiles * 8 * (size_t)s->scan_fstride, 16) * 16,
+                 tbytes = ceil_div(ntiles * st, 16) * 16;
     Scratch& sc = s->scratch_scan[g];
     const bool fresh = sc.bytes < fbytes + 2 * tbytes;
     char* base = (char*)scratch(s, s->scratch_scan, g, fbytes + 2 * tbytes, true);
@@ -503,15 +525,22 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
     void* flags = base;
     void* aggs = base + fbytes;
     void* incls = base + fbytes + tbytes;
-    const void* pin = part_ptr(in, g, r.lo);
-    void* pout = part_ptr(o, g, r.lo);
     unsigned long long nn = n;
     const void* cptr = carry ? totals[g] : nullptr;
     int ncarry = carry ? i : 0;
     void* args[] = {(void*)&pin, &pout, &nn, &flags, &aggs, &incls, &ep, (void*)&cptr, &ncarry};
-    const bool vec = chunked && aligned16(pin) && aligned16(pout);
-    launch(ctx, g, s->prog, vec ? "skl_scan_vec" : "skl_scan_sc", dim3((unsigned)ntiles),
-           dim3(ctx->block_threads), 0, args);
+    if (vec && per_tile) {
+      const size_t smem = (size_t)s->block * (size_t)s->scan_ch * 16;
+      launch(ctx, g, s->prog, "skl_scan_pt", dim3((unsigned)ntiles), dim3(s->block), smem, args);
+    } else if (vec) {
+      // persistent grid (one wave of resident blocks), two shared-memory stages
+      const size_t smem = 2 * (size_t)s->block * (size_t)s->scan_ch * 16;
+      const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_scan_vec", s->block, smem));
+      const size_t grid = std::min(ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
+      launch(ctx, g, s->prog, "skl_scan_vec", dim3((unsigned)grid), dim3(s->block), smem, args);
+    } else {
+      launch(ctx, g, s->prog, "skl_scan_sc", dim3((unsigned)ntiles), dim3(s->block), 0, args);
+    }
   }
   mark_written(o);
 }
@@ -549,15 +578,15 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                       s->neutral.data(), &vec_ok};
       const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
                       (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
-      launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(ctx->block_threads), 0, args);
+      launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(s->block), 0, args);
     }
   } else {
     // vector form: compile the 1-D variant once
     if (!s->prog1d) {
       const size_t epc = 16 / si;
       const int A = (int)(ceil_div((size_t)d, epc) * epc);
-      const int cw = 4, tw = ctx->block_threads * cw;
-      std::string defs = defs_common(ctx, s->entry);
+      const int cw = 4, tw = s->block * cw;
+      std::string defs = defs_common(ctx, s->entry, s->block);
       defs += "#define SKL_TIN " + tname(ctx, s->tin) + "\n#define SKL_TOUT " + tname(ctx, s->tout) + "\n";
       defs += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(s->boundary) + "\n";
       defs += "#define SKL_A " + std::to_string(A) + "\n#define SKL_PITCH 0\n";
@@ -570,7 +599,7 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                                 nullptr);
       s->mo_1d = true;
     }
-    const int tw = ctx->block_threads * 4;
+    const int tw = s->block * 4;
     for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
       const Range r = core_range(in->units(), ctx->G, dout, g);
       if (r.empty()) continue;
@@ -584,7 +613,7 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       void* args[] = {(void*)&pin, &in_lo, &in_n, &pout, &out_lo, &N, &unused, &rb, &re,
                       s->neutral.data(), &vec_ok};
       launch(ctx, g, s->prog1d, "skl_mo1d", dim3((unsigned)ceil_div(r.size(), (size_t)tw)),
-             dim3(ctx->block_threads), 0, args);
+             dim3(s->block), 0, args);
     }
   }
   mark_written(o);

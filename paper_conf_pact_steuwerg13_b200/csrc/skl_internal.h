@@ -108,6 +108,16 @@ struct Ctx {
   int block_threads = 256;
   int debug_bounds = 0;
   int map_unroll = 4;
+  int scan_chunks = 8;         // 16-byte chunks per thread in a Scan tile
+  int scan_persistent = 1;     // (unused since the chunked Scan; kept for the option API)
+  int scan_sub = 4;            // Scan tiles per look-back chunk
+  int scan_fstride = 16;       // Scan status word spacing (8-byte units; 16 = one L2 line)
+  int scan_spin_ns = 0;        // Scan look-back spin back-off (__nanosleep)
+  int scan_minb = 4;           // Scan per-tile kernel: min resident blocks (launch bounds)
+  // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest
+  // measured); 2 = one block per tile, warp-wide look-back; 0 = persistent
+  // chunked (L2 re-read); 1 = measurement only: no look-back (wrong results)
+  int scan_variant = 3;
   // counters
   std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0};
   // NVRTC cache: source hash -> program
@@ -186,6 +196,7 @@ Program* compile(Ctx* ctx, const std::string& source, std::string* log_out);
 void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 block,
             size_t smem, void** args);
 int max_smem_optin(Ctx* ctx, int g);
+int occupancy(Ctx* ctx, int g, Program* prog, const char* kernel, int block, size_t smem);
 std::string detect_entry(const std::string& src);
 std::string kernel_template(const char* name);  // embedded kernels/*.cuh
 
@@ -212,6 +223,12 @@ struct Skel {
   // MapOverlap tile geometry (compile-time constants of prog)
   int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0;
   bool mo_1d = false;
+  int scan_ch = 0;   // Scan: 16-byte chunks per thread (0 = generic path)
+  int scan_sub = 4;  // Scan: tiles per look-back chunk (vector path)
+  int scan_variant = 0;
+  int scan_fstride = 16;  // Scan: status word spacing in 8-byte units
+  int block = 256;   // threads per block the program was compiled for
+  int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
 };
 Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int tin, int tin2,
                   int tout, const int* extra, int nextra, int d, int boundary, const void* neutral);

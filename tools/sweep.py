@@ -1,0 +1,147 @@
+"""Parameter sweeps on one GPU (work-group size / unroll knobs, user-function
+variants).  Prints one line per configuration: device ms per call (CUDA events,
+L2 flushed), plus a parity flag against the oracle where cheap.
+
+  python tools/sweep.py mandel|lmosem|scan|mo
+"""
+import os
+import sys
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import torch  # noqa: E402
+
+import oracle as O  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import apps as A  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import inputs as I  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
+
+FLUSH = None
+
+
+def ctx_with(opts):
+    global FLUSH
+    c = S.Context(1)
+    s = torch.cuda.Stream()
+    torch.cuda.set_stream(s)
+    c.set_stream(0, s.cuda_stream)
+    for k, v in opts.items():
+        c.set_option(k, v)
+    if FLUSH is None:
+        FLUSH = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
+    return c
+
+
+def timeit(fn, reps=10, warm=3):
+    for _ in range(warm):
+        fn()
+    ts = []
+    for _ in range(reps):
+        FLUSH.zero_()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record()
+        fn()
+        b.record()
+        ts.append((a, b))
+    torch.cuda.synchronize()
+    return float(np.median([a.elapsed_time(b) for a, b in ts]))
+
+
+def mandel():
+    grid = I.mandel_grid(3072, 4096)
+    ref = None
+    for name, src in (("plain", A.mandelbrot(1000)), ("unroll4", A.mandelbrot_unrolled(1000))):
+        for bt in (128, 256, 512):
+            for un in (1, 2, 4):
+                c = ctx_with({"block_threads": bt, "map_unroll": un})
+                m = S.Map(c, src, S.F32X2, S.U32)
+                x = S.Matrix(c, S.F32X2, 3072, 4096).copy_in(grid)
+                o = m(x)
+                ms = timeit(lambda: m(x, out=o))
+                out = o.to_numpy()
+                if ref is None:
+                    ref, tot = O.mandelbrot(grid, 1000)
+                ok = np.array_equal(out, ref)
+                print(f"mandel {name:8s} block={bt:4d} unroll={un}: {ms:.4f} ms  "
+                      f"{8 * tot / (ms / 1e3) / 1e12:.2f} TFLOP/s  bitexact={ok}", flush=True)
+                c.finalize()
+
+
+def lmosem():
+    N, nev = 150, 10_000_000
+    events = I.lmosem_events(7, nev, N)
+    for bt in (128, 256):
+        for un in (1, 4):
+            c = ctx_with({"block_threads": bt, "map_unroll": un})
+            evd = c.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
+            lm = S.Map(c, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
+            ev = S.Vector(c, evd, nev).set_distribution(S.BLOCK)
+            ev.copy_in(events)
+            f = S.Vector(c, S.F32, N ** 3).set_distribution(S.COPY).fill(1.0)
+            cc = S.Vector(c, S.F32, N ** 3).set_distribution(S.COPY).fill(0.0)
+            ms = timeit(lambda: lm(ev, f, (cc, S.WRITE)), reps=5, warm=1)
+            print(f"lmosem block={bt} unroll={un}: {ms:.3f} ms  {nev / (ms / 1e3) / 1e9:.3f} Gevents/s", flush=True)
+            c.finalize()
+
+
+def scan():
+    n = 1 << 30
+    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 3), (3, 1, 256, 8, 16, 4), (3, 1, 256, 8, 8, 3),
+                                      (3, 1, 256, 8, 16, 2), (3, 1, 384, 8, 16, 2), (3, 1, 192, 8, 16, 4),
+                                      (3, 1, 256, 6, 16, 4) if False else (3, 1, 128, 8, 16, 8),
+                                      (2, 1, 256, 8, 16, 3), (1, 1, 256, 8, 16, 3)):
+        if True:
+            if True:
+                c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_sub": pers,
+                              "scan_variant": var, "scan_fstride": fs, "scan_minb": ns})
+                sc = S.Scan(c, A.ADD_I32, S.I32)
+                v = S.Vector(c, S.I32, n).set_distribution(S.BLOCK).fill(1)
+                o = sc(v)
+                ms = timeit(lambda: sc(v, out=o), reps=5)
+                p, f, cnt = o.local_part(0)
+                print(f"scan i32 variant={var} sub={pers} block={bt} chunks={ch} fstride={fs} spin={ns}: {ms:.3f} ms  "
+                      f"{8 * n / (ms / 1e3) / 1e9:.0f} GB/s", flush=True)
+                c.finalize()
+
+
+def copy():
+    """Map identity over 2^30 int32 (read 4 B + write 4 B per element): the
+    skeleton's streaming ceiling, for comparison with Scan and the measured copy."""
+    n = 1 << 30
+    for bt in (256, 512):
+        for un in (1, 2, 4, 8):
+            c = ctx_with({"block_threads": bt, "map_unroll": un})
+            m = S.Map(c, "int id(int x){ return x; }", S.I32, S.I32)
+            v = S.Vector(c, S.I32, n).set_distribution(S.BLOCK).fill(1)
+            o = m(v)
+            ms = timeit(lambda: m(v, out=o), reps=5)
+            print(f"map-copy i32 block={bt} unroll={un}: {ms:.3f} ms  {8 * n / (ms / 1e3) / 1e9:.0f} GB/s", flush=True)
+            c.finalize()
+
+
+def mo():
+    img8 = I.image_u8(5, 8192, 8192)
+    imgf = I.image_f32(6, 8192, 8192)
+    for bt in (128, 256, 512):
+        c = ctx_with({"block_threads": bt})
+        for name, src, t, d, bnd, img in (("ident_u8", A.IDENT2D_U8, S.U8, 1, S.NEUTRAL, img8),
+                                          ("sobel", A.SOBEL, S.U8, 1, S.NEUTRAL, img8),
+                                          ("ident_f32", A.IDENT2D, S.F32, 2, S.NEAREST, imgf),
+                                          ("gauss", A.gaussian5(), S.F32, 2, S.NEAREST, imgf)):
+            m = S.MapOverlap(c, src, t, t, d, bnd, 0)
+            x = S.Matrix.from_numpy(c, img)
+            o = m(x)
+            ms = timeit(lambda: m(x, out=o))
+            bpp = 2 * img.itemsize
+            print(f"mo {name:9s} block={bt}: {ms:.4f} ms  {bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s", flush=True)
+            x.destroy()
+            o.destroy()
+        c.finalize()
+
+
+if __name__ == "__main__":
+    for w in sys.argv[1:]:
+        globals()[w]()
