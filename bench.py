@@ -209,7 +209,14 @@ def bench_mandelbrot(args, D: Dist, P: dict):
     from paper_conf_pact_steuwerg13_b200 import inputs as I
     from paper_conf_pact_steuwerg13_b200 import skl as S
     ctx, g = make_context(D)
-    m = S.Map(ctx, A.mandelbrot(MAX_ITER), S.F32X2, S.U32)
+    # user-side tuning (the paper's optional work-group size):
+    # 512-thread blocks, 2 chunks per thread; the customising function checks the
+    # escape once per 4 iterations and replays the block (bit-identical counts)
+    ctx.set_option("block_threads", 512)
+    ctx.set_option("map_unroll", 2)
+    m = S.Map(ctx, A.mandelbrot_unrolled(MAX_ITER), S.F32X2, S.U32)
+    ctx.set_option("block_threads", 256)
+    ctx.set_option("map_unroll", 4)
     grid = I.mandel_grid(ROWS, COLS)
     cin = S.Matrix(ctx, S.F32X2, ROWS, COLS).set_distribution(S.BLOCK)
     cin.copy_in(grid)
@@ -422,7 +429,9 @@ def bench_skeletons(args, D: Dist, P: dict, which):
     if "lmosem" in which:
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
+        ctx.set_option("map_unroll", 1)   # divergent per-event work: one chunk per thread
         lm = S.Map(ctx, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
+        ctx.set_option("map_unroll", 4)
         upd = S.Zip(ctx, A.LMOSEM_UPDATE, S.F32, S.F32, S.F32)
         addf = S.Reduce(ctx, A.ADD, S.F32)
         events = I.lmosem_events(I.SEED_LMOSEM, nev, N)
