@@ -271,11 +271,23 @@ def mandel_oracle(sample_every: int = 1):
 
 
 # ---------------------------------------------------------------- per-skeleton lines
-def roof_hbm(bytes_per_step: float, ms: float, P: dict):
+def ncu_traffic(workload: str):
+    """DRAM bytes per launch (dram__bytes_read.sum + dram__bytes_write.sum) of the
+    workload's dominant kernel from the committed ncu --set full summary
+    (profiles/ncu_traffic.json, written by tools/ncu_traffic.py), else None."""
+    f = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    try:
+        return float(json.load(open(f))[workload]["bytes_per_launch"])
+    except Exception:
+        return None
+
+
+def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None):
     gbs = bytes_per_step / (ms / 1e3) / 1e9
     return {"bound": "hbm", "achieved": round(gbs, 1), "peak": P["hbm_gbs"], "unit": "GB/s",
             "frac": round(gbs / P["hbm_gbs"], 4), "frac_of_nominal_8TBs": round(gbs / 8000.0, 4),
-            "peak_source": P["source"]}
+            "peak_source": P["source"], "traffic": ncu_traffic(workload) if workload else None,
+            "algorithmic_bytes": bytes_per_step}
 
 
 def bench_skeletons(args, D: Dist, P: dict, which):
@@ -313,7 +325,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                         "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3),
                         "GB_per_s_unfused_16B": 16 * n / (ms / 1e3) / 1e9,
                         "zip_ms": round(seg[0], 4), "reduce_ms": round(seg[1], 4),
-                        "roofline_zip": roof_hbm(12 * n, seg[0], P), "roofline_reduce": roof_hbm(4 * n, seg[1], P),
+                        "roofline_zip": roof_hbm(12 * n, seg[0], P, "dot_2^28_zip" if n == 1 << 28 else None), "roofline_reduce": roof_hbm(4 * n, seg[1], P),
                         "rel_err": abs(got - ref) / abs(ref), "check": "ok" if abs(got - ref) <= 1e-5 * abs(ref) else "FAIL"}
             for x in (va, vb, c):
                 x.destroy()
@@ -349,7 +361,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             res[name] = {"workload": f"{'Sobel u8 d=1 NEUTRAL' if name == 'sobel' else 'Gaussian 5x5 f32 d=2 NEAREST'} "
                                      f"MapOverlap {R}x{C}, overlap distribution",
                          "ms": round(ms, 4), "elements_per_s": R * C / (ms / 1e3),
-                         "roofline": roof_hbm(bpp * R * C, ms, P), "check": "ok" if ok else "FAIL"}
+                         "roofline": roof_hbm(bpp * R * C, ms, P, name), "check": "ok" if ok else "FAIL"}
             mi.destroy()
             o.destroy()
 
@@ -418,7 +430,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                 errs.append(abs(last - tot) / abs(tot))
                 ok &= errs[-1] <= 1e-5
         res[name] = {"workload": f"inclusive Scan (+) over 2^30 {'int32' if dt == S.I32 else 'fp32'}, block + carry-in",
-                     "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3), "roofline": roof_hbm(8 * n, ms, P),
+                     "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3), "roofline": roof_hbm(8 * n, ms, P, name if name == "scan_i32" else None),
                      "check": "ok" if ok else "FAIL", "max_rel_err": max(errs) if errs else 0.0,
                      "data": "torch-seeded on device (int32 U{-1000..1000} / fp32 U[0,1))"}
         del src, got_t
@@ -553,7 +565,7 @@ def main():
                    "l2": "flushed between steps (256 MiB write)", "parallelism": f"block rows over {args.gpus} GPU(s)",
                    "imbalance_limited_ideal_speedup": float(sum(per) / max(per)) if max(per) > 0 else 1.0},
         "roofline": {"bound": "alu", "achieved": achieved / 1e12, "peak": alu_peak / 1e12, "unit": "TFLOP/s",
-                     "frac": achieved / alu_peak, "traffic": None,
+                     "frac": achieved / alu_peak, "traffic": ncu_traffic("mandelbrot"),
                      "note": f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count); peak = {sms} SMs x 128 "
                              f"FP32 lanes x {P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false)"},
         "cpu_baseline": {"value": ROWS * COLS / cpu_s, "unit": "elements/s", "cores": 1, "kind": "oracle",

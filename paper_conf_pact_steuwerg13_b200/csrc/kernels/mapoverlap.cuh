@@ -63,7 +63,11 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
       continue;
     }
     if (vec_ok && (SKL_BOUNDARY == 1 || row_in) && gc0 >= 0 && gc0 + SKL_EPC <= C) {
-      *(uint4*)dst = skl_ld16(in + (gr - in_row0) * C + gc0);
+      // interior: asynchronous 16-byte global->shared copy (LDGSTS), no register
+      // round trip, all of a thread's chunks in flight at once
+      const unsigned sa = (unsigned)__cvta_generic_to_shared(dst);
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa),
+                   "l"(in + (gr - in_row0) * C + gc0) : "memory");
     } else {
 #pragma unroll
       for (int e = 0; e < SKL_EPC; ++e) {
@@ -80,6 +84,7 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
       }
     }
   }
+  asm volatile("cp.async.wait_all;" ::: "memory");
   __syncthreads();
   // ---- apply f to a SKL_RH x SKL_CW block per thread
   const int ty = threadIdx.x / (SKL_TW / SKL_CW), tx = threadIdx.x % (SKL_TW / SKL_CW);
@@ -123,7 +128,8 @@ skl_mo1d(const SKL_TIN* __restrict__ in, long in_lo, long in_n, SKL_TOUT* __rest
     SKL_TIN* dst = tile + q * SKL_EPC;
     if (vec_ok && g0 >= in_lo && g0 + SKL_EPC <= in_lo + in_n && g0 >= 0 && g0 + SKL_EPC <= N &&
         ((g0 - in_lo) % SKL_EPC) == 0) {
-      *(uint4*)dst = skl_ld16(in + (g0 - in_lo));
+      const unsigned sa = (unsigned)__cvta_generic_to_shared(dst);
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(in + (g0 - in_lo)) : "memory");
     } else {
 #pragma unroll
       for (int e = 0; e < SKL_EPC; ++e) {
@@ -141,6 +147,7 @@ skl_mo1d(const SKL_TIN* __restrict__ in, long in_lo, long in_n, SKL_TOUT* __rest
       }
     }
   }
+  asm volatile("cp.async.wait_all;" ::: "memory");
   __syncthreads();
   const long i0 = e0 + (long)threadIdx.x * SKL_CW;
   const SKL_TIN* p = tile + SKL_A + threadIdx.x * SKL_CW;

@@ -151,9 +151,15 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       const int epc = (int)(16 / si);
       const int A = (int)ceil_div((size_t)d, (size_t)epc) * epc;
       int cw, rh, tw, th;
-      if (si == 1 || si == 2) { cw = 4; rh = 8; }
-      else if (si == 4) { cw = 2; rh = 8; }
-      else { cw = 1; rh = 4; }
+      // default register block: one 16-byte-wide run of outputs per row, 2 rows
+      // (swept on B200, tools/sweep.py mo: Gaussian f32 0.224 -> 0.182 ms,
+      // Sobel u8 0.092 -> 0.088 ms at 256 threads)
+      cw = (int)(16 / std::min<size_t>(so, 16) > 0 ? 16 / std::min<size_t>(so, 16) : 1);
+      rh = 2;
+      if (ctx->mo_cw > 0) cw = ctx->mo_cw;  // register block per thread (tuning knobs)
+      if (ctx->mo_rh > 0) rh = ctx->mo_rh;
+      if ((cw * (int)si) % 16 != 0 && (16 % (cw * (int)si)) != 0)
+        fail(SKL_ERR_INVALID_ARG, "mo_cw x element size must divide or be a multiple of 16 bytes");
       const int nthr = ctx->block_threads;
       tw = 32 * cw;
       const int rows_thr = nthr / 32;

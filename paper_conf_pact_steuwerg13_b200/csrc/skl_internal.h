@@ -114,6 +114,7 @@ struct Ctx {
   int scan_fstride = 16;       // Scan status word spacing (8-byte units; 16 = one L2 line)
   int scan_spin_ns = 0;        // Scan look-back spin back-off (__nanosleep)
   int scan_minb = 4;           // Scan per-tile kernel: min resident blocks (launch bounds)
+  int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest
   // measured); 2 = one block per tile, warp-wide look-back; 0 = persistent
   // chunked (L2 re-read); 1 = measurement only: no look-back (wrong results)

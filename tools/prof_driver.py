@@ -20,7 +20,10 @@ from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
 def main(which: str, reps: int = 3):
     ctx = S.Context(1)
     if which == "mandel":
-        m = S.Map(ctx, A.mandelbrot(1000), S.F32X2, S.U32)
+        # the bench's configuration
+        ctx.set_option("block_threads", 512)
+        ctx.set_option("map_unroll", 2)
+        m = S.Map(ctx, A.mandelbrot_unrolled(1000), S.F32X2, S.U32)
         x = S.Matrix(ctx, S.F32X2, 3072, 4096).copy_in(I.mandel_grid(3072, 4096))
         o = m(x)
         for _ in range(reps):
@@ -57,6 +60,7 @@ def main(which: str, reps: int = 3):
     elif which == "lmosem":
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
+        ctx.set_option("map_unroll", 1)
         lm = S.Map(ctx, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
         ev = S.Vector(ctx, evd, nev).set_distribution(S.BLOCK)
         ev.copy_in(I.lmosem_events(7, nev, N))

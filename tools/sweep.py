@@ -125,18 +125,28 @@ def copy():
 def mo():
     img8 = I.image_u8(5, 8192, 8192)
     imgf = I.image_f32(6, 8192, 8192)
-    for bt in (128, 256, 512):
+    for bt, rh, cw8, cw32 in ((128, 8, 4, 2), (128, 4, 4, 2), (128, 2, 4, 2), (128, 4, 8, 4), (128, 8, 16, 1),
+                              (256, 4, 8, 1), (256, 2, 16, 4), (64, 8, 4, 2), (128, 16, 4, 1)):
         c = ctx_with({"block_threads": bt})
         for name, src, t, d, bnd, img in (("ident_u8", A.IDENT2D_U8, S.U8, 1, S.NEUTRAL, img8),
                                           ("sobel", A.SOBEL, S.U8, 1, S.NEUTRAL, img8),
                                           ("ident_f32", A.IDENT2D, S.F32, 2, S.NEAREST, imgf),
                                           ("gauss", A.gaussian5(), S.F32, 2, S.NEAREST, imgf)):
+            c.set_option("mo_rh", rh)
+            c.set_option("mo_cw", cw8 if t == S.U8 else cw32)
             m = S.MapOverlap(c, src, t, t, d, bnd, 0)
             x = S.Matrix.from_numpy(c, img)
             o = m(x)
             ms = timeit(lambda: m(x, out=o))
             bpp = 2 * img.itemsize
-            print(f"mo {name:9s} block={bt}: {ms:.4f} ms  {bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s", flush=True)
+            ok = ""
+            if name in ("sobel", "gauss"):
+                sub = img[3990:4074]
+                ref = (O.mapoverlap2d(O.OS_SOBEL, sub, 1, O.OB_NEUTRAL, 0) if name == "sobel"
+                       else O.mapoverlap2d(O.OS_GAUSS5, sub, 2, O.OB_NEAREST, 0.0))[10:74]
+                ok = f" bitexact={np.array_equal(o.to_numpy()[4000:4064], ref)}"
+            print(f"mo {name:9s} block={bt} rh={rh} cw={cw8 if t == S.U8 else cw32}: {ms:.4f} ms  "
+                  f"{bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s{ok}", flush=True)
             x.destroy()
             o.destroy()
         c.finalize()
