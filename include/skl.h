@@ -234,6 +234,21 @@ skl_status skl_mapoverlap_run(skl_skel* sk, skl_cont* in, skl_cont** out);
 /* Scalar<T>::getValue(): download the 1-element result.           */
 skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes);
 
+/* ------------------------------------------------------------------ CUDA graphs
+ * Record a sequence of skeleton calls once and replay it with one launch (for
+ * latency-bound steps; the paper's runtime has no equivalent).  Between
+ * skl_capture_begin and skl_capture_end the calls are recorded on the device
+ * stream instead of executed; calls that hand data to the host (copy_out,
+ * scalar_get, host_data, sync) are not allowed inside.  Containers and
+ * skeletons used by a graph must outlive it, keep their sizes and
+ * distributions, and have been used once before capture (so that nothing is
+ * allocated or compiled while capturing).  One local device only.            */
+typedef struct skl_graph skl_graph;
+skl_status skl_capture_begin(skl_ctx* ctx);
+skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out);
+skl_status skl_graph_launch(skl_graph* g);
+skl_status skl_graph_destroy(skl_graph* g);
+
 /* ------------------------------------------------------------------ offline compilation
  * skl_init_offline: a context without devices (no GPU needed) in which
  * skeleton creation runs the full NVRTC compilation for sm_100a but loads

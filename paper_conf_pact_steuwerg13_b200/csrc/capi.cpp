@@ -147,6 +147,7 @@ skl_status skl_get_stream(skl_ctx* ctx, int g, void** stream) {
 skl_status skl_sync(skl_ctx* ctx) {
   return guard([&] {
     Ctx* c = C(ctx);
+    if (c->capturing) fail(SKL_ERR_INVALID_ARG, "skl_sync while capturing a graph");
     for (auto& d : c->dev) {
       SKL_CUDA(cudaSetDevice(d.phys));
       SKL_CUDA(cudaStreamSynchronize(d.stream));
@@ -271,6 +272,8 @@ skl_status skl_copy_in(skl_cont* c, const void* host, size_t bytes) {
   return guard([&] {
     Cont* k = K(c);
     if (!host || bytes != k->bytes()) fail(SKL_ERR_SIZE_MISMATCH, "copy_in: byte count must equal the container size");
+    materialize_dependents(k);  // deferred readers of the old value run first
+    drop_lazy(k);
     if (k->dist.kind == DNONE) {
       void* m = host_mirror(k, SKL_WRITE);
       std::memcpy(m, host, bytes);
@@ -338,6 +341,7 @@ skl_status skl_set_distribution(skl_cont* c, int kind, int arg, skl_skel* combin
       if (s->kind != K_REDUCE || ctx->type(s->tin).size != k->elt)
         fail(SKL_ERR_TYPE, "combine must be a Reduce skeleton over the container's element type");
     }
+    materialize(k);  // a deferred Zip/Map result exists before it is moved
     if (!k->dev_valid) {
       k->dist = d;  // data moves lazily (upload at first use)
     } else {
@@ -361,6 +365,7 @@ skl_status skl_local_part(skl_cont* c, int g, void** dptr, size_t* first_unit, s
     if (first_unit) *first_unit = 0;
     if (nunits) *nunits = 0;
     if (g < 0 || g >= k->ctx->G || !k->ctx->is_local(g)) return;
+    materialize(k);
     // a distribution set on host data becomes resident here (implicit upload)
     if (k->dist.kind != DNONE && !k->dev_valid && k->host_valid) ensure(k, k->dist, k->dist.kind == DOVERLAP);
     Part& p = k->parts[(size_t)g];
@@ -456,6 +461,57 @@ skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes) {
     Cont* k = K(scalar);
     if (!value || bytes != k->bytes()) fail(SKL_ERR_SIZE_MISMATCH, "scalar_get: byte count must equal the element size");
     host_download(k, value);
+  });
+}
+
+// ---- CUDA graphs
+struct skl_graph {
+  Ctx* ctx;
+  int g;
+  cudaGraph_t graph;
+  cudaGraphExec_t exec;
+};
+skl_status skl_capture_begin(skl_ctx* ctx) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (c->nlocal != 1) fail(SKL_ERR_UNSUPPORTED, "graph capture needs exactly one local device");
+    if (c->capturing) fail(SKL_ERR_INVALID_ARG, "already capturing");
+    c->set_device(c->first_local);
+    SKL_CUDA(cudaStreamBeginCapture(c->D(c->first_local).stream, cudaStreamCaptureModeRelaxed));
+    c->capturing = true;
+  });
+}
+skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if (!c->capturing || !out) fail(SKL_ERR_INVALID_ARG, "not capturing / NULL out");
+    c->capturing = false;
+    c->set_device(c->first_local);
+    cudaGraph_t graph = nullptr;
+    SKL_CUDA(cudaStreamEndCapture(c->D(c->first_local).stream, &graph));
+    cudaGraphExec_t exec = nullptr;
+    cudaError_t e = cudaGraphInstantiate(&exec, graph, 0);
+    if (e != cudaSuccess) {
+      cudaGraphDestroy(graph);
+      cuda_check(e, "cudaGraphInstantiate");
+    }
+    *out = new skl_graph{c, c->first_local, graph, exec};
+  });
+}
+skl_status skl_graph_launch(skl_graph* gr) {
+  return guard([&] {
+    if (!gr) fail(SKL_ERR_INVALID_ARG, "NULL graph");
+    gr->ctx->set_device(gr->g);
+    SKL_CUDA(cudaGraphLaunch(gr->exec, gr->ctx->D(gr->g).stream));
+    gr->ctx->n_launch += 1;
+  });
+}
+skl_status skl_graph_destroy(skl_graph* gr) {
+  return guard([&] {
+    if (!gr) return;
+    cudaGraphExecDestroy(gr->exec);
+    cudaGraphDestroy(gr->graph);
+    delete gr;
   });
 }
 

@@ -140,10 +140,14 @@ static cudaKernel_t get_kernel(Program* prog, const char* kernel, size_t smem) {
 
 // Resident blocks per SM for a kernel at a block size / dynamic smem (persistent grids).
 int occupancy(Ctx* ctx, int g, Program* prog, const char* kernel, int block, size_t smem) {
+  const std::string key = std::string(kernel) + "/" + std::to_string(block) + "/" + std::to_string(smem);
+  auto it = prog->occ.find(key);
+  if (it != prog->occ.end()) return it->second;
   ctx->set_device(g);
   cudaKernel_t k = get_kernel(prog, kernel, smem);
   int nb = 0;
   SKL_CUDA(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, (const void*)k, block, smem));
+  prog->occ[key] = nb;
   return nb;
 }
 

@@ -43,6 +43,8 @@ static void free_part(Cont* c, int g) {
 
 void cont_destroy(Cont* c) {
   Ctx* ctx = c->ctx;
+  materialize_dependents(c);
+  drop_lazy(c);
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) free_part(c, g);
   if (c->host) cudaFreeHost(c->host);
   ctx->conts.erase(c);
@@ -103,6 +105,8 @@ void mark_written(Cont* c) {
 }
 
 void prepare_output(Cont* c, const Dist& d, size_t spare) {
+  materialize_dependents(c);  // deferred readers of c's old value run first
+  drop_lazy(c);               // a deferred value of c itself is discarded
   if (spare > c->spare_halo) c->spare_halo = spare;
   // buffers that must move would lose data; outputs are overwritten anyway
   set_layout(c, d);
@@ -143,6 +147,7 @@ void host_upload(Cont* c, const void* host) {
 }
 
 static void sync_local(Ctx* ctx) {
+  if (ctx->capturing) fail(SKL_ERR_INVALID_ARG, "host-visible results are not available while capturing a graph");
   for (auto& d : ctx->dev) {
     SKL_CUDA(cudaSetDevice(d.phys));
     SKL_CUDA(cudaStreamSynchronize(d.stream));
@@ -171,6 +176,8 @@ struct GatherPtrs : PtrFn {
 
 void host_download(Cont* c, void* host) {
   Ctx* ctx = c->ctx;
+  if (ctx->capturing) fail(SKL_ERR_INVALID_ARG, "host-visible results are not available while capturing a graph");
+  materialize(c);
   const size_t ub = c->unit_bytes();
   if (!c->dev_valid) {
     if (c->host_valid && c->host && host != c->host) std::memcpy(host, c->host, c->bytes());
@@ -224,6 +231,7 @@ void host_download(Cont* c, void* host) {
 void download_part(Cont* c, int g, void* host, size_t* first, size_t* n) {
   Ctx* ctx = c->ctx;
   if (!ctx->is_local(g)) fail(SKL_ERR_INVALID_ARG, "device is not local to this process");
+  materialize(c);
   if (!c->dev_valid) fail(SKL_ERR_DISTRIBUTION, "container has no device data");
   if (c->dist.kind == DCOPY && c->diverged && c->combine) copy_combine_to_copy(c);
   const Range r = core_range(c->units(), ctx->G, c->dist, g);
@@ -238,6 +246,9 @@ void download_part(Cont* c, int g, void* host, size_t* first, size_t* n) {
 }
 
 void* host_mirror(Cont* c, int mode) {
+  if (mode & SKL_WRITE) materialize_dependents(c);
+  if (mode & SKL_READ) materialize(c);
+  else drop_lazy(c);
   if (!c->host) SKL_CUDA(cudaHostAlloc(&c->host, std::max<size_t>(c->bytes(), 1), cudaHostAllocPortable));
   if ((mode & SKL_READ) && !c->host_valid) {
     host_download(c, c->host);
@@ -253,6 +264,8 @@ void* host_mirror(Cont* c, int mode) {
 
 void fill(Cont* c, const void* value) {
   Ctx* ctx = c->ctx;
+  materialize_dependents(c);
+  drop_lazy(c);
   if (c->dist.kind == DNONE) {
     char* h = (char*)host_mirror(c, SKL_WRITE);
     for (size_t i = 0; i < c->rows * c->cols; ++i) std::memcpy(h + i * c->elt, value, c->elt);
@@ -385,6 +398,7 @@ static void redistribute(Cont* c, const Dist& to) {
 
 void ensure(Cont* c, const Dist& d, bool halo) {
   if (d.kind == DNONE) fail(SKL_ERR_DISTRIBUTION, "no distribution");
+  materialize(c);  // a deferred Zip/Map result is computed before it is used
   if (c->dev_valid && c->dist.kind == DCOPY && c->diverged && c->combine && !(d == c->dist)) {
     combine_to_block(c);
   }

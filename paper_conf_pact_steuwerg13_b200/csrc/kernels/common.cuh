@@ -8,7 +8,8 @@ typedef unsigned long long skl_u64;
 // stores are evict-first, the right policy for read-once / write-once streams.
 __device__ __forceinline__ uint4 skl_ld16(const void* p) {
   uint4 r;
-  asm volatile("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
+  // not volatile: a read-only load the compiler may hoist / batch (MLP)
+  asm("ld.global.nc.L1::no_allocate.v4.u32 {%0,%1,%2,%3}, [%4];"
                : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
   return r;
 }

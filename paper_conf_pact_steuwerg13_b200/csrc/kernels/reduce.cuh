@@ -15,8 +15,69 @@
 #define SKL_NW (SKL_BLOCK / 32)
 #define SKL_RTILE (32 * SKL_RVEC)
 
-template <int RVEC>
-__device__ __forceinline__ void skl_reduce_body(const SKL_T* __restrict__ in, skl_u64 n, skl_u64 wseg,
+// Element loaders: the plain Reduce reads its input; the fused form (lazy
+// Zip/Map -> Reduce) computes each element from the Zip's inputs
+// on the fly, so the intermediate vector never exists (8 instead of 16 bytes per
+// element for the dot product of Listing 1.1).
+struct SklLoadPlain {
+  const SKL_T* __restrict__ in;
+  template <int RVEC>
+  __device__ __forceinline__ void load(skl_u64 e, int cnt, SKL_T (&x)[RVEC]) const {
+    if (RVEC > 1 && cnt == RVEC) {
+      SklChunk<SKL_T, RVEC> ch;
+      ch.q[0] = skl_ld16(in + e);
+#pragma unroll
+      for (int k = 0; k < RVEC; ++k) x[k] = ch.e[k];
+    } else {
+#pragma unroll
+      for (int k = 0; k < RVEC; ++k)
+        if (k < cnt) x[k] = in[e + k];
+    }
+  }
+};
+#if SKL_FUSED
+struct SklLoadZip {
+  const SKL_ZL* __restrict__ l;
+  const SKL_ZR* __restrict__ r;
+  __device__ __forceinline__ SKL_T f(const SKL_ZL& a, const SKL_ZR& b) const {
+#if SKL_ZMAP
+    (void)b;
+    return SKL_ZFUNC(a);
+#else
+    return SKL_ZFUNC(a, b);
+#endif
+  }
+  template <int RVEC>
+  __device__ __forceinline__ void load(skl_u64 e, int cnt, SKL_T (&x)[RVEC]) const {
+    if (RVEC > 1 && cnt == RVEC) {
+      SklChunk<SKL_ZL, RVEC> a;
+      a.q[0] = skl_ld16(l + e);
+#if SKL_ZMAP
+#pragma unroll
+      for (int k = 0; k < RVEC; ++k) x[k] = f(a.e[k], a.e[k]);
+#else
+      SklChunk<SKL_ZR, RVEC> b;
+      b.q[0] = skl_ld16(r + e);
+#pragma unroll
+      for (int k = 0; k < RVEC; ++k) x[k] = f(a.e[k], b.e[k]);
+#endif
+    } else {
+#pragma unroll
+      for (int k = 0; k < RVEC; ++k)
+        if (k < cnt) {
+#if SKL_ZMAP
+          x[k] = f(l[e + k], l[e + k]);
+#else
+          x[k] = f(l[e + k], r[e + k]);
+#endif
+        }
+    }
+  }
+};
+#endif
+
+template <int RVEC, class Loader>
+__device__ __forceinline__ void skl_reduce_body(const Loader& ld, skl_u64 n, skl_u64 wseg,
                                                 SKL_T* partials, unsigned* counter, SKL_T* result) {
   SklOp op;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -25,23 +86,34 @@ __device__ __forceinline__ void skl_reduce_body(const SKL_T* __restrict__ in, sk
   const skl_u64 hi = lo + wseg < n ? lo + wseg : n;
   bool has = false;
   SKL_T acc;
-  for (skl_u64 t = lo; t < hi; t += (skl_u64)SKL_RTILE * SKL_RU) {
+  skl_u64 t = lo;
+  // fast path: SKL_RU full warp-tiles, no per-tile branches, so all loads of the
+  // iteration are issued before the first use (memory-level parallelism)
+  for (; t + (skl_u64)SKL_RTILE * SKL_RU <= hi; t += (skl_u64)SKL_RTILE * SKL_RU) {
+    SKL_T x[SKL_RU][RVEC];
+#pragma unroll
+    for (int u = 0; u < SKL_RU; ++u)
+      ld.template load<RVEC>(t + (skl_u64)u * SKL_RTILE + (skl_u64)lane * RVEC, RVEC, x[u]);
+#pragma unroll
+    for (int u = 0; u < SKL_RU; ++u) {
+      SKL_T v = x[u][0];
+#pragma unroll
+      for (int k = 1; k < RVEC; ++k) v = op(v, x[u][k]);
+      v = skl_warp_fold(v, 32, op);
+      v = skl_shfl(v, 0);
+      acc = has ? op(acc, v) : v;
+      has = true;
+    }
+  }
+  // ragged end of the segment
+  for (; t < hi; t += (skl_u64)SKL_RTILE * SKL_RU) {
     SKL_T x[SKL_RU][RVEC];
     int cnt[SKL_RU];
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u) {
       const skl_u64 e = t + (skl_u64)u * SKL_RTILE + (skl_u64)lane * RVEC;
       cnt[u] = e >= hi ? 0 : (hi - e >= (skl_u64)RVEC ? RVEC : (int)(hi - e));
-      if (RVEC > 1 && cnt[u] == RVEC) {
-        SklChunk<SKL_T, RVEC> ch;
-        ch.q[0] = skl_ld16(in + e);
-#pragma unroll
-        for (int k = 0; k < RVEC; ++k) x[u][k] = ch.e[k];
-      } else {
-#pragma unroll
-        for (int k = 0; k < RVEC; ++k)
-          if (k < cnt[u]) x[u][k] = in[e + k];
-      }
+      ld.template load<RVEC>(e, cnt[u], x[u]);
     }
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u) {
@@ -83,13 +155,18 @@ __device__ __forceinline__ void skl_reduce_body(const SKL_T* __restrict__ in, sk
   }
   if (gridDim.x == 1) return;
   __syncthreads();
-  if (!s_last || warp != 0) return;
-  // last block: fold the block partials in block order
+  if (!s_last) return;
+  // last block: fold the block partials in block order, every warp folding one
+  // contiguous slice (one L2 round trip per 32 x SKL_NW partials), then the warp
+  // results in warp order
   __threadfence();
+  const unsigned per = (gridDim.x + SKL_NW - 1) / SKL_NW;
+  const unsigned wlo = warp * per;
+  const unsigned whi = wlo + per < gridDim.x ? wlo + per : gridDim.x;
   bool h2 = false;
   SKL_T a2;
-  for (unsigned b0 = 0; b0 < gridDim.x; b0 += 32) {
-    const unsigned nb = gridDim.x - b0 < 32 ? gridDim.x - b0 : 32;
+  for (unsigned b0 = wlo; b0 < whi; b0 += 32) {
+    const unsigned nb = whi - b0 < 32 ? whi - b0 : 32;
     SKL_T v;
     if ((unsigned)lane < nb) v = skl_ldcg(partials + b0 + lane);
     v = skl_warp_fold(v, (int)nb, op);
@@ -97,8 +174,17 @@ __device__ __forceinline__ void skl_reduce_body(const SKL_T* __restrict__ in, sk
     a2 = h2 ? op(a2, v) : v;
     h2 = true;
   }
+  __syncthreads();  // s_w / s_h reused
   if (lane == 0) {
-    *result = a2;
+    s_h[warp] = h2;
+    if (h2) s_w[warp] = a2;
+  }
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    SKL_T r = s_w[0];
+    for (int i = 1; i < SKL_NW; ++i)
+      if (s_h[i]) r = op(r, s_w[i]);
+    *result = r;
     *counter = 0u;  // ready for the next launch (stream-ordered)
   }
 }
@@ -106,13 +192,26 @@ __device__ __forceinline__ void skl_reduce_body(const SKL_T* __restrict__ in, sk
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_reduce_vec(const SKL_T* __restrict__ in, skl_u64 n, skl_u64 wseg, SKL_T* partials,
                unsigned* counter, SKL_T* result) {
-  skl_reduce_body<SKL_RVEC>(in, n, wseg, partials, counter, result);
+  skl_reduce_body<SKL_RVEC>(SklLoadPlain{in}, n, wseg, partials, counter, result);
 }
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_reduce_sc(const SKL_T* __restrict__ in, skl_u64 n, skl_u64 wseg, SKL_T* partials,
               unsigned* counter, SKL_T* result) {
-  skl_reduce_body<1>(in, n, wseg, partials, counter, result);
+  skl_reduce_body<1>(SklLoadPlain{in}, n, wseg, partials, counter, result);
 }
+
+#if SKL_FUSED
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_reduce_zip_vec(const SKL_ZL* __restrict__ l, const SKL_ZR* __restrict__ r, skl_u64 n, skl_u64 wseg,
+                   SKL_T* partials, unsigned* counter, SKL_T* result) {
+  skl_reduce_body<SKL_RVEC>(SklLoadZip{l, r}, n, wseg, partials, counter, result);
+}
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_reduce_zip_sc(const SKL_ZL* __restrict__ l, const SKL_ZR* __restrict__ r, skl_u64 n, skl_u64 wseg,
+                  SKL_T* partials, unsigned* counter, SKL_T* result) {
+  skl_reduce_body<1>(SklLoadZip{l, r}, n, wseg, partials, counter, result);
+}
+#endif
 
 // Ordered fold of `nrep` staged values per element (copy(+) -> block combine,
 // reading A25; and the cross-GPU fold of Reduce partials): out[i] =

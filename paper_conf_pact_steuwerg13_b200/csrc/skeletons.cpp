@@ -196,6 +196,10 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
 
 void skel_destroy(Skel* s) {
   Ctx* ctx = s->ctx;
+  // deferred results of this skeleton must exist before it goes away
+  for (Cont* c : std::vector<Cont*>(ctx->conts.begin(), ctx->conts.end()))
+    if (c->lazy.s == s) materialize(c);
+  for (Skel* k : ctx->skels) k->fused.erase(s);
   for (auto* m : {&s->scratch_red, &s->scratch_scan, &s->scratch_stage})
     for (auto& kv : *m)
       if (kv.second.ptr && ctx->is_local(kv.first)) device_free(ctx, kv.first, kv.second.ptr);
@@ -248,6 +252,7 @@ ExtraArgs prepare_extras(Skel* s, const skl_arg* extra, int nextra) {
       // A27: a container argument is read at arbitrary indices: every device needs
       // the whole container, i.e. the copy distribution.
       ensure(c, Dist{DCOPY, 0}, false);
+      if (extra[k].mode & SKL_WRITE) materialize_dependents(c);  // c changes in place
       ea.conts[(size_t)k] = c;
       ea.modes[(size_t)k] = extra[k].mode ? extra[k].mode : SKL_READ;
     } else {
@@ -290,6 +295,17 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     // A7: the right input follows the left input's distribution
     if (!(elementwise(in2->dist) == din && in2->dev_valid)) ensure(in2, din, false);
     else ensure(in2, in2->dist, false);
+  }
+  if (*out == nullptr && nextra == 0 && s->tout != SKL_VOID && ctx->lazy_fusion &&
+      in->dist.kind != DOVERLAP && (!in2 || in2->dist.kind != DOVERLAP)) {
+    // deferred (lazy fusion): nothing runs until the result is used
+    Cont* o = cont_create(ctx, s->tout, in->rows, in->cols, in->matrix);
+    o->lazy = Lazy{s, in, in2, din};
+    o->dist = din;
+    in->dependents.push_back(o);
+    if (in2 && in2 != in) in2->dependents.push_back(o);
+    *out = o;
+    return;
   }
   ExtraArgs ea = prepare_extras(s, extra, nextra);
   Cont* o = nullptr;
@@ -341,6 +357,40 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
   finish_extras(ctx, ea, ndev);
 }
 
+// ------------------------------------------------------------------ lazy fusion
+void drop_lazy(Cont* c) {
+  if (!c->lazy.s) return;
+  for (Cont* in : {c->lazy.l, c->lazy.r})
+    if (in) {
+      auto& v = in->dependents;
+      v.erase(std::remove(v.begin(), v.end(), c), v.end());
+    }
+  c->lazy = Lazy();
+}
+
+void materialize(Cont* c) {
+  if (!c->lazy.s) return;
+  const Lazy L = c->lazy;
+  drop_lazy(c);
+  Cont* o = c;
+  c->dist = Dist();  // run_elementwise sets the output distribution
+  // containers deferred on c want exactly the value computed now: keep them
+  // deferred (prepare_output would otherwise materialise them first)
+  std::vector<Cont*> deps;
+  deps.swap(c->dependents);
+  try {
+    run_elementwise(L.s, L.l, L.r, &o, nullptr, 0);
+  } catch (...) {
+    c->dependents.swap(deps);
+    throw;
+  }
+  c->dependents.swap(deps);
+}
+
+void materialize_dependents(Cont* c) {
+  while (!c->dependents.empty()) materialize(c->dependents.back());
+}
+
 void run_map(Skel* s, Cont* in, Cont** out, const skl_arg* extra, int nextra) {
   if (s->kind != K_MAP) fail(SKL_ERR_INVALID_ARG, "not a Map skeleton");
   run_elementwise(s, in, nullptr, out, extra, nextra);
@@ -352,15 +402,30 @@ void run_zip(Skel* s, Cont* l, Cont* r, Cont** out, const skl_arg* extra, int ne
 }
 
 // ------------------------------------------------------------------ Reduce
-// One device's fold of n elements at `in` into `result` (device pointer).
-static void reduce_on_device(Skel* s, int g, const void* in, size_t n, void* result) {
+// What a device folds: the plain input, or (lazy fusion) the elements of a
+// deferred Zip/Map computed from its inputs on the fly.
+struct RedSrc {
+  Program* prog;
+  const char* kvec;
+  const char* ksc;
+  const void* p1;
+  const void* p2;  // fused Zip: right input (Map: unused)
+  bool vec_ok;
+};
+
+// One device's fold of n elements into `result` (device pointer).
+static void reduce_on_device(Skel* s, int g, const RedSrc& src, size_t n, void* result) {
   Ctx* ctx = s->ctx;
   const size_t st = ctx->type(s->tin).size;
   const int nw = s->block / 32;
-  const bool vec = (16 % st == 0) && aligned16(in);
+  const bool vec = (16 % st == 0) && src.vec_ok;
   const size_t rtile = 32 * (vec ? 16 / st : 1);
   const size_t ru = 4;
-  const size_t max_blocks = (size_t)ctx->D(g).sm_count * (2048 / (size_t)s->block);
+  // one wave of resident blocks (each warp owns a long segment: a second wave
+  // would double the time)
+  const char* kname = vec ? src.kvec : src.ksc;
+  const size_t occ = (size_t)std::max(1, occupancy(ctx, g, src.prog, kname, s->block, 0));
+  const size_t max_blocks = (size_t)ctx->D(g).sm_count * occ;
   size_t nblocks = std::min(max_blocks, std::max<size_t>(1, ceil_div(n, (size_t)nw * rtile * ru)));
   size_t wseg = ceil_div(ceil_div(n, nblocks * (size_t)nw), rtile) * rtile;
   nblocks = ceil_div(n, (size_t)nw * wseg);
@@ -369,9 +434,12 @@ static void reduce_on_device(Skel* s, int g, const void* in, size_t n, void* res
   void* counter = sc;
   void* partials = sc + 16;
   unsigned long long nn = n, ws = wseg;
-  void* args[] = {(void*)&in, &nn, &ws, &partials, &counter, &result};
-  launch(ctx, g, s->prog, vec ? "skl_reduce_vec" : "skl_reduce_sc", dim3((unsigned)nblocks),
-         dim3(s->block), 0, args);
+  const void* p1 = src.p1;
+  const void* p2 = src.p2;
+  void* args1[] = {(void*)&p1, &nn, &ws, &partials, &counter, &result};
+  void* args2[] = {(void*)&p1, (void*)&p2, &nn, &ws, &partials, &counter, &result};
+  launch(ctx, g, src.prog, vec ? src.kvec : src.ksc, dim3((unsigned)nblocks), dim3(s->block), 0,
+         src.p2 || std::strcmp(src.kvec, "skl_reduce_zip_vec") == 0 ? args2 : args1);
 }
 
 void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
@@ -385,15 +453,71 @@ void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int n
   launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(s->block), 0, args);
 }
 
+// Fused program: the Zip/Map's and the Reduce's customising functions in one
+// NVRTC program (each renamed by a macro, so both may be called "func"), the
+// Reduce template reading through SklLoadZip.  nullptr if they do not compile
+// together (then the Zip/Map is materialised instead).
+static Program* fused_program(Skel* s, Skel* z) {
+  auto it = s->fused.find(z);
+  if (it != s->fused.end()) return it->second;
+  Ctx* ctx = s->ctx;
+  const size_t st = ctx->type(s->tin).size;
+  const std::string zf = "skl_zf_" + z->entry, rf = "skl_rf_" + s->entry;
+  std::string defs = defs_common(ctx, rf, s->block);
+  defs += "#define SKL_T " + tname(ctx, s->tin) + "\n";
+  defs += "#define SKL_RVEC " + std::to_string((16 % st == 0) ? 16 / st : 1) + "\n#define SKL_RU 4\n";
+  defs += "#define SKL_FUSED 1\n#define SKL_ZL " + tname(ctx, z->tin) + "\n";
+  defs += "#define SKL_ZR " + tname(ctx, z->kind == K_ZIP ? z->tin2 : z->tin) + "\n";
+  defs += std::string("#define SKL_ZMAP ") + (z->kind == K_MAP ? "1" : "0") + "\n#define SKL_ZFUNC " + zf + "\n";
+  const std::string body =
+      "\n#define " + z->entry + " " + zf + "\n#line 1 \"user_source_zip\"\n" + z->user_src + "\n#undef " +
+      z->entry + "\n#define " + s->entry + " " + rf + "\n#line 1 \"user_source_reduce\"\n" + s->user_src +
+      "\n#undef " + s->entry + "\n#line 1 \"skeleton_template\"\n" + kernel_template("common.cuh") +
+      kernel_template("op.cuh") + kernel_template("reduce.cuh");
+  Program* p = nullptr;
+  try {
+    p = compile(ctx, defs + program_source(ctx, body), nullptr);
+  } catch (const Error&) {
+    p = nullptr;
+  }
+  s->fused[z] = p;
+  return p;
+}
+
 void run_reduce(Skel* s, Cont* in, Cont** out) {
   if (s->kind != K_REDUCE) fail(SKL_ERR_INVALID_ARG, "not a Reduce skeleton");
   Ctx* ctx = s->ctx;
   if (in->elt != ctx->type(s->tin).size) fail(SKL_ERR_TYPE, "input type does not match the skeleton");
   if (in->rows * in->cols == 0) fail(SKL_ERR_EMPTY, "reduce of an empty container (A11)");
-  if (in->dist.kind == DCOPY && in->diverged && in->combine) ensure(in, Dist{DCOPY, 0}, false);
-  const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));
-  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  // lazy fusion: fold a deferred Zip/Map straight from its inputs
+  Lazy L = in->lazy;
+  Program* fp = (L.s && ctx->lazy_fusion) ? fused_program(s, L.s) : nullptr;
+  Dist din;
+  if (fp) {
+    din = L.d;
+    ensure(L.l, L.l->dist.kind == DOVERLAP ? L.l->dist : din, false);
+    if (L.r) {
+      if (!(elementwise(L.r->dist) == din && L.r->dev_valid)) ensure(L.r, din, false);
+      else ensure(L.r, L.r->dist, false);
+    }
+  } else {
+    if (in->dist.kind == DCOPY && in->diverged && in->combine) ensure(in, Dist{DCOPY, 0}, false);
+    din = elementwise(default_dist(in, Dist{DBLOCK, 0}));
+    ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  }
   Cont* o = output_for(ctx, out, s->tin, 1, 1, false);
+  auto source = [&](int g, const Range& r) {
+    if (fp) {
+      const void* a = part_ptr(L.l, g, r.lo);
+      const void* b = L.r ? part_ptr(L.r, g, r.lo) : nullptr;
+      const bool eq = ctx->type(L.s->tin).size == in->elt &&
+                      (!L.r || ctx->type(L.s->tin2).size == in->elt);
+      return RedSrc{fp, "skl_reduce_zip_vec", "skl_reduce_zip_sc", a, b,
+                    eq && aligned16(a) && (!b || aligned16(b))};
+    }
+    const void* a = part_ptr(in, g, r.lo);
+    return RedSrc{s->prog, "skl_reduce_vec", "skl_reduce_sc", a, nullptr, aligned16(a)};
+  };
   // participants, in device order: devices whose core holds elements.  A copy
   // input is reduced once per process (replicas are identical).
   std::vector<int> parts;
@@ -405,7 +529,7 @@ void run_reduce(Skel* s, Cont* in, Cont** out) {
     if (!core_range(in->units(), ctx->G, din, g).empty()) parts.push_back(g);
   }
   // result distribution: single(first participant) in one process; copy across
-  // processes so every rank's getValue() works (SPMD).
+  // processes so every rank's getValue() works (SPMD, A33).
   const bool cross = parts.size() > 1;
   Dist dout = ctx->dist_mode ? Dist{DCOPY, 0} : Dist{DSINGLE, parts[0]};
   if (!ctx->dist_mode && cross) dout = Dist{DSINGLE, 0};
@@ -416,7 +540,7 @@ void run_reduce(Skel* s, Cont* in, Cont** out) {
     for (int g : parts) {
       if (!ctx->is_local(g)) continue;
       const Range r = core_range(in->units(), ctx->G, din, g);
-      reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, part_ptr(o, g, 0));
+      reduce_on_device(s, g, source(g, r), r.size() * in->cols, part_ptr(o, g, 0));
     }
     mark_written(o);
     return;
@@ -434,7 +558,7 @@ void run_reduce(Skel* s, Cont* in, Cont** out) {
     if (!ctx->is_local(g)) continue;
     const Range r = core_range(in->units(), ctx->G, din, g);
     // partial lands in its own slot i on its own device
-    reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, (char*)stage[g] + (size_t)i * st);
+    reduce_on_device(s, g, source(g, r), r.size() * in->cols, (char*)stage[g] + (size_t)i * st);
   }
   std::vector<Transfer> tr;
   for (int dg : dsts)
@@ -485,7 +609,11 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
       const int g = parts[(size_t)i];
       if (!ctx->is_local(g)) continue;
       const Range r = core_range(in->units(), ctx->G, din, g);
-      reduce_on_device(s, g, part_ptr(in, g, r.lo), r.size() * in->cols, (char*)totals[g] + (size_t)i * st);
+      {
+        const void* a = part_ptr(in, g, r.lo);
+        reduce_on_device(s, g, RedSrc{s->prog, "skl_reduce_vec", "skl_reduce_sc", a, nullptr, aligned16(a)},
+                         r.size() * in->cols, (char*)totals[g] + (size_t)i * st);
+      }
     }
     std::vector<Transfer> tr;
     for (int j = 0; j < P; ++j)

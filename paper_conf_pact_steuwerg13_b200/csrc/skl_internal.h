@@ -79,6 +79,7 @@ struct Program {
   cudaLibrary_t lib = nullptr;
   std::map<std::string, cudaKernel_t> kernels;
   std::map<std::string, size_t> smem_set;  // dynamic smem attribute already raised
+  std::map<std::string, int> occ;          // resident blocks/SM per (kernel, block, smem)
 };
 
 // ------------------------------------------------------------------ devices
@@ -98,6 +99,7 @@ struct Ctx {
   int first_local = 0, nlocal = 1;
   bool dist_mode = false;      // one process per GPU, NCCL between ranks
   bool offline = false;        // no devices: compile only (skl_init_offline)
+  bool capturing = false;      // a CUDA graph capture is open on the device stream
   int rank = 0, world = 1;
   void* nccl_comm = nullptr;   // ncclComm_t
   std::vector<Device> dev;     // local devices, index g - first_local
@@ -115,6 +117,7 @@ struct Ctx {
   int scan_spin_ns = 0;        // Scan look-back spin back-off (__nanosleep)
   int scan_minb = 4;           // Scan per-tile kernel: min resident blocks (launch bounds)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
+  int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest
   // measured); 2 = one block per tile, warp-wide look-back; 0 = persistent
   // chunked (L2 re-read); 1 = measurement only: no look-back (wrong results)
@@ -138,8 +141,20 @@ struct Part {
   size_t cap_bytes = 0;
 };
 
+// A Zip/Map called without an output container is deferred (lazy fusion,
+// SURVEY §8(f)1): a Reduce that consumes it computes the elements on the fly;
+// any other use, or a write to an input, materialises it first.
+struct Lazy {
+  Skel* s = nullptr;  // the deferred Zip/Map (nullptr: not lazy)
+  Cont* l = nullptr;
+  Cont* r = nullptr;  // Zip's right input
+  Dist d;             // distribution the elements are computed in
+};
+
 struct Cont {
   Ctx* ctx = nullptr;
+  Lazy lazy;
+  std::vector<Cont*> dependents;  // lazy containers that read this one
   int type = 0;
   size_t elt = 0;          // element bytes
   bool matrix = false;
@@ -176,6 +191,10 @@ void download_part(Cont* c, int g, void* host, size_t* first, size_t* n);
 void fill(Cont* c, const void* value);
 void* host_mirror(Cont* c, int mode);
 void copy_combine_to_copy(Cont* c);  // fold diverged replicas, keep copy
+// lazy fusion (skeletons.cpp)
+void materialize(Cont* c);             // run c's deferred Zip/Map, if any
+void materialize_dependents(Cont* c);  // before c's values change
+void drop_lazy(Cont* c);               // c is overwritten or destroyed
 
 // comm.cpp — execute transfers between per-device buffers.  srcp/dstp resolve
 // (device, unit) to a device pointer for LOCAL devices.
@@ -230,6 +249,7 @@ struct Skel {
   int scan_fstride = 16;  // Scan: status word spacing in 8-byte units
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
+  std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
 };
 Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int tin, int tin2,
                   int tout, const int* extra, int nextra, int d, int boundary, const void* neutral);

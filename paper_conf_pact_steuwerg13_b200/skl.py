@@ -89,6 +89,8 @@ def lib():
         "skl_reduce_run": [vp, vp, pp], "skl_scan_run": [vp, vp, pp], "skl_mapoverlap_run": [vp, vp, pp],
         "skl_scalar_get": [vp, vp, sz],
         "skl_skel_cubin": [vp, vp, sz, C.POINTER(sz)], "skl_skel_source": [vp, C.c_char_p, sz, C.POINTER(sz)],
+        "skl_capture_begin": [vp], "skl_capture_end": [vp, pp], "skl_graph_launch": [vp],
+        "skl_graph_destroy": [vp],
         "skl_plan_range": [sz, i, i, i, i, i, C.POINTER(sz), C.POINTER(sz)],
         "skl_plan_transfers": [sz, i, i, i, i, i, C.POINTER(C.c_int64), sz, C.POINTER(sz)],
     }
@@ -184,6 +186,21 @@ class Context:
         check(lib().skl_type_struct(self._h, name.encode(), decl.encode(), size, align, C.byref(t)))
         return t.value
 
+    def capture(self, fn) -> "Graph":
+        """Record fn() (skeleton calls on this context) as a CUDA graph."""
+        check(lib().skl_capture_begin(self._h))
+        try:
+            fn()
+        except BaseException:
+            h = C.c_void_p()
+            lib().skl_capture_end(self._h, C.byref(h))
+            if h.value:
+                lib().skl_graph_destroy(h)
+            raise
+        h = C.c_void_p()
+        check(lib().skl_capture_end(self._h, C.byref(h)))
+        return Graph(self, h)
+
     def finalize(self):
         if self._live:
             check(lib().skl_finalize(self._h))
@@ -194,6 +211,22 @@ class Context:
 
     def __exit__(self, *a):
         self.finalize()
+
+
+class Graph:
+    """A recorded sequence of skeleton calls (skl_capture_begin/end)."""
+
+    def __init__(self, ctx: Context, h):
+        self.ctx = ctx
+        self._h = h
+
+    def launch(self):
+        check(lib().skl_graph_launch(self._h))
+
+    def destroy(self):
+        if self._h:
+            check(lib().skl_graph_destroy(self._h))
+            self._h = None
 
 
 # ---------------------------------------------------------------- containers
@@ -295,6 +328,16 @@ class Container:
         if self._h:
             check(lib().skl_cont_destroy(self._h))
             self._h = None
+
+    def __del__(self):
+        # containers die with their Python object (device memory freed stream-
+        # ordered); after Context.finalize() the library already freed them
+        try:
+            if self._h and self.ctx._live:
+                lib().skl_cont_destroy(self._h)
+                self._h = None
+        except Exception:
+            pass
 
 
 class Vector(Container):

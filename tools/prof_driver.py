@@ -52,11 +52,9 @@ def main(which: str, reps: int = 3):
         a = S.Vector(ctx, S.F32, n).set_distribution(S.BLOCK).fill(1.0)
         b = S.Vector(ctx, S.F32, n).set_distribution(S.BLOCK).fill(2.0)
         mult, sm = S.Zip(ctx, A.MULT, S.F32, S.F32, S.F32), S.Reduce(ctx, A.SUM, S.F32)
-        c = mult(a, b)
-        s = sm(c)
+        s = sm(mult(a, b))
         for _ in range(reps):
-            mult(a, b, out=c)
-            sm(c, out=s)
+            sm(mult(a, b), out=s)   # fused Zip -> Reduce (one kernel)
     elif which == "lmosem":
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
