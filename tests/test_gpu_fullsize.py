@@ -1,0 +1,146 @@
+"""Parity at BASELINE.json's full sizes, in the launch configurations bench.py
+times: whole-output comparison where the oracle finishes in seconds
+(Mandelbrot 4096x3072, dot 2^20), sampled outputs otherwise (row bands of the
+8192^2 stencils computed by the oracle with their halo; chunks of the 2^30 scan
+carried from the GPU's preceding element, which pins each chunk exactly; a
+1/50 sample of the 10^7 LM OSEM events)."""
+import numpy as np
+import pytest
+
+import oracle as O
+from gpu_util import rel_l2, require_gpu
+from paper_conf_pact_steuwerg13_b200 import apps as A
+from paper_conf_pact_steuwerg13_b200 import inputs as I
+from paper_conf_pact_steuwerg13_b200 import skl as S
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def ctx():
+    require_gpu()
+    c = S.Context(1)
+    yield c
+    c.finalize()
+
+
+def test_mandelbrot_full_image_bitexact(ctx):
+    ctx.set_option("block_threads", 512)
+    ctx.set_option("map_unroll", 2)
+    m = S.Map(ctx, A.mandelbrot_unrolled(1000), S.F32X2, S.U32)
+    ctx.set_option("block_threads", 256)
+    ctx.set_option("map_unroll", 4)
+    grid = I.mandel_grid(3072, 4096)
+    x = S.Matrix(ctx, S.F32X2, 3072, 4096).set_distribution(S.BLOCK)
+    x.copy_in(grid)
+    got = m(x).to_numpy()
+    ref, tot = O.mandelbrot(grid, 1000)
+    assert np.array_equal(got, ref)
+    assert int(got.astype(np.uint64).sum()) == tot == 2888511137
+
+
+def test_dot_product_2_20_fused(ctx):
+    n = 1 << 20
+    a, b = I.uniform_f32(I.SEED_DOT_A, n), I.uniform_f32(I.SEED_DOT_B, n)
+    va = S.Vector.from_numpy(ctx, a).set_distribution(S.BLOCK)
+    vb = S.Vector.from_numpy(ctx, b).set_distribution(S.BLOCK)
+    s = S.Reduce(ctx, A.SUM, S.F32)(S.Zip(ctx, A.MULT, S.F32, S.F32, S.F32)(va, vb))
+    ref = O.reduce_(O.OP_ADD_F32, O.zip_(O.OZ_MULT_F32, a, b))
+    assert abs(float(s.scalar()) - ref) <= 1e-5 * abs(ref)
+
+
+@pytest.mark.parametrize("name", ["sobel", "gauss"])
+def test_stencils_8192_bands(ctx, name):
+    R = C = 8192
+    if name == "sobel":
+        img = I.image_u8(I.SEED_SOBEL, R, C)
+        mo = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+    else:
+        img = I.image_f32(I.SEED_GAUSS, R, C)
+        mo = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    out = mo(S.Matrix.from_numpy(ctx, img)).to_numpy()
+    for r0 in (0, 4000, R - 64):  # top edge, interior, bottom edge
+        lo, hi = max(0, r0 - 8), min(R, r0 + 72)
+        sub = img[lo:hi]
+        ref = (O.mapoverlap2d(O.OS_SOBEL, sub, 1, O.OB_NEUTRAL, 0) if name == "sobel"
+               else O.mapoverlap2d(O.OS_GAUSS5, sub, 2, O.OB_NEAREST, 0.0))
+        # rows of the band whose window lies inside [lo, hi) (or at a true edge)
+        a = r0 - lo if r0 > 0 else 0
+        b = a + 64
+        assert np.array_equal(out[lo + a:lo + b], ref[a:b]), (name, r0)
+
+
+@pytest.mark.parametrize("dt", ["i32", "f32"])
+def test_scan_2_30_sampled_chunks(ctx, dt):
+    import torch
+    n = 1 << 30
+    gen = torch.Generator(device="cuda").manual_seed(3 if dt == "i32" else 4)
+    src = (torch.randint(-1000, 1001, (n,), dtype=torch.int32, device="cuda", generator=gen) if dt == "i32"
+           else torch.rand((n,), dtype=torch.float32, device="cuda", generator=gen))
+    t = S.I32 if dt == "i32" else S.F32
+    sc = S.Scan(ctx, A.ADD_I32 if dt == "i32" else A.ADD, t)
+    v = S.Vector(ctx, t, n).set_distribution(S.BLOCK)
+    v.fill(0)
+    ptr, first, cnt = v.local_part(0)
+
+    class View:
+        __cuda_array_interface__ = {"shape": (cnt,), "typestr": "<i4" if dt == "i32" else "<f4",
+                                    "data": (ptr, False), "version": 3, "strides": None}
+    ctx.sync()
+    torch.as_tensor(View(), device="cuda").copy_(src)
+    torch.cuda.synchronize()
+    out = sc(v)
+    optr, _, ocnt = out.local_part(0)
+
+    class OView:
+        __cuda_array_interface__ = {"shape": (ocnt,), "typestr": "<i4" if dt == "i32" else "<f4",
+                                    "data": (optr, False), "version": 3, "strides": None}
+    ctx.sync()
+    got = torch.as_tensor(OView(), device="cuda")
+    for c0 in (0, 8191, 1 << 20, n // 2 + 12345, n - 100000):
+        xin = src[c0:c0 + 100000].cpu().numpy()
+        g = got[c0:c0 + 100000].cpu().numpy()
+        if dt == "i32":
+            prev = 0 if c0 == 0 else int(got[c0 - 1].item())
+            ref = (O.scan(O.OP_ADD_I32, xin).astype(np.int64) + prev).astype(np.int32)
+            assert np.array_equal(g, ref), c0
+        else:
+            prev = 0.0 if c0 == 0 else float(got[c0 - 1].item())
+            assert rel_l2(g, O.scan(O.OP_ADD_F32, xin) + prev) <= 1e-5, c0
+    if dt == "i32":
+        assert int(got[-1].item()) == int(np.int32(np.int64(src.to(torch.int64).sum().item())))
+    else:
+        tot = src.to(torch.float64).sum().item()
+        assert abs(got[-1].item() - tot) <= 1e-5 * tot
+
+
+def test_lmosem_10_7_sampled(ctx):
+    N, nev = 150, 10_000_000
+    events = I.lmosem_events(I.SEED_LMOSEM, nev, N)
+    evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
+    ctx.set_option("map_unroll", 1)
+    lm = S.Map(ctx, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
+    ctx.set_option("map_unroll", 4)
+    addf = S.Reduce(ctx, A.ADD, S.F32)
+    f0 = np.ones(N ** 3, np.float32)
+    f = S.Vector.from_numpy(ctx, f0).set_distribution(S.COPY)
+    # full-size run (the bench's step) must complete and conserve the invariant
+    ev = S.Vector(ctx, evd, nev).set_distribution(S.BLOCK)
+    ev.copy_in(events)
+    c = S.Vector(ctx, S.F32, N ** 3).set_distribution(S.COPY, 0, addf)
+    c.fill(0.0)
+    lm(ev, f, (c, S.WRITE))
+    c.set_distribution(S.BLOCK)
+    cf = c.to_numpy().astype(np.float64)
+    # sample parity against the oracle (1/50 of the events)
+    sub = events[::50].copy()
+    evs = S.Vector(ctx, evd, sub.shape[0]).set_distribution(S.BLOCK)
+    evs.copy_in(sub)
+    c2 = S.Vector(ctx, S.F32, N ** 3).set_distribution(S.COPY, 0, addf)
+    c2.fill(0.0)
+    lm(evs, f, (c2, S.WRITE))
+    c2.set_distribution(S.BLOCK)
+    c_ref, _, nhit_s, _ = O.lmosem(sub, N, f0)
+    assert rel_l2(c2.to_numpy(), c_ref) <= 1e-4
+    # full run: sum f*c equals the number of events that hit (oracle count on the sample x 50 ~)
+    assert abs(cf.sum() / (nhit_s * 50) - 1.0) < 0.01
