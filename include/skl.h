@@ -207,6 +207,12 @@ skl_status skl_mapoverlap_create(skl_ctx* ctx, const char* src, const char* entr
                                  skl_type out, int d, int boundary, const void* neutral,
                                  skl_skel** sk);
 skl_status skl_skel_destroy(skl_skel* sk);
+/* MapOverlap: *proven = 1 if every get() offset in the customising function was
+ * proven within [-d, d] at creation (literal offsets, or counted for-loops with
+ * literal bounds as in Listing 1.2) - the static check the paper names as future
+ * work; 0 if not provable (a provable violation already made
+ * skl_mapoverlap_create fail with SKL_ERR_OUT_OF_RANGE).                     */
+skl_status skl_mapoverlap_bounds(skl_skel* sk, int* proven);
 
 /* One extra argument at run time.                                             */
 #define SKL_ARG_SCALAR 1

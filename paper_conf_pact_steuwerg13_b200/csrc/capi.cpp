@@ -411,6 +411,13 @@ skl_status skl_mapoverlap_create(skl_ctx* ctx, const char* src, const char* entr
     *sk = wrap(skel_create(C(ctx), K_MAPOVERLAP, src, entry, in, 0, out, nullptr, 0, d, boundary, neutral));
   });
 }
+skl_status skl_mapoverlap_bounds(skl_skel* sk, int* proven) {
+  return guard([&] {
+    Skel* s = S(sk);
+    if (s->kind != K_MAPOVERLAP || !proven) fail(SKL_ERR_INVALID_ARG, "not a MapOverlap skeleton / NULL out");
+    *proven = s->bounds == 1;
+  });
+}
 skl_status skl_skel_destroy(skl_skel* sk) {
   return guard([&] {
     Skel* s = S(sk);

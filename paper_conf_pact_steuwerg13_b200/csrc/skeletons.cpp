@@ -146,6 +146,18 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       if (16 % si != 0) fail(SKL_ERR_TYPE, "MapOverlap element size must divide 16 bytes");
       if (d < 0) fail(SKL_ERR_INVALID_ARG, "negative overlap size");
       if (boundary != SKL_NEUTRAL && boundary != SKL_NEAREST) fail(SKL_ERR_INVALID_ARG, "bad boundary mode");
+      {
+        // static get() bounds (P:L366-368 future work): reject provable violations
+        // now; proven functions need no runtime check even in debug mode
+        std::string why;
+        s->bounds = check_get_bounds(s->user_src, d, &why);
+        if (s->bounds < 0) fail(SKL_ERR_OUT_OF_RANGE, "static get() check (P:L362-368): " + why);
+        if (s->bounds == 1 && ctx->debug_bounds) {
+          const std::string on = "#define SKL_DEBUG_BOUNDS 1\n", off = "#define SKL_DEBUG_BOUNDS 0\n";
+          const size_t at = defs.find(on);
+          if (at != std::string::npos) defs.replace(at, on.size(), off);
+        }
+      }
       s->neutral.assign(si, 0);
       if (neutral) std::memcpy(s->neutral.data(), neutral, si);
       const int epc = (int)(16 / si);

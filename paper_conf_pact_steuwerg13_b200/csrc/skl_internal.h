@@ -247,6 +247,7 @@ struct Skel {
   int scan_sub = 4;  // Scan: tiles per look-back chunk (vector path)
   int scan_variant = 0;
   int scan_fstride = 16;  // Scan: status word spacing in 8-byte units
+  int bounds = 0;         // MapOverlap: 1 = get() offsets statically proven within d
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
   std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
@@ -265,6 +266,8 @@ void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int n
 void* device_alloc(Ctx* ctx, int g, size_t bytes);
 void device_free(Ctx* ctx, int g, void* p);
 void check_debug_flag(Ctx* ctx);
+// bounds.cpp: 1 proven, 0 unknown, -1 violation (reason in *why)
+int check_get_bounds(const std::string& src, int d, std::string* why);
 
 }  // namespace skl
 

@@ -89,6 +89,7 @@ def lib():
         "skl_reduce_run": [vp, vp, pp], "skl_scan_run": [vp, vp, pp], "skl_mapoverlap_run": [vp, vp, pp],
         "skl_scalar_get": [vp, vp, sz],
         "skl_skel_cubin": [vp, vp, sz, C.POINTER(sz)], "skl_skel_source": [vp, C.c_char_p, sz, C.POINTER(sz)],
+        "skl_mapoverlap_bounds": [vp, C.POINTER(i)],
         "skl_capture_begin": [vp], "skl_capture_end": [vp, pp], "skl_graph_launch": [vp],
         "skl_graph_destroy": [vp],
         "skl_plan_range": [sz, i, i, i, i, i, C.POINTER(sz), C.POINTER(sz)],
@@ -510,6 +511,13 @@ class MapOverlap(Skeleton):
         o = C.c_void_p(out.handle.value if out is not None else None)
         check(lib().skl_mapoverlap_run(self._h, inp.handle, C.byref(o)))
         return out if out is not None else _wrap_out(self.ctx, o, self.tout)
+
+    @property
+    def bounds_proven(self) -> bool:
+        """get() offsets statically proven within [-d, d]."""
+        v = C.c_int()
+        check(lib().skl_mapoverlap_bounds(self._h, C.byref(v)))
+        return bool(v.value)
 
 
 # ---------------------------------------------------------------- host-only planning

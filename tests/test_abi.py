@@ -171,3 +171,29 @@ def test_planned_redistribution_is_exact(lib, fk, fa, tk, ta, units, G):
     if (fk == S.SINGLE and fa >= G) or (tk == S.SINGLE and ta >= G):
         pytest.skip()
     _simulate(units, G, fk, fa, tk, ta)
+
+
+# ------------------------------------------------------------------ static get() bounds
+def test_static_get_bounds(offline):
+    c = offline
+    # Listing 1.2 (counted loops), Listing 1.5 (literals), the 5x5 Gaussian: proven
+    assert S.MapOverlap(c, A.BOX3, S.F32, S.F32, 1).bounds_proven
+    assert S.MapOverlap(c, A.SOBEL, S.U8, S.U8, 1).bounds_proven
+    assert S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST).bounds_proven
+    assert S.MapOverlap(c, A.BOX1D, S.F32, S.F32, 1).bounds_proven
+    # provable violations are rejected at creation, before any kernel runs
+    for src, d in (("float f(const float* p){ return get(p, 2, 0); }", 1),
+                   ("float f(const float* p){ return get(p, 0, -3); }", 2),
+                   ("float f(float* m){ float s=0; for (int i = -2; i <= 2; ++i) s += get(m, i, 0); return s; }", 1),
+                   ("float f(float* m){ float s=0; for (int j = 0; j <= 3; j++) s += get(m, 0, j); return s; }", 2)):
+        with pytest.raises(S.SklError) as e:
+            S.MapOverlap(c, src, S.F32, S.F32, d)
+        assert e.value.name == "OUT_OF_RANGE"
+    # the same loops within d are proven; a runtime offset is not provable
+    assert S.MapOverlap(c, "float f(float* m){ float s=0; for (int j = 0; j < 3; j++) s += get(m, 0, j); return s; }",
+                        S.F32, S.F32, 2).bounds_proven
+    assert not S.MapOverlap(c, "float f(const float* p){ int k = 1; return get(p, k, 0); }",
+                            S.F32, S.F32, 1).bounds_proven
+    # comments do not count
+    assert S.MapOverlap(c, "float f(const float* p){ /* get(p, 9, 9) */ return get(p, 1, 1); }",
+                        S.F32, S.F32, 1).bounds_proven

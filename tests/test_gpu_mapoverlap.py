@@ -106,7 +106,10 @@ def test_debug_bounds_flags_access_beyond_d():
     require_gpu()
     with S.Context(1) as c:
         c.set_option("debug_bounds", 1)
-        bad = S.MapOverlap(c, "float f(const float* p){ return get(p, 2, 0); }", S.F32, S.F32, 1)
+        # an offset the static check cannot prove (a runtime value) -> runtime check
+        bad = S.MapOverlap(c, "float f(const float* p){ int k = (int)(p[0] * 0.0f) + 2; return get(p, k, 0); }",
+                           S.F32, S.F32, 1)
+        assert not bad.bounds_proven
         with pytest.raises(S.SklError) as e:
             bad(S.Matrix.from_numpy(c, np.ones((8, 8), np.float32)))
         assert e.value.name == "OUT_OF_RANGE"
