@@ -89,10 +89,9 @@ def lmosem():
 
 def scan():
     n = 1 << 30
-    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 3), (3, 1, 256, 8, 16, 4), (3, 1, 256, 8, 8, 3),
-                                      (3, 1, 256, 8, 16, 2), (3, 1, 384, 8, 16, 2), (3, 1, 192, 8, 16, 4),
-                                      (3, 1, 256, 6, 16, 4) if False else (3, 1, 128, 8, 16, 8),
-                                      (2, 1, 256, 8, 16, 3), (1, 1, 256, 8, 16, 3)):
+    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 4), (3, 1, 128, 8, 16, 8), (3, 1, 128, 8, 16, 10),
+                                      (3, 1, 128, 8, 16, 12), (3, 1, 192, 8, 16, 6), (3, 1, 256, 8, 16, 5),
+                                      (2, 1, 128, 8, 16, 8), (3, 1, 64, 8, 16, 16)):
         if True:
             if True:
                 c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_sub": pers,
