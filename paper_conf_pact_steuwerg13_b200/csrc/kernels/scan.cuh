@@ -111,7 +111,7 @@ __device__ __forceinline__ unsigned skl_status(const unsigned* flags, const SKL_
 __device__ __forceinline__ void skl_lookback_block(unsigned tile, unsigned* flags, SKL_T* aggs,
                                                    SKL_T* incls, unsigned epoch, const SKL_T* carry,
                                                    int ncarry, const SKL_T* s_agg, SKL_T* s_excl,
-                                                   int* s_has) {
+                                                   int* s_has, bool publish_agg = true) {
   SklOp op;
   const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
   __shared__ int s_p;
@@ -133,7 +133,7 @@ __device__ __forceinline__ void skl_lookback_block(unsigned tile, unsigned* flag
     }
     return;
   }
-  if (tid == 0) skl_publish(flags, aggs, incls, tile, epoch, 1u, *s_agg);
+  if (tid == 0 && publish_agg) skl_publish(flags, aggs, incls, tile, epoch, 1u, *s_agg);
   bool have = false;  // thread 0 only
   long base = (long)tile - 1;
   while (true) {
@@ -395,6 +395,128 @@ __device__ __forceinline__ void skl_warp_range_fold(const SKL_T* __restrict__ in
       has = true;
     }
   }
+}
+
+// ---- persistent, 3-stage software pipeline (SKL_SCAN_VARIANT 4) -------------
+// Block b owns tiles t_k = b + k * grid.  Iteration k:
+//   issue the load of t_{k+2} (cp.async, stage (k+2) % 3)
+//   look back for t_k            (its aggregate was published one iteration ago,
+//                                 so predecessors in the same round are ready)
+//   apply the tile prefix to t_k's locally scanned values, stream them out
+//   local scan of t_{k+1} (landed meanwhile), publish its aggregate
+// so the look-back latency overlaps loads already in flight instead of stalling
+// the memory pipeline (the per-tile kernel's top stalls were barriers and the
+// look-back spin; the same tile pipeline without look-back runs at copy speed).
+#ifndef SKL_MINB_P
+#define SKL_MINB_P 1
+#endif
+__device__ __forceinline__ int skl_nvalid(skl_u64 n, unsigned t) {
+  const skl_u64 tlo = (skl_u64)t * SKL_TILE;
+  return n - tlo >= (skl_u64)SKL_TILE ? SKL_TILE : (int)(n - tlo);
+}
+
+// local (within-tile) inclusive scan of the tile in stage sm, written back in
+// place; returns the tile aggregate (all threads)
+__device__ __forceinline__ SKL_T skl_tile_local(uint4* sm, int nvalid) {
+  SklChunk<SKL_T, SKL_ITEMS> my;
+#pragma unroll
+  for (int q = 0; q < SKL_CH; ++q) my.q[q] = sm[skl_swz(threadIdx.x * SKL_CH + q)];
+  SKL_T items[SKL_ITEMS];
+#pragma unroll
+  for (int q = 0; q < SKL_ITEMS; ++q) items[q] = my.e[q];
+  const int first = threadIdx.x * SKL_ITEMS;
+  const int cnt = nvalid - first >= SKL_ITEMS ? SKL_ITEMS : (nvalid - first > 0 ? nvalid - first : 0);
+  const int nthr = (nvalid + SKL_ITEMS - 1) / SKL_ITEMS;
+  SKL_T agg;
+  skl_scan_tile<SKL_ITEMS, false>(items, cnt, nthr, 0, nullptr, nullptr, nullptr, 0, nullptr, 0, false,
+                                  nullptr, &agg);
+#pragma unroll
+  for (int q = 0; q < SKL_ITEMS; ++q) my.e[q] = items[q];
+#pragma unroll
+  for (int q = 0; q < SKL_CH; ++q) sm[skl_swz(threadIdx.x * SKL_CH + q)] = my.q[q];
+  return agg;
+}
+
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MINB_P)
+skl_scan_pipe(const SKL_T* __restrict__ in, SKL_T* __restrict__ out, skl_u64 n, unsigned* flags,
+              SKL_T* aggs, SKL_T* incls, unsigned epoch, const SKL_T* carry, int ncarry) {
+  extern __shared__ uint4 skl_dyn[];
+  __shared__ SKL_T p_agg[3];
+  __shared__ SKL_T p_excl;
+  __shared__ int p_has;
+  SklOp op;
+  const unsigned ntiles = (unsigned)((n + SKL_TILE - 1) / SKL_TILE);
+  const unsigned G = gridDim.x;
+  const unsigned t0 = blockIdx.x;
+  if (t0 >= ntiles) return;
+#define SKL_STAGE(k) (skl_dyn + ((k) % 3u) * (SKL_BLOCK * SKL_CH))
+  skl_scan_issue(in, (skl_u64)t0 * SKL_TILE, skl_nvalid(n, t0), SKL_STAGE(0u));
+  skl_cp_commit();
+  if (t0 + G < ntiles) skl_scan_issue(in, (skl_u64)(t0 + G) * SKL_TILE, skl_nvalid(n, t0 + G), SKL_STAGE(1u));
+  skl_cp_commit();
+  skl_cp_wait1();
+  __syncthreads();
+  {
+    const SKL_T agg = skl_tile_local(SKL_STAGE(0u), skl_nvalid(n, t0));
+    if (threadIdx.x == 0) {
+      p_agg[0] = agg;
+      if (t0 != 0) skl_publish(flags, aggs, incls, t0, epoch, 1u, agg);  // tile 0 publishes P
+    }
+  }
+  __syncthreads();
+  for (unsigned k = 0;; ++k) {
+    const unsigned t = t0 + k * G;
+    if (t >= ntiles) break;
+    const unsigned t1 = t + G, t2 = t + 2 * G;
+    if (t2 < ntiles) skl_scan_issue(in, (skl_u64)t2 * SKL_TILE, skl_nvalid(n, t2), SKL_STAGE(k + 2));
+    skl_cp_commit();
+    // ---- look-back for t (aggregate already public)
+#if SKL_SCAN_VARIANT == 5
+    if (threadIdx.x == 0) p_has = 0;  // measurement only: no look-back
+#else
+    skl_lookback_block(t, flags, aggs, incls, epoch, carry, ncarry, &p_agg[k % 3], &p_excl, &p_has, false);
+#endif
+    __syncthreads();
+    // ---- apply the tile prefix, stream out
+    {
+      uint4* sm = SKL_STAGE(k);
+      const int nvalid = skl_nvalid(n, t);
+      const bool has = p_has != 0;
+      const SKL_T pre = p_excl;
+      const skl_u64 tlo = (skl_u64)t * SKL_TILE;
+      char* gout = (char*)(out + tlo);
+      if (nvalid == SKL_TILE) {
+#pragma unroll
+        for (int i = 0; i < SKL_CH; ++i) {
+          const unsigned c = i * SKL_BLOCK + threadIdx.x;
+          SklChunk<SKL_T, SKL_EPC> ch;
+          ch.q[0] = sm[skl_swz(c)];
+          if (has) {
+#pragma unroll
+            for (int e = 0; e < SKL_EPC; ++e) ch.e[e] = op(pre, ch.e[e]);
+          }
+          skl_st16(gout + 16 * (skl_u64)c, ch.q[0]);
+        }
+      } else {
+        for (int e = threadIdx.x; e < nvalid; e += SKL_BLOCK) {
+          SKL_T v = *((const SKL_T*)&sm[skl_swz(e / SKL_EPC)] + (e % SKL_EPC));
+          out[tlo + e] = has ? op(pre, v) : v;
+        }
+      }
+    }
+    // ---- local scan of t1 (landed while this tile looked back)
+    if (t1 < ntiles) {
+      skl_cp_wait1();
+      __syncthreads();  // t1 visible; every thread is past this tile's apply
+      const SKL_T agg = skl_tile_local(SKL_STAGE(k + 1), skl_nvalid(n, t1));
+      if (threadIdx.x == 0) {
+        p_agg[(k + 1) % 3] = agg;
+        skl_publish(flags, aggs, incls, t1, epoch, 1u, agg);
+      }
+    }
+    __syncthreads();  // stage k is refilled by the next iteration's prefetch
+  }
+#undef SKL_STAGE
 }
 
 // One block per tile (tile = blockIdx.x; blocks start in index order), tile

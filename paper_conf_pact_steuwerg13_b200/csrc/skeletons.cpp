@@ -134,6 +134,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
         defs += "#define SKL_FSTRIDE " + std::to_string(s->scan_fstride) + "\n";
         defs += "#define SKL_SPIN_NS " + std::to_string(ctx->scan_spin_ns) + "\n";
         defs += "#define SKL_MINB " + std::to_string(ctx->scan_minb) + "\n";
+        defs += "#define SKL_MINB_P " + std::to_string(ctx->scan_minb_pipe) + "\n";
         defs += "#define SKL_SUB " + std::to_string(s->scan_sub) + "\n";
       }
       body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +
@@ -675,7 +676,13 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
     const void* cptr = carry ? totals[g] : nullptr;
     int ncarry = carry ? i : 0;
     void* args[] = {(void*)&pin, &pout, &nn, &flags, &aggs, &incls, &ep, (void*)&cptr, &ncarry};
-    if (vec && per_tile) {
+    if (vec && per_tile && s->scan_variant >= 4) {
+      // persistent 3-stage pipeline: one wave of resident blocks
+      const size_t smem = 3 * (size_t)s->block * (size_t)s->scan_ch * 16;
+      const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_scan_pipe", s->block, smem));
+      const size_t grid = std::min(ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
+      launch(ctx, g, s->prog, "skl_scan_pipe", dim3((unsigned)grid), dim3(s->block), smem, args);
+    } else if (vec && per_tile) {
       const size_t smem = (size_t)s->block * (size_t)s->scan_ch * 16;
       launch(ctx, g, s->prog, "skl_scan_pt", dim3((unsigned)ntiles), dim3(s->block), smem, args);
     } else if (vec) {

@@ -89,20 +89,29 @@ def lmosem():
 
 def scan():
     n = 1 << 30
-    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 4), (3, 1, 128, 8, 16, 8), (3, 1, 128, 8, 16, 10),
-                                      (3, 1, 128, 8, 16, 12), (3, 1, 192, 8, 16, 6), (3, 1, 256, 8, 16, 5),
-                                      (2, 1, 128, 8, 16, 8), (3, 1, 64, 8, 16, 16)):
+    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 4), (5, 1, 256, 8, 16, 2), (4, 1, 256, 8, 16, 2),
+                                      (4, 1, 256, 8, 16, 1), (4, 1, 128, 8, 16, 4), (4, 1, 512, 4, 16, 1),
+                                      (4, 1, 256, 4, 16, 3), (4, 1, 512, 8, 16, 1)):
         if True:
             if True:
                 c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_sub": pers,
-                              "scan_variant": var, "scan_fstride": fs, "scan_minb": ns})
+                              "scan_variant": var, "scan_fstride": fs, "scan_minb": 4,
+                              "scan_minb_pipe": ns})
                 sc = S.Scan(c, A.ADD_I32, S.I32)
                 v = S.Vector(c, S.I32, n).set_distribution(S.BLOCK).fill(1)
                 o = sc(v)
                 ms = timeit(lambda: sc(v, out=o), reps=5)
                 p, f, cnt = o.local_part(0)
-                print(f"scan i32 variant={var} sub={pers} block={bt} chunks={ch} fstride={fs} spin={ns}: {ms:.3f} ms  "
-                      f"{8 * n / (ms / 1e3) / 1e9:.0f} GB/s", flush=True)
+
+                class View:
+                    __cuda_array_interface__ = {"shape": (cnt,), "typestr": "<i4", "data": (p, False),
+                                                "version": 3, "strides": None}
+                c.sync()
+                got = torch.as_tensor(View(), device="cuda")
+                idx = torch.tensor([0, 1, 8191, 8192, 123456789, n // 2, n - 2, n - 1], device="cuda")
+                ok = bool(torch.equal(got[idx].long(), idx + 1))   # scan of ones = 1..n
+                print(f"scan i32 variant={var} sub={pers} block={bt} chunks={ch} fstride={fs} minb={ns}: {ms:.3f} ms  "
+                      f"{8 * n / (ms / 1e3) / 1e9:.0f} GB/s ok={ok}", flush=True)
                 c.finalize()
 
 
