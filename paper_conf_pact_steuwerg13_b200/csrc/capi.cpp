@@ -176,6 +176,9 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "scan_spin_ns") {
       if (value < 0 || value > 100000) fail(SKL_ERR_INVALID_ARG, "scan_spin_ns in [0,100000]");
       c->scan_spin_ns = (int)value;
+    } else if (k == "scan_lbw") {
+      if (value < 1 || value > 8) fail(SKL_ERR_INVALID_ARG, "scan_lbw in [1,8]");
+      c->scan_lbw = (int)value;
     } else if (k == "scan_minb_pipe") {
       if (value < 1 || value > 8) fail(SKL_ERR_INVALID_ARG, "scan_minb_pipe in [1,8]");
       c->scan_minb_pipe = (int)value;

@@ -57,7 +57,24 @@ __device__ __forceinline__ unsigned skl_ld_relaxed32(const unsigned* p) {
 #define SKL_SPIN_NS 0
 #endif
 
+#ifndef SKL_LBW
+#define SKL_LBW 3
+#endif
+
 #if SKL_PACKED
+// one look at tile j's status: 0 if not published yet, else state (*v = value)
+__device__ __forceinline__ unsigned skl_status_try(const unsigned* flags, const SKL_T* aggs,
+                                                   const SKL_T* incls, long j, unsigned epoch, SKL_T* v) {
+  const unsigned long long w = skl_ld_relaxed64((const unsigned long long*)flags + (skl_u64)j * SKL_FSTRIDE);
+  const unsigned st = ((unsigned)w >> 2) == epoch ? ((unsigned)w & 3u) : 0u;
+  if (st) {
+    const unsigned bits = (unsigned)(w >> 32);
+    memcpy(v, &bits, sizeof(SKL_T));
+  }
+  (void)aggs;
+  (void)incls;
+  return st;
+}
 __device__ __forceinline__ void skl_publish(unsigned* flags, SKL_T* aggs, SKL_T* incls, unsigned tile,
                                             unsigned epoch, unsigned state, const SKL_T& v) {
   unsigned bits = 0;
@@ -84,6 +101,16 @@ __device__ __forceinline__ unsigned skl_status(const unsigned* flags, const SKL_
   return st;
 }
 #else
+__device__ __forceinline__ unsigned skl_status_try(const unsigned* flags, const SKL_T* aggs,
+                                                   const SKL_T* incls, long j, unsigned epoch, SKL_T* v) {
+  const unsigned f = skl_ld_relaxed32(&flags[(skl_u64)j * 2 * SKL_FSTRIDE]);
+  const unsigned st = (f >> 2) == epoch ? (f & 3u) : 0u;
+  if (st) {
+    __threadfence();  // acquire
+    *v = st == 2u ? skl_ldcg(incls + j) : skl_ldcg(aggs + j);
+  }
+  return st;
+}
 __device__ __forceinline__ void skl_publish(unsigned* flags, SKL_T* aggs, SKL_T* incls, unsigned tile,
                                             unsigned epoch, unsigned state, const SKL_T& v) {
   if (state == 1u) aggs[tile] = v;
@@ -136,17 +163,48 @@ __device__ __forceinline__ void skl_lookback_block(unsigned tile, unsigned* flag
   if (tid == 0 && publish_agg) skl_publish(flags, aggs, incls, tile, epoch, 1u, *s_agg);
   bool have = false;  // thread 0 only
   long base = (long)tile - 1;
+  // each thread watches SKL_LBW consecutive predecessors (distances tid*W ..
+  // tid*W + W-1), their loads issued together: one round trip covers
+  // SKL_BLOCK x SKL_LBW tiles (>= the tiles in flight, so usually one round)
+  constexpr int W = SKL_LBW;
   while (true) {
-    const long j = base - tid;
+    SKL_T val[W];
+    unsigned st[W];
+#pragma unroll
+    for (int r = 0; r < W; ++r) st[r] = 0u;
+    for (bool pending = true; pending;) {
+      pending = false;
+#pragma unroll
+      for (int r = 0; r < W; ++r) {
+        const long j = base - (long)(tid * W + r);
+        if (j >= 0 && st[r] == 0u) {
+          st[r] = skl_status_try(flags, aggs, incls, j, epoch, &val[r]);
+          pending |= st[r] == 0u;
+        }
+      }
+    }
+    int myp = W * SKL_BLOCK;
+#pragma unroll
+    for (int r = W - 1; r >= 0; --r)
+      if (st[r] == 2u) myp = tid * W + r;  // nearest prefix among mine
+    if (tid == 0) s_p = W * SKL_BLOCK;
+    __syncthreads();
+    if (myp < W * SKL_BLOCK) atomicMin(&s_p, myp);
+    __syncthreads();
+    const int pfound = s_p;  // distance of the nearest inclusive prefix
+    const int plim = pfound < W * SKL_BLOCK ? pfound : W * SKL_BLOCK - 1;
+    // thread-local fold of my distances <= plim, the larger distance on the left
     SKL_T v;
-    unsigned st = 0;
-    if (j >= 0) st = skl_status(flags, aggs, incls, j, epoch, &v);
-    if (tid == 0) s_p = SKL_BLOCK;
-    __syncthreads();
-    if (st == 2u) atomicMin(&s_p, tid);
-    __syncthreads();
-    const int pfound = s_p;
-    const int p = pfound < SKL_BLOCK ? pfound : SKL_BLOCK - 1;  // threads 0..p contribute
+    bool hv = false;
+#pragma unroll
+    for (int r = W - 1; r >= 0; --r) {
+      const int dist = tid * W + r;
+      if (dist <= plim && base - (long)dist >= 0) {
+        v = hv ? op(v, val[r]) : val[r];
+        hv = true;
+      }
+    }
+    const int p = plim / W;  // threads 0..p contribute
     // fold threads p..0 (a higher thread is an earlier tile: the left operand)
     const int wp = p - warp * 32;  // last contributing lane of this warp
 #pragma unroll
@@ -162,8 +220,8 @@ __device__ __forceinline__ void skl_lookback_block(unsigned tile, unsigned* flag
       s_acc = have ? op(w, s_acc) : w;
       have = true;
     }
-    if (pfound < SKL_BLOCK) break;
-    base -= SKL_BLOCK;
+    if (pfound < W * SKL_BLOCK) break;
+    base -= W * SKL_BLOCK;
     __syncthreads();  // s_p / s_wv are reused by the next round
   }
   if (tid == 0) {

@@ -135,6 +135,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
         defs += "#define SKL_SPIN_NS " + std::to_string(ctx->scan_spin_ns) + "\n";
         defs += "#define SKL_MINB " + std::to_string(ctx->scan_minb) + "\n";
         defs += "#define SKL_MINB_P " + std::to_string(ctx->scan_minb_pipe) + "\n";
+        defs += "#define SKL_LBW " + std::to_string(ctx->scan_lbw) + "\n";
         defs += "#define SKL_SUB " + std::to_string(s->scan_sub) + "\n";
       }
       body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +

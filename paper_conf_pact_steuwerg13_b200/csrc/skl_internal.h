@@ -117,6 +117,7 @@ struct Ctx {
   int scan_spin_ns = 0;        // Scan look-back spin back-off (__nanosleep)
   int scan_minb = 4;           // Scan per-tile kernel: min resident blocks (launch bounds)
   int scan_minb_pipe = 2;      // Scan pipelined kernel: min resident blocks
+  int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest

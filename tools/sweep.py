@@ -89,14 +89,14 @@ def lmosem():
 
 def scan():
     n = 1 << 30
-    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 4), (5, 1, 256, 8, 16, 2), (4, 1, 256, 8, 16, 2),
-                                      (4, 1, 256, 8, 16, 1), (4, 1, 128, 8, 16, 4), (4, 1, 512, 4, 16, 1),
-                                      (4, 1, 256, 4, 16, 3), (4, 1, 512, 8, 16, 1)):
+    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 1), (3, 1, 256, 8, 16, 2), (3, 1, 256, 8, 16, 3),
+                                      (3, 1, 256, 8, 16, 4), (3, 1, 256, 8, 16, 6), (4, 1, 256, 8, 16, 3),
+                                      (3, 1, 128, 8, 16, 6)):
         if True:
             if True:
                 c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_sub": pers,
-                              "scan_variant": var, "scan_fstride": fs, "scan_minb": 4,
-                              "scan_minb_pipe": ns})
+                              "scan_variant": var, "scan_fstride": fs, "scan_minb": 4 if bt == 256 else 8,
+                              "scan_lbw": ns})
                 sc = S.Scan(c, A.ADD_I32, S.I32)
                 v = S.Vector(c, S.I32, n).set_distribution(S.BLOCK).fill(1)
                 o = sc(v)
