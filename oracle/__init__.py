@@ -190,6 +190,23 @@ def gauss5_weights() -> np.ndarray:
     return w.reshape(5, 5)
 
 
+AP_MANHATTAN, AP_DOT, AP_DOT_F64 = 0, 1, 2
+
+
+def allpairs(fn: int, a: np.ndarray, b: np.ndarray) -> np.ndarray:
+    """C[i][j] = A_i (+) B_j; rows of a (n x d) and b (m x d)."""
+    a = np.ascontiguousarray(a, dtype=np.float32)
+    b = np.ascontiguousarray(b, dtype=np.float32)
+    n, d = a.shape
+    m = b.shape[0]
+    c = np.empty((n, m), dtype=np.float64 if fn == AP_DOT_F64 else np.float32)
+    L = lib()
+    L.oracle_allpairs.argtypes = [C.c_int, C.c_void_p, C.c_void_p, C.c_void_p, C.c_size_t, C.c_size_t, C.c_size_t]
+    L.oracle_allpairs.restype = C.c_int
+    assert L.oracle_allpairs(fn, _p(a), _p(b), _p(c), n, m, d) == 0
+    return c
+
+
 def block_range(n: int, G: int, g: int):
     lo, hi = C.c_size_t(), C.c_size_t()
     lib().oracle_block_range(n, G, g, C.byref(lo), C.byref(hi))

@@ -97,6 +97,18 @@ int oracle_mapoverlap1d(int stencil, const float* in, float* out, size_t n, int 
 /* The 25 Gaussian weights the oracle uses, row-major [dy+2][dx+2]. */
 void oracle_gauss5_weights(float* w25);
 
+/* ---- Allpairs ----------------------------------------------- */
+/* C[i][j] = A_i (+) B_j for rows A_i of the n x d matrix A and B_j of the m x d
+ * matrix B.  The row function is a zip followed by a
+ * left fold (reading A36): acc = z(a_0, b_0); acc = acc (+) z(a_k, b_k), k = 1..d-1
+ *   AP_MANHATTAN  z = |a - b|, (+) = +   (the pairwise Manhattan distance)
+ *   AP_DOT        z = a * b,   (+) = +   (dotProduct, Eq. (1))
+ * in fp32 with every operation rounded (-ffp-contract=off); AP_DOT_F64 is the
+ * same dot product accumulated in double (for the Eq. (2) pin A x B = allpairs(
+ * dotProduct)(A, B^T)).  C is float (double for AP_DOT_F64).                   */
+enum oracle_allpairs_fn { AP_MANHATTAN = 0, AP_DOT = 1, AP_DOT_F64 = 2 };
+int oracle_allpairs(int fn, const float* A, const float* B, void* C, size_t n, size_t m, size_t d);
+
 /* ---- Distributions (A1-A6, A25) ----------------------------- */
 /* block: chunk = ceil(n/G); part g = [g*chunk, min((g+1)*chunk, n)) (A1)      */
 void oracle_block_range(size_t n, int G, int g, size_t* lo, size_t* hi);

@@ -308,6 +308,30 @@ def test_mapoverlap1d_pins():
     assert np.array_equal(O.mapoverlap1d(O.OS_BOX3, v, 1, O.OB_NEUTRAL, 0.0), m[0])
 
 
+# ------------------------------------------------------------------ Allpairs
+def test_golden_allpairs():
+    g = read_golden("allpairs_small.txt")
+    a, b = np.array(g["A"], np.float32), np.array(g["B"], np.float32)
+    assert np.array_equal(O.allpairs(O.AP_DOT, a, b), np.array(g["dot"], np.float32))
+    assert np.array_equal(O.allpairs(O.AP_MANHATTAN, a, b), np.array(g["manhattan"], np.float32))
+
+
+def test_allpairs_eq2_matrix_multiply_and_cityblock():
+    from scipy.spatial.distance import cdist
+    a = I.uniform_f32(71, 37 * 19).reshape(37, 19) - np.float32(0.5)
+    bt = I.uniform_f32(72, 19 * 23).reshape(19, 23) - np.float32(0.5)   # B is d x m
+    # Eq. (2): A x B = allpairs(dotProduct)(A, B^T)
+    c64 = O.allpairs(O.AP_DOT_F64, a, np.ascontiguousarray(bt.T))
+    assert np.allclose(c64, a.astype(np.float64) @ bt.astype(np.float64), rtol=1e-12, atol=1e-12)
+    c32 = O.allpairs(O.AP_DOT, a, np.ascontiguousarray(bt.T))
+    assert np.allclose(c32, c64, rtol=0, atol=19 * 2e-7)
+    b = I.uniform_f32(73, 23 * 19).reshape(23, 19)
+    man = O.allpairs(O.AP_MANHATTAN, a, b)
+    assert np.allclose(man, cdist(a.astype(np.float64), b.astype(np.float64), "cityblock"), rtol=1e-6)
+    # the fold is left to right in fp32: first column of a 1-column problem is |a-b|
+    assert np.array_equal(O.allpairs(O.AP_MANHATTAN, a[:, :1], b[:, :1]), np.abs(a[:, :1] - b[:, :1].T))
+
+
 # ------------------------------------------------------------------ Distributions
 def test_golden_block_partition():
     for row in read_golden("block_partition.txt")[None]:
