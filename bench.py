@@ -470,6 +470,41 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         out.destroy()
         torch.cuda.empty_cache()
 
+    if "allpairs" in which:
+        # Allpairs: zip-reduce rows on the FP32 pipes
+        import torch as _t
+        for name, zsrc, nn, mm, dd, ops in (("allpairs_dot_4096", A.MULT, 4096, 4096, 4096, 2),
+                                             ("allpairs_manhattan_4096x4096x128", A.ABSDIFF, 4096, 4096, 128, 2)):
+            a = I.uniform_f32(81, nn * dd).reshape(nn, dd)
+            b = I.uniform_f32(82, mm * dd).reshape(mm, dd)
+            ap = S.Allpairs(ctx, zsrc, S.F32, S.F32, reduce=A.ADD)
+            ma = S.Matrix.from_numpy(ctx, a).set_distribution(S.BLOCK)
+            mb = S.Matrix.from_numpy(ctx, b).set_distribution(S.COPY)
+            c = ap(ma, mb)
+
+            def step(_):
+                ap(ma, mb, out=c)
+
+            ms, _ = timer.run(step, max(3, K // 2), 2, D)
+            ms = D.max(ms)
+            # parity on a 32 x 32 corner + a strip (oracle, same fold order: bit-exact)
+            cg = c.to_numpy()
+            fn = O.AP_DOT if zsrc == A.MULT else O.AP_MANHATTAN
+            ok = np.array_equal(cg[:32, :32], O.allpairs(fn, a[:32], b[:32])) and np.array_equal(
+                cg[nn - 7:, mm - 40:], O.allpairs(fn, a[nn - 7:], b[mm - 40:]))
+            flops = float(ops) * nn * mm * dd
+            sms = _t.cuda.get_device_properties(D.local).multi_processor_count
+            peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
+            res[name] = {"workload": f"allpairs zip-reduce {'dotProduct (Eq. 2 matrix multiply)' if zsrc == A.MULT else 'Manhattan distance'} "
+                                     f"{nn}x{mm}, d={dd}, block(A) x copy(B)",
+                         "ms": round(ms, 4), "pairs_per_s": nn * mm / (ms / 1e3),
+                         "roofline": {"bound": "alu", "achieved": flops / (ms / 1e3) / 1e12, "peak": peak / 1e12,
+                                      "unit": "TFLOP/s", "frac": flops / (ms / 1e3) / peak,
+                                      "note": f"{ops} fp32 ops per (i,j,k), no FMA (-fmad=false)"},
+                         "check": "ok" if ok else "FAIL"}
+            for x in (ma, mb, c):
+                x.destroy()
+
     if "lmosem" in which:
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
@@ -571,7 +606,7 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, D, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "sobel", "gauss", "scan_i32", "scan_f32", "lmosem"] if args.skeletons == "all"
+        ["dot", "sobel", "gauss", "scan_i32", "scan_f32", "lmosem", "allpairs"] if args.skeletons == "all"
         else args.skeletons.split(","))
     sk = bench_skeletons(args, D, P, which) if which else {}
     if D.rank != 0:

@@ -214,6 +214,23 @@ skl_status skl_skel_destroy(skl_skel* sk);
  * skl_mapoverlap_create fail with SKL_ERR_OUT_OF_RANGE).                     */
 skl_status skl_mapoverlap_bounds(skl_skel* sk, int* proven);
 
+/* Allpairs: for an n x d matrix A and an
+ * m x d matrix B, C (n x m) has C[i][j] = A_i (+) B_j over rows.
+ * skl_allpairs_create: the customising function receives both rows and d,
+ *   `TOUT f(const TIN* a, const TIN* b, int d)` (reading A35).
+ * skl_allpairs_zr_create: C[i][j] = fold((+), zip((x), A_i, B_j)) with two
+ *   binary customising functions - z = zip(a_k, b_k) (TIN x TIN -> TOUT) and
+ *   the left fold acc = z_0, acc = (+)(acc, z_k) (TOUT x TOUT -> TOUT), e.g. the
+ *   Manhattan distance or dotProduct (Eq. (1)); register-tiled on the
+ *   FP32 pipes, each element folded in k order (reading A36).
+ * Distributions: A as set (default block rows), B made copy, C like A.       */
+skl_status skl_allpairs_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in,
+                               skl_type out, skl_skel** sk);
+skl_status skl_allpairs_zr_create(skl_ctx* ctx, const char* zip_src, const char* zip_entry,
+                                  const char* reduce_src, const char* reduce_entry, skl_type in,
+                                  skl_type out, skl_skel** sk);
+skl_status skl_allpairs_run(skl_skel* sk, skl_cont* A, skl_cont* B, skl_cont** C);
+
 /* One extra argument at run time.                                             */
 #define SKL_ARG_SCALAR 1
 #define SKL_ARG_CONT 2

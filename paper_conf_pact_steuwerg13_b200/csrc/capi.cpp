@@ -417,6 +417,24 @@ skl_status skl_mapoverlap_create(skl_ctx* ctx, const char* src, const char* entr
     *sk = wrap(skel_create(C(ctx), K_MAPOVERLAP, src, entry, in, 0, out, nullptr, 0, d, boundary, neutral));
   });
 }
+skl_status skl_allpairs_create(skl_ctx* ctx, const char* src, const char* entry, skl_type in,
+                               skl_type out, skl_skel** sk) {
+  return guard([&] {
+    if (!sk) fail(SKL_ERR_INVALID_ARG, "NULL out");
+    *sk = wrap(allpairs_create(C(ctx), src, entry, nullptr, nullptr, in, out));
+  });
+}
+skl_status skl_allpairs_zr_create(skl_ctx* ctx, const char* zip_src, const char* zip_entry,
+                                  const char* reduce_src, const char* reduce_entry, skl_type in,
+                                  skl_type out, skl_skel** sk) {
+  return guard([&] {
+    if (!sk || !reduce_src) fail(SKL_ERR_INVALID_ARG, "NULL out / reduce source");
+    *sk = wrap(allpairs_create(C(ctx), zip_src, zip_entry, reduce_src, reduce_entry, in, out));
+  });
+}
+skl_status skl_allpairs_run(skl_skel* sk, skl_cont* a, skl_cont* b, skl_cont** c) {
+  return run_out(c, [&](Cont** o) { run_allpairs(S(sk), K(a), K(b), o); });
+}
 skl_status skl_mapoverlap_bounds(skl_skel* sk, int* proven) {
   return guard([&] {
     Skel* s = S(sk);

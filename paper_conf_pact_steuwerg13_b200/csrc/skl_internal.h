@@ -223,7 +223,7 @@ std::string detect_entry(const std::string& src);
 std::string kernel_template(const char* name);  // embedded kernels/*.cuh
 
 // ------------------------------------------------------------------ skeletons
-enum SkelKind { K_MAP = 1, K_ZIP, K_REDUCE, K_SCAN, K_MAPOVERLAP };
+enum SkelKind { K_MAP = 1, K_ZIP, K_REDUCE, K_SCAN, K_MAPOVERLAP, K_ALLPAIRS };
 struct Scratch {  // per-device persistent scratch (reduce partials, scan status)
   void* ptr = nullptr;
   size_t bytes = 0;
@@ -250,6 +250,7 @@ struct Skel {
   int scan_variant = 0;
   int scan_fstride = 16;  // Scan: status word spacing in 8-byte units
   int bounds = 0;         // MapOverlap: 1 = get() offsets statically proven within d
+  bool ap_zr = false;     // Allpairs: zip-reduce form
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
   std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
@@ -262,6 +263,9 @@ void run_zip(Skel* s, Cont* l, Cont* r, Cont** out, const skl_arg* extra, int ne
 void run_reduce(Skel* s, Cont* in, Cont** out);
 void run_scan(Skel* s, Cont* in, Cont** out);
 void run_mapoverlap(Skel* s, Cont* in, Cont** out);
+Skel* allpairs_create(Ctx* ctx, const char* src, const char* entry, const char* rsrc,
+                      const char* rentry, int tin, int tout);  // rsrc != NULL: zip-reduce form
+void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out);
 // ordered combine of G staged replica slices into dst (A25), on device g
 void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
                  size_t nelem);

@@ -90,6 +90,9 @@ def lib():
         "skl_scalar_get": [vp, vp, sz],
         "skl_skel_cubin": [vp, vp, sz, C.POINTER(sz)], "skl_skel_source": [vp, C.c_char_p, sz, C.POINTER(sz)],
         "skl_mapoverlap_bounds": [vp, C.POINTER(i)],
+        "skl_allpairs_create": [vp, C.c_char_p, C.c_char_p, i, i, pp],
+        "skl_allpairs_zr_create": [vp, C.c_char_p, C.c_char_p, C.c_char_p, C.c_char_p, i, i, pp],
+        "skl_allpairs_run": [vp, vp, vp, pp],
         "skl_capture_begin": [vp], "skl_capture_end": [vp, pp], "skl_graph_launch": [vp],
         "skl_graph_destroy": [vp],
         "skl_plan_range": [sz, i, i, i, i, i, C.POINTER(sz), C.POINTER(sz)],
@@ -518,6 +521,31 @@ class MapOverlap(Skeleton):
         v = C.c_int()
         check(lib().skl_mapoverlap_bounds(self._h, C.byref(v)))
         return bool(v.value)
+
+
+class Allpairs(Skeleton):
+    """allpairs(+)(A, B): C[i][j] = A_i (+) B_j over rows.
+
+    Allpairs(ctx, "float f(const float* a, const float* b, int d){...}", F32, F32)
+    Allpairs(ctx, zip_src, F32, F32, reduce=reduce_src)   # fold((+), zip((x), A_i, B_j))
+    """
+
+    def __init__(self, ctx, src: str, tin: int, tout: int, reduce: str = None, entry=None,
+                 reduce_entry=None):
+        h = C.c_void_p()
+        if reduce is None:
+            check(lib().skl_allpairs_create(ctx.handle, src.encode(), entry.encode() if entry else None,
+                                            tin, tout, C.byref(h)))
+        else:
+            check(lib().skl_allpairs_zr_create(ctx.handle, src.encode(), entry.encode() if entry else None,
+                                               reduce.encode(), reduce_entry.encode() if reduce_entry else None,
+                                               tin, tout, C.byref(h)))
+        super().__init__(ctx, h, tout)
+
+    def __call__(self, a: Container, b: Container, out: Container = None) -> Container:
+        o = C.c_void_p(out.handle.value if out is not None else None)
+        check(lib().skl_allpairs_run(self._h, a.handle, b.handle, C.byref(o)))
+        return out if out is not None else _wrap_out(self.ctx, o, self.tout)
 
 
 # ---------------------------------------------------------------- host-only planning

@@ -1,0 +1,72 @@
+"""Allpairs on the GPU vs the oracle: both forms (row function;
+zip + reduce), bit-exact (every C element is folded over k in order in fp32,
+-fmad=false, as the oracle does), ragged tile edges, block(A) x copy(B) on
+several logical devices."""
+import numpy as np
+import pytest
+
+import oracle as O
+from gpu_util import require_gpu
+from paper_conf_pact_steuwerg13_b200 import apps as A
+from paper_conf_pact_steuwerg13_b200 import inputs as I
+from paper_conf_pact_steuwerg13_b200 import skl as S
+
+pytestmark = pytest.mark.gpu
+
+SHAPES = [(1, 1, 1), (2, 3, 3), (70, 33, 13), (130, 200, 64), (257, 129, 100), (64, 64, 16)]
+
+
+@pytest.fixture(scope="module", params=[1, 3])
+def ctx(request):
+    require_gpu()
+    G = request.param
+    c = S.Context(G, devices=[0] * G)
+    yield c
+    c.finalize()
+
+
+@pytest.fixture(scope="module")
+def sk(ctx):
+    return dict(
+        man=S.Allpairs(ctx, A.MANHATTAN_ROWS, S.F32, S.F32),
+        dot=S.Allpairs(ctx, A.DOT_ROWS, S.F32, S.F32),
+        man_zr=S.Allpairs(ctx, A.ABSDIFF, S.F32, S.F32, reduce=A.ADD),
+        dot_zr=S.Allpairs(ctx, A.MULT, S.F32, S.F32, reduce=A.ADD),
+    )
+
+
+@pytest.mark.parametrize("shape", SHAPES)
+def test_allpairs_bitexact(ctx, sk, shape):
+    n, m, d = shape
+    a = I.uniform_f32(81, n * d).reshape(n, d) - np.float32(0.5)
+    b = I.uniform_f32(82, m * d).reshape(m, d) - np.float32(0.5)
+    ma = S.Matrix.from_numpy(ctx, a).set_distribution(S.BLOCK)
+    mb = S.Matrix.from_numpy(ctx, b)
+    man = O.allpairs(O.AP_MANHATTAN, a, b)
+    dot = O.allpairs(O.AP_DOT, a, b)
+    assert np.array_equal(sk["man"](ma, mb).to_numpy(), man)
+    assert np.array_equal(sk["dot"](ma, mb).to_numpy(), dot)
+    assert np.array_equal(sk["man_zr"](ma, mb).to_numpy(), man)
+    c = sk["dot_zr"](ma, mb)
+    assert c.distribution()[0] == S.BLOCK
+    assert np.array_equal(c.to_numpy(), dot)
+
+
+def test_golden_and_eq2(ctx, sk, golden):
+    g = golden("allpairs_small.txt")
+    a, b = np.array(g["A"], np.float32), np.array(g["B"], np.float32)
+    ma, mb = S.Matrix.from_numpy(ctx, a), S.Matrix.from_numpy(ctx, b)
+    assert np.array_equal(sk["dot_zr"](ma, mb).to_numpy(), np.array(g["dot"], np.float32))
+    assert np.array_equal(sk["man"](ma, mb).to_numpy(), np.array(g["manhattan"], np.float32))
+    # Eq. (2): A x B = allpairs(dotProduct)(A, B^T)
+    x = I.uniform_f32(83, 96 * 40).reshape(96, 40)
+    y = I.uniform_f32(84, 40 * 72).reshape(40, 72)
+    c = sk["dot_zr"](S.Matrix.from_numpy(ctx, x), S.Matrix.from_numpy(ctx, np.ascontiguousarray(y.T))).to_numpy()
+    assert np.allclose(c, x.astype(np.float64) @ y.astype(np.float64), rtol=1e-5, atol=1e-5)
+
+
+def test_size_mismatch(ctx, sk):
+    with pytest.raises(S.SklError) as e:
+        sk["man"](S.Matrix.from_numpy(ctx, np.zeros((3, 4), np.float32)),
+                  S.Matrix.from_numpy(ctx, np.zeros((3, 5), np.float32)))
+    assert e.value.name == "SIZE_MISMATCH"
