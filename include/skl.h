@@ -106,10 +106,17 @@ skl_status skl_get_stream(skl_ctx* ctx, int g, void** cuda_stream);
 skl_status skl_sync(skl_ctx* ctx);
 /* Options: "block_threads" (work-group size; default 256),
  * "debug_bounds" (1 = get() range-checked, A21), "map_unroll" (chunks per
- * thread, default 4).                                                          */
+ * thread, default 4), "lazy_fusion" (1 = a Map/Zip without an output is
+ * deferred and fused into the Reduce that consumes it; default 1),
+ * "halo_push" (1 = a MapOverlap on several devices of this process stores its
+ * border units into the neighbours' halo units, so the next overlap read
+ * exchanges nothing; default 1), plus the Scan/MapOverlap tuning
+ * keys listed in DESIGN.md 6.                                                  */
 skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
 /* Counters: "launches" (kernels this library launched), "compiles" (NVRTC runs),
- * "cache_hits", "h2d_bytes", "d2h_bytes", "p2p_bytes" (device-to-device bytes). */
+ * "cache_hits", "h2d_bytes", "d2h_bytes", "p2p_bytes" (device-to-device copy
+ * bytes), "halo_push_bytes" (halo bytes stored by MapOverlap kernels directly
+ * into neighbour devices' memory).                                             */
 skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value);
 const char* skl_last_error(void);
 

@@ -188,6 +188,10 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "mo_rh" || k == "mo_cw") {
       if (value < 0 || value > 32) fail(SKL_ERR_INVALID_ARG, k + " in [0,32]");
       (k == "mo_rh" ? c->mo_rh : c->mo_cw) = (int)value;
+    } else if (k == "lazy_fusion") {
+      c->lazy_fusion = value ? 1 : 0;
+    } else if (k == "halo_push") {
+      c->halo_push = value ? 1 : 0;
     } else if (k == "scan_variant") {
       c->scan_variant = (int)value;
     } else if (k == "scan_persistent") {
@@ -211,6 +215,7 @@ skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value) {
     else if (k == "h2d_bytes") *value = c->h2d;
     else if (k == "d2h_bytes") *value = c->d2h;
     else if (k == "p2p_bytes") *value = c->p2p;
+    else if (k == "halo_push_bytes") *value = c->pushed;
     else fail(SKL_ERR_INVALID_ARG, "unknown counter " + k);
   });
 }

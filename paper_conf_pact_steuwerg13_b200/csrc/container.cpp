@@ -101,6 +101,7 @@ void mark_written(Cont* c) {
   c->dev_valid = true;
   c->host_valid = false;
   c->halo_valid = false;
+  c->halo_ready = 0;
   set_valid(c, c->dist, false);
 }
 
@@ -114,6 +115,7 @@ void prepare_output(Cont* c, const Dist& d, size_t spare) {
   c->diverged = false;
   c->dev_valid = false;
   c->halo_valid = false;
+  c->halo_ready = 0;
 }
 
 // ------------------------------------------------------------------ host <-> device
@@ -143,6 +145,7 @@ void host_upload(Cont* c, const void* host) {
   set_valid(c, d, true);
   c->dev_valid = true;
   c->halo_valid = true;
+  c->halo_ready = 0;
   c->diverged = false;
 }
 
@@ -257,6 +260,7 @@ void* host_mirror(Cont* c, int mode) {
   if (mode & SKL_WRITE) {
     c->host_valid = true;
     c->dev_valid = false;  // devices become stale
+    c->halo_ready = 0;
     c->diverged = false;
   }
   return c->host;
@@ -280,6 +284,7 @@ void fill(Cont* c, const void* value) {
   set_valid(c, c->dist, true);
   c->dev_valid = true;
   c->halo_valid = true;
+  c->halo_ready = 0;
   c->host_valid = false;
   c->diverged = false;
 }
@@ -344,6 +349,7 @@ static void combine_to_block(Cont* c) {
   c->diverged = false;
   c->dev_valid = true;
   c->halo_valid = false;
+  c->halo_ready = 0;
   set_valid(c, blk, false);
 }
 
@@ -393,7 +399,17 @@ static void redistribute(Cont* c, const Dist& to) {
   c->dist = to;
   c->dev_valid = true;
   c->halo_valid = to_halo;
+  c->halo_ready = 0;
   set_valid(c, to, to_halo);
+}
+
+static bool halos_allocated(Cont* c, const Dist& d) {
+  for (int g = c->ctx->first_local; g < c->ctx->first_local + c->ctx->nlocal; ++g) {
+    const Range n = need_range(c->units(), c->ctx->G, d, g);
+    const Part& p = c->parts[(size_t)g];
+    if (!n.empty() && (!p.ptr || !p.buf.contains(n))) return false;
+  }
+  return true;
 }
 
 void ensure(Cont* c, const Dist& d, bool halo) {
@@ -404,6 +420,15 @@ void ensure(Cont* c, const Dist& d, bool halo) {
   }
   if (c->dev_valid && c->dist.kind == DCOPY && c->diverged && d.kind == DCOPY && c->combine) {
     copy_combine_to_copy(c);
+    return;
+  }
+  if (c->dev_valid && c->halo_ready && c->dist.kind == DBLOCK && d.kind == DOVERLAP &&
+      (size_t)d.arg <= c->halo_ready && halos_allocated(c, d)) {
+    // the producing MapOverlap already stored the border units into the
+    // neighbours' halo rows (fused halo push): block -> overlap moves nothing
+    c->dist = d;
+    c->halo_valid = true;
+    set_valid(c, d, true);
     return;
   }
   if (c->dist == d && c->dev_valid) {
@@ -432,6 +457,7 @@ void ensure(Cont* c, const Dist& d, bool halo) {
       set_valid(c, d, true);
       c->dev_valid = true;
       c->halo_valid = true;
+      c->halo_ready = 0;
     }
     return;
   }

@@ -91,17 +91,24 @@ Ctx* ctx_create_local(int ndev, const int* devices) {
       init_device(c, c->dev[(size_t)g]);
     }
     // peer access between distinct physical GPUs (NVLink / NVSwitch)
+    c->peer_ok.assign((size_t)c->G, std::vector<char>((size_t)c->G, 0));
     for (auto& a : c->dev)
-      for (auto& b : c->dev)
-        if (a.phys != b.phys) {
-          int can = 0;
-          cudaDeviceCanAccessPeer(&can, a.phys, b.phys);
-          if (can) {
-            cudaSetDevice(a.phys);
-            cudaError_t pe = cudaDeviceEnablePeerAccess(b.phys, 0);
-            if (pe != cudaSuccess) cudaGetLastError();  // already enabled is fine
-          }
+      for (auto& b : c->dev) {
+        char& ok = c->peer_ok[(size_t)a.global][(size_t)b.global];
+        if (a.phys == b.phys) {
+          ok = 1;
+          continue;
         }
+        int can = 0;
+        cudaDeviceCanAccessPeer(&can, a.phys, b.phys);
+        if (can) {
+          cudaSetDevice(a.phys);
+          cudaError_t pe = cudaDeviceEnablePeerAccess(b.phys, 0);
+          if (pe == cudaErrorPeerAccessAlreadyEnabled) pe = cudaSuccess;
+          if (pe != cudaSuccess) cudaGetLastError();
+          ok = pe == cudaSuccess;
+        }
+      }
   } catch (...) {
     delete c;
     throw;

@@ -43,7 +43,8 @@ __device__ __forceinline__ long skl_clampl(long v, long lo, long hi) {
 
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
-         long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok) {
+         long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
+         SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
   __shared__ __align__(16) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
   const long r0 = r_begin + (long)blockIdx.y * SKL_TH;
   const long c0 = (long)blockIdx.x * SKL_TW;
@@ -101,16 +102,26 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
     // f may declare a non-const pointer (Listing 1.2: "float func(float* m_in)")
     for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
     if (r < r_end) {
-      SKL_TOUT* o = out + (r - out_row0) * C + cc;
+      // fused halo push: the first / last hd rows of this device's block are
+      // also stored into the neighbours' halo rows (peer memory), so the next
+      // overlap read needs no exchange
+      SKL_TOUT* dst[3] = {out + (r - out_row0) * C + cc, nullptr, nullptr};
+      if (push_up && r < r_begin + hd) dst[1] = push_up + (r - r_begin) * C + cc;
+      if (push_down && r >= r_end - hd) dst[2] = push_down + (r - (r_end - hd)) * C + cc;
+#pragma unroll
+      for (int k = 0; k < 3; ++k) {
+        SKL_TOUT* o = dst[k];
+        if (!o) continue;
 #if SKL_OUT_PACK
-      if (cc + SKL_CW <= C && vec_ok) {
-        *(typename SklRaw<SKL_OUTB>::type*)o = res.raw;
-        continue;
-      }
+        if (cc + SKL_CW <= C && vec_ok) {
+          *(typename SklRaw<SKL_OUTB>::type*)o = res.raw;
+          continue;
+        }
 #endif
 #pragma unroll
-      for (int j = 0; j < SKL_CW; ++j)
-        if (cc + j < C) o[j] = res.e[j];
+        for (int j = 0; j < SKL_CW; ++j)
+          if (cc + j < C) o[j] = res.e[j];
+      }
     }
   }
   (void)in_rows;
@@ -120,7 +131,8 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
 #define SKL_SLEN (SKL_TW + 2 * SKL_A)
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_mo1d(const SKL_TIN* __restrict__ in, long in_lo, long in_n, SKL_TOUT* __restrict__ out,
-         long out_lo, long N, long unused, long i_begin, long i_end, SKL_TIN neutral, int vec_ok) {
+         long out_lo, long N, long unused, long i_begin, long i_end, SKL_TIN neutral, int vec_ok,
+         SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
   __shared__ __align__(16) SKL_TIN tile[SKL_SLEN];
   const long e0 = i_begin + (long)blockIdx.x * SKL_TW;
   for (int q = threadIdx.x; q < SKL_SLEN / SKL_EPC; q += SKL_BLOCK) {
@@ -154,7 +166,12 @@ skl_mo1d(const SKL_TIN* __restrict__ in, long in_lo, long in_n, SKL_TOUT* __rest
 #pragma unroll
   for (int j = 0; j < SKL_CW; ++j) {
     const long i = i0 + j;
-    if (i < i_end) out[i - out_lo] = SKL_FUNC((SKL_TIN*)(p + j));
+    if (i < i_end) {
+      const SKL_TOUT v = SKL_FUNC((SKL_TIN*)(p + j));
+      out[i - out_lo] = v;
+      if (push_up && i < i_begin + hd) push_up[i - i_begin] = v;          // fused halo push
+      if (push_down && i >= i_end - hd) push_down[i - (i_end - hd)] = v;
+    }
   }
   (void)unused;
 }

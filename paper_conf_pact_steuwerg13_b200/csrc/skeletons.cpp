@@ -700,6 +700,35 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
 }
 
 // ------------------------------------------------------------------ MapOverlap
+// Fused halo push: with every device of a block-distributed
+// output in this process, device g's kernel also stores its first / last d
+// units into the halo units of devices g-1 / g+1 (peer memory over NVLink, or
+// the same GPU for logical devices), so a following overlap(d) read moves no
+// data.  Taken only when every core holds >= d units (each halo unit then has
+// exactly one producer, the adjacent device) and peer stores are possible.
+static bool plan_halo_push(Ctx* ctx, Cont* o, size_t d, std::vector<void*>& up, std::vector<void*>& down) {
+  const int G = ctx->G;
+  if (!ctx->halo_push || ctx->dist_mode || G < 2 || ctx->nlocal != G || d == 0) return false;
+  if (o->dist.kind != DBLOCK) return false;
+  up.assign((size_t)G, nullptr);
+  down.assign((size_t)G, nullptr);
+  for (int g = 0; g < G; ++g) {
+    const Range r = core_range(o->units(), G, o->dist, g);
+    if (r.size() < d) return false;
+    const Range want = need_range(o->units(), G, Dist{DOVERLAP, (int)d}, g);
+    const Part& p = o->parts[(size_t)g];
+    if (!p.ptr || !p.buf.contains(want)) return false;
+    if (g > 0 && !ctx->peer_ok[(size_t)g][(size_t)g - 1]) return false;
+    if (g + 1 < G && !ctx->peer_ok[(size_t)g][(size_t)g + 1]) return false;
+  }
+  for (int g = 0; g < G; ++g) {
+    const Range r = core_range(o->units(), G, o->dist, g);
+    if (g > 0) up[(size_t)g] = part_ptr(o, g - 1, r.lo);
+    if (g + 1 < G) down[(size_t)g] = part_ptr(o, g + 1, r.hi - d);
+  }
+  return true;
+}
+
 void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   if (s->kind != K_MAPOVERLAP) fail(SKL_ERR_INVALID_ARG, "not a MapOverlap skeleton");
   Ctx* ctx = s->ctx;
@@ -715,6 +744,17 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   if (o == in) fail(SKL_ERR_INVALID_ARG, "MapOverlap cannot run in place");
   prepare_output(o, dout, dout.kind == DBLOCK ? (size_t)d : 0);
   const size_t si = in->elt, so = o->elt;
+  std::vector<void*> push_up, push_down;
+  const bool push = plan_halo_push(ctx, o, (size_t)d, push_up, push_down);
+  long hd = push ? (long)d : 0;
+  // the pushes overwrite halo units the neighbours may still be reading
+  if (push) barrier_streams(ctx);
+  auto push_ptrs = [&](int g, void** pu, void** pd) {
+    *pu = push ? push_up[(size_t)g] : nullptr;
+    *pd = push ? push_down[(size_t)g] : nullptr;
+    if (*pu) ctx->pushed += (long long)((size_t)d * o->unit_bytes());
+    if (*pd) ctx->pushed += (long long)((size_t)d * o->unit_bytes());
+  };
   if (in->matrix) {
     for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
       const Range r = core_range(in->units(), ctx->G, dout, g);
@@ -726,10 +766,13 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       long in_row0 = (long)pi.buf.lo, in_rows = (long)pi.buf.size(), out_row0 = (long)po.buf.lo;
       long R = (long)in->rows, C = (long)in->cols, rb = (long)r.lo, re = (long)r.hi;
       const int cw = s->mo_tw / 32;
-      int vec_ok = ((size_t)C * si) % 16 == 0 && aligned16(pin) && ((size_t)C * so) % ((size_t)cw * so) == 0 &&
-                   ((uintptr_t)pout % ((size_t)cw * so) == 0);
+      void *pu, *pd;
+      push_ptrs(g, &pu, &pd);
+      const size_t ow = (size_t)cw * so;
+      int vec_ok = ((size_t)C * si) % 16 == 0 && aligned16(pin) && ((size_t)C * so) % ow == 0 &&
+                   (uintptr_t)pout % ow == 0 && (uintptr_t)pu % ow == 0 && (uintptr_t)pd % ow == 0;
       void* args[] = {(void*)&pin, &in_row0, &in_rows, &pout, &out_row0, &R, &C, &rb, &re,
-                      s->neutral.data(), &vec_ok};
+                      s->neutral.data(), &vec_ok, &pu, &pd, &hd};
       const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
                       (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
       launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(s->block), 0, args);
@@ -764,13 +807,19 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       long in_lo = (long)pi.buf.lo, in_n = (long)pi.buf.size(), out_lo = (long)po.buf.lo;
       long N = (long)in->rows, unused = 0, rb = (long)r.lo, re = (long)r.hi;
       int vec_ok = aligned16(pin);
+      void *pu, *pd;
+      push_ptrs(g, &pu, &pd);
       void* args[] = {(void*)&pin, &in_lo, &in_n, &pout, &out_lo, &N, &unused, &rb, &re,
-                      s->neutral.data(), &vec_ok};
+                      s->neutral.data(), &vec_ok, &pu, &pd, &hd};
       launch(ctx, g, s->prog1d, "skl_mo1d", dim3((unsigned)ceil_div(r.size(), (size_t)tw)),
              dim3(s->block), 0, args);
     }
   }
   mark_written(o);
+  if (push) {
+    o->halo_ready = (size_t)d;
+    barrier_streams(ctx);  // the neighbours' next reads of their halos wait for the pushes
+  }
   if (ctx->debug_bounds) check_debug_flag(ctx);
 }
 

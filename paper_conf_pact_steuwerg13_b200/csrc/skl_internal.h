@@ -120,12 +120,14 @@ struct Ctx {
   int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
+  int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
+  std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest
   // measured); 2 = one block per tile, warp-wide look-back; 0 = persistent
   // chunked (L2 re-read); 1 = measurement only: no look-back (wrong results)
   int scan_variant = 3;
   // counters
-  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0};
+  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0};
   // NVRTC cache: source hash -> program
   std::map<std::string, std::unique_ptr<Program>> programs;
   // builtin kernels (fill) per element size
@@ -173,6 +175,9 @@ struct Cont {
   void* host = nullptr;      // pinned host mirror (lazily allocated)
   bool host_valid = false;
   size_t spare_halo = 0;     // allocate parts with this many extra halo units
+  // block-distributed, but the buffers already hold valid halos of this many
+  // units (pushed by the producing MapOverlap): overlap(d <= halo_ready) is free
+  size_t halo_ready = 0;
 };
 
 // container.cpp
