@@ -165,7 +165,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "debug_bounds") {
       c->debug_bounds = value ? 1 : 0;
     } else if (k == "scan_chunks") {
-      if (value != 2 && value != 4 && value != 8) fail(SKL_ERR_INVALID_ARG, "scan_chunks in {2,4,8}");
+      if (value != 2 && value != 4 && value != 6 && value != 8 && value != 12 && value != 16)
+        fail(SKL_ERR_INVALID_ARG, "scan_chunks in {2,4,6,8,12,16}");
       c->scan_chunks = (int)value;
     } else if (k == "scan_sub") {
       if (value < 1 || value > 64) fail(SKL_ERR_INVALID_ARG, "scan_sub in [1,64]");

@@ -293,7 +293,8 @@ __device__ __forceinline__ void skl_scan_tile(SKL_T (&items)[ITEMS], int cnt, in
                                               unsigned tile, unsigned* flags, SKL_T* aggs, SKL_T* incls,
                                               unsigned epoch, const SKL_T* carry, int ncarry,
                                               bool pre_has = false, const SKL_T* pre_in = nullptr,
-                                              SKL_T* agg_out = nullptr) {
+                                              SKL_T* agg_out = nullptr, int* pre_has_out = nullptr,
+                                              SKL_T* pre_out = nullptr) {
   SklOp op;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   // 1. sequential inclusive scan inside the thread
@@ -336,7 +337,7 @@ __device__ __forceinline__ void skl_scan_tile(SKL_T (&items)[ITEMS], int cnt, in
       if (pre_has) s_excl = *pre_in;
     }
   } else {
-#if SKL_SCAN_VARIANT == 1
+#if SKL_SCAN_VARIANT == 1 || SKL_SCAN_VARIANT == 7
     // measurement variant only (skl_set_option "scan_variant" 1): no look-back,
     // i.e. per-tile scans - the load/scan/store pipeline's own ceiling
     if (threadIdx.x == 0) s_has = 0;
@@ -360,6 +361,11 @@ __device__ __forceinline__ void skl_scan_tile(SKL_T (&items)[ITEMS], int cnt, in
   if (lane > 0) {
     pre = hp ? op(pre, lane_excl) : lane_excl;
     hp = true;
+  }
+  if (pre_has_out) {  // the caller applies the prefix itself
+    *pre_has_out = hp;
+    if (hp) *pre_out = pre;
+    return;
   }
   if (hp) {
 #pragma unroll
@@ -608,6 +614,90 @@ skl_scan_pt(const SKL_T* __restrict__ in, SKL_T* __restrict__ out, skl_u64 n, un
   for (int q = 0; q < SKL_ITEMS; ++q) my.e[q] = items[q];
 #pragma unroll
   for (int q = 0; q < SKL_CH; ++q) sm[skl_swz(threadIdx.x * SKL_CH + q)] = my.q[q];
+  __syncthreads();
+  char* gout = (char*)(out + tlo);
+  if (nvalid == SKL_TILE) {
+#pragma unroll
+    for (int i = 0; i < SKL_CH; ++i) {
+      const unsigned cc = i * SKL_BLOCK + threadIdx.x;
+      skl_st16(gout + 16 * (skl_u64)cc, sm[skl_swz(cc)]);
+    }
+  } else {
+    for (int e = threadIdx.x; e < nvalid; e += SKL_BLOCK)
+      out[tlo + e] = *((const SKL_T*)&sm[skl_swz(e / SKL_EPC)] + (e % SKL_EPC));
+  }
+}
+
+// Low-register per-tile variant (SKL_SCAN_VARIANT 6): the tile stays in shared
+// memory; a thread folds its SKL_ITEMS elements to one total (16-byte reads),
+// the block scans the totals and looks back, then the thread re-reads its
+// elements and writes pre (+) x0, (pre (+) x0) (+) x1, ... in place.  No item
+// array lives in registers, so more tiles (SKL_MINB) fit per SM: the look-back
+// latency of one tile is hidden behind the loads of the others.
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MINB)
+skl_scan_lr(const SKL_T* __restrict__ in, SKL_T* __restrict__ out, skl_u64 n, unsigned* flags,
+            SKL_T* aggs, SKL_T* incls, unsigned epoch, const SKL_T* carry, int ncarry) {
+  extern __shared__ uint4 skl_dyn[];
+  uint4* sm = skl_dyn;
+  SklOp op;
+  const unsigned t = blockIdx.x;
+  const skl_u64 tlo = (skl_u64)t * SKL_TILE;
+  const int nvalid = n - tlo >= (skl_u64)SKL_TILE ? SKL_TILE : (int)(n - tlo);
+  skl_scan_issue(in, tlo, nvalid, sm);
+  skl_cp_commit();
+  asm volatile("cp.async.wait_group 0;" ::: "memory");
+  __syncthreads();
+  const int first = threadIdx.x * SKL_ITEMS;
+  const int cnt = nvalid - first >= SKL_ITEMS ? SKL_ITEMS : (nvalid - first > 0 ? nvalid - first : 0);
+  const int nthr = (nvalid + SKL_ITEMS - 1) / SKL_ITEMS;
+#define SKL_LR_ELT(k) (*((SKL_T*)&sm[skl_swz((unsigned)(first + (k)) / SKL_EPC)] + ((first + (k)) % SKL_EPC)))
+  SKL_T tot[1];
+  if (cnt == SKL_ITEMS) {
+    SklChunk<SKL_T, SKL_EPC> c0;
+    c0.q[0] = sm[skl_swz(threadIdx.x * SKL_CH)];
+    tot[0] = c0.e[0];
+#pragma unroll
+    for (int e = 1; e < SKL_EPC; ++e) tot[0] = op(tot[0], c0.e[e]);
+#pragma unroll
+    for (int q = 1; q < SKL_CH; ++q) {
+      SklChunk<SKL_T, SKL_EPC> c;
+      c.q[0] = sm[skl_swz(threadIdx.x * SKL_CH + q)];
+#pragma unroll
+      for (int e = 0; e < SKL_EPC; ++e) tot[0] = op(tot[0], c.e[e]);
+    }
+  } else if (cnt > 0) {
+    tot[0] = SKL_LR_ELT(0);
+    for (int k = 1; k < cnt; ++k) tot[0] = op(tot[0], SKL_LR_ELT(k));
+  }
+  int hp = 0;
+  SKL_T pre;
+  skl_scan_tile<1, true>(tot, cnt > 0 ? 1 : 0, nthr, t, flags, aggs, incls, epoch, carry, ncarry, false,
+                         nullptr, nullptr, &hp, &pre);
+  if (cnt == SKL_ITEMS) {
+#pragma unroll
+    for (int q = 0; q < SKL_CH; ++q) {
+      SklChunk<SKL_T, SKL_EPC> c;
+      c.q[0] = sm[skl_swz(threadIdx.x * SKL_CH + q)];
+#pragma unroll
+      for (int e = 0; e < SKL_EPC; ++e) {
+        if (q == 0 && e == 0) {
+          if (hp) c.e[0] = op(pre, c.e[0]);
+        } else {
+          c.e[e] = op(pre, c.e[e]);
+        }
+        pre = c.e[e];
+      }
+      sm[skl_swz(threadIdx.x * SKL_CH + q)] = c.q[0];
+    }
+  } else if (cnt > 0) {
+    for (int k = 0; k < cnt; ++k) {
+      SKL_T v = SKL_LR_ELT(k);
+      if (k > 0 || hp) v = op(pre, v);
+      SKL_LR_ELT(k) = v;
+      pre = v;
+    }
+  }
+#undef SKL_LR_ELT
   __syncthreads();
   char* gout = (char*)(out + tlo);
   if (nvalid == SKL_TILE) {

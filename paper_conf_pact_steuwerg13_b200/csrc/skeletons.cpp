@@ -677,7 +677,11 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
     const void* cptr = carry ? totals[g] : nullptr;
     int ncarry = carry ? i : 0;
     void* args[] = {(void*)&pin, &pout, &nn, &flags, &aggs, &incls, &ep, (void*)&cptr, &ncarry};
-    if (vec && per_tile && s->scan_variant >= 4) {
+    if (vec && per_tile && (s->scan_variant == 6 || s->scan_variant == 7)) {
+      // low-register per-tile kernel (tile in shared memory)
+      const size_t smem = (size_t)s->block * (size_t)s->scan_ch * 16;
+      launch(ctx, g, s->prog, "skl_scan_lr", dim3((unsigned)ntiles), dim3(s->block), smem, args);
+    } else if (vec && per_tile && s->scan_variant >= 4) {
       // persistent 3-stage pipeline: one wave of resident blocks
       const size_t smem = 3 * (size_t)s->block * (size_t)s->scan_ch * 16;
       const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_scan_pipe", s->block, smem));

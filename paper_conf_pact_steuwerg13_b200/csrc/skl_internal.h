@@ -115,17 +115,20 @@ struct Ctx {
   int scan_sub = 4;            // Scan tiles per look-back chunk
   int scan_fstride = 16;       // Scan status word spacing (8-byte units; 16 = one L2 line)
   int scan_spin_ns = 0;        // Scan look-back spin back-off (__nanosleep)
-  int scan_minb = 4;           // Scan per-tile kernel: min resident blocks (launch bounds)
+  int scan_minb = 5;           // Scan per-tile kernels: min resident blocks (launch bounds)
   int scan_minb_pipe = 2;      // Scan pipelined kernel: min resident blocks
   int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
-  // Scan schedule: 3 = one block per tile, block-wide look-back (default, fastest
-  // measured); 2 = one block per tile, warp-wide look-back; 0 = persistent
-  // chunked (L2 re-read); 1 = measurement only: no look-back (wrong results)
-  int scan_variant = 3;
+  // Scan schedule: 6 = one block per tile, tile kept in shared memory, low
+  // register count so 5 tiles fit per SM (default, fastest measured: 5.8 TB/s
+  // on 2^30 int32); 3 = one block per tile, items in registers, block-wide
+  // look-back; 2 = as 3 with a warp-wide look-back; 4 = persistent 3-stage
+  // pipeline; 0 = persistent chunked (L2 re-read); 1 / 5 / 7 = measurement
+  // only: 3 / 4 / 6 without look-back (wrong results, the pipeline's ceiling)
+  int scan_variant = 6;
   // counters
   std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0};
   // NVRTC cache: source hash -> program

@@ -88,15 +88,14 @@ def lmosem():
 
 
 def scan():
+    """configurations from SCAN_CFGS="variant,block,chunks,minb;..." (default: the shipped one)"""
     n = 1 << 30
-    for var, pers, bt, ch, fs, ns in ((3, 1, 256, 8, 16, 1), (3, 1, 256, 8, 16, 2), (3, 1, 256, 8, 16, 3),
-                                      (3, 1, 256, 8, 16, 4), (3, 1, 256, 8, 16, 6), (4, 1, 256, 8, 16, 3),
-                                      (3, 1, 128, 8, 16, 6)):
+    cfgs = [tuple(int(x) for x in t.split(",")) for t in os.environ.get("SCAN_CFGS", "3,256,8,4").split(";")]
+    for var, bt, ch, mb in cfgs:
+        pers, fs, ns = 1, 16, 1
         if True:
             if True:
-                c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_sub": pers,
-                              "scan_variant": var, "scan_fstride": fs, "scan_minb": 4 if bt == 256 else 8,
-                              "scan_lbw": ns})
+                c = ctx_with({"block_threads": bt, "scan_chunks": ch, "scan_variant": var, "scan_minb": mb})
                 sc = S.Scan(c, A.ADD_I32, S.I32)
                 v = S.Vector(c, S.I32, n).set_distribution(S.BLOCK).fill(1)
                 o = sc(v)
@@ -110,7 +109,7 @@ def scan():
                 got = torch.as_tensor(View(), device="cuda")
                 idx = torch.tensor([0, 1, 8191, 8192, 123456789, n // 2, n - 2, n - 1], device="cuda")
                 ok = bool(torch.equal(got[idx].long(), idx + 1))   # scan of ones = 1..n
-                print(f"scan i32 variant={var} sub={pers} block={bt} chunks={ch} fstride={fs} minb={ns}: {ms:.3f} ms  "
+                print(f"scan i32 variant={var} block={bt} chunks={ch} minb={mb}: {ms:.3f} ms  "
                       f"{8 * n / (ms / 1e3) / 1e9:.0f} GB/s ok={ok}", flush=True)
                 c.finalize()
 
