@@ -29,6 +29,7 @@ Skel* allpairs_create(Ctx* ctx, const char* src, const char* entry, const char* 
   s->block = 256;
   s->ap_zr = rsrc != nullptr;
   std::string defs = "#define SKL_BLOCK 256\n#define SKL_DEBUG_BOUNDS 0\n";
+  defs += std::string("#define SKL_AP_FAST ") + (si == 4 ? "1" : "0") + "\n";
   defs += "#define SKL_TIN " + ctx->type(tin).name + "\n#define SKL_TOUT " + ctx->type(tout).name + "\n";
   std::string body;
   if (s->ap_zr) {
@@ -83,8 +84,14 @@ void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out) {
     long nn = (long)r.size(), mm = (long)m, dd = (long)d;
     if (s->ap_zr) {
       void* args[] = {(void*)&pa, (void*)&pb, &pc, &nn, &mm, &dd};
-      launch(ctx, g, s->prog, "skl_ap_zr", dim3((unsigned)cdiv(m, 64), (unsigned)cdiv(r.size(), 64)),
-             dim3(256), 0, args);
+      const bool fast = si == 4 && d % 4 == 0 && ((uintptr_t)pa % 16) == 0 && ((uintptr_t)pb % 16) == 0 &&
+                        ctx->ap_fast;
+      if (fast)
+        launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)cdiv(r.size(), 128)),
+               dim3(256), 0, args);
+      else
+        launch(ctx, g, s->prog, "skl_ap_zr", dim3((unsigned)cdiv(m, 64), (unsigned)cdiv(r.size(), 64)),
+               dim3(256), 0, args);
     } else {
       const size_t smem = 32 * (d + 1) * si;
       int use_smem = smem <= 96 * 1024;

@@ -78,6 +78,124 @@ skl_ap_zr(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT
     }
   }
 }
+
+#if SKL_AP_FAST
+// 4-byte inputs, d % 4 == 0, 16-byte aligned rows: a 128 x 128 tile of C per
+// block, 8 x 8 per thread (rows ty + 16 r, columns tx + 16 c: consecutive
+// lanes read consecutive rows, so the 16-byte shared loads are conflict-free
+// with an 80-byte row pitch), k-slices of 16 staged row-major by cp.async into
+// a double buffer; per k-quad a thread issues 16 LDS.128 for 512 FP32 ops.
+// Every accumulator is still folded in k order (bit-exact with the oracle).
+#define AQ_BM 128
+#define AQ_BK 16
+#define AQ_P (AQ_BK + 4)
+#define AQ_STAGE (2 * AQ_BM * AQ_P)
+union SklAp4 {
+  uint4 q;
+  SKL_TIN e[4];
+};
+__device__ __forceinline__ void skl_ap_cp16(void* smem, const void* g) {
+  const unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
+  asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(g) : "memory");
+}
+template <bool FIRST>
+__device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][8], const SKL_TIN* As, const SKL_TIN* Bs,
+                                             int tx, int ty) {
+#pragma unroll
+  for (int kq = 0; kq < AQ_BK; kq += 4) {
+    SklAp4 a[8];
+#pragma unroll
+    for (int r = 0; r < 8; ++r) a[r].q = *(const uint4*)&As[(ty + 16 * r) * AQ_P + kq];
+#pragma unroll
+    for (int c = 0; c < 8; ++c) {
+      SklAp4 b;
+      b.q = *(const uint4*)&Bs[(tx + 16 * c) * AQ_P + kq];
+#pragma unroll
+      for (int j = 0; j < 4; ++j)
+#pragma unroll
+        for (int r = 0; r < 8; ++r) {
+          const SKL_TOUT z = SKL_ZFUNC(a[r].e[j], b.e[j]);
+          acc[r][c] = (FIRST && kq == 0 && j == 0) ? z : SKL_RFUNC(acc[r][c], z);
+        }
+    }
+  }
+}
+extern "C" __global__ void __launch_bounds__(256, 2)
+skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
+           long n, long m, long d) {
+  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE];
+  const int tx = threadIdx.x & 15, ty = threadIdx.x >> 4;
+  const long i0 = (long)blockIdx.y * AQ_BM, j0 = (long)blockIdx.x * AQ_BM;
+  const long nfull = d / AQ_BK;
+  // chunk q of a 128 x 16 slab: row q / 4, k-quad q % 4 (rows beyond n / m are
+  // clamped to the last one: loaded, never stored)
+  long ra[2], rb[2];
+#pragma unroll
+  for (int h = 0; h < 2; ++h) {
+    const int r = (threadIdx.x + h * 256) >> 2;
+    ra[h] = (i0 + r < n ? i0 + r : n - 1) * d;
+    rb[h] = (j0 + r < m ? j0 + r : m - 1) * d;
+  }
+  auto stage = [&](int st, long k0) {
+    SKL_TIN* As = sm + st * AQ_STAGE;
+    SKL_TIN* Bs = As + AQ_BM * AQ_P;
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {
+      const int q = threadIdx.x + h * 256, r = q >> 2, kq = (q & 3) * 4;
+      skl_ap_cp16(&As[r * AQ_P + kq], A + ra[h] + k0 + kq);
+      skl_ap_cp16(&Bs[r * AQ_P + kq], B + rb[h] + k0 + kq);
+    }
+  };
+  SKL_TOUT acc[8][8];
+  if (nfull > 0) stage(0, 0);
+  asm volatile("cp.async.commit_group;" ::: "memory");
+  for (long s = 0; s < nfull; ++s) {
+    if (s + 1 < nfull) stage((int)((s + 1) & 1), (s + 1) * AQ_BK);
+    asm volatile("cp.async.commit_group;" ::: "memory");
+    asm volatile("cp.async.wait_group 1;" ::: "memory");
+    __syncthreads();
+    const SKL_TIN* As = sm + (s & 1) * AQ_STAGE;
+    if (s == 0) skl_ap_slice<true>(acc, As, As + AQ_BM * AQ_P, tx, ty);
+    else skl_ap_slice<false>(acc, As, As + AQ_BM * AQ_P, tx, ty);
+    __syncthreads();  // the next stage() overwrites this buffer
+  }
+  // tail k-slice (d % 16 elements): scalar, guarded
+  const int kt = (int)(d - nfull * AQ_BK);
+  if (kt > 0) {
+    asm volatile("cp.async.wait_group 0;" ::: "memory");
+    SKL_TIN* As = sm;
+    SKL_TIN* Bs = As + AQ_BM * AQ_P;
+    const long k0 = nfull * AQ_BK;
+    for (int e = threadIdx.x; e < AQ_BM * AQ_BK; e += 256) {
+      const int r = e / AQ_BK, k = e % AQ_BK;
+      if (k < kt) {
+        const long ia = i0 + r < n ? i0 + r : n - 1, jb = j0 + r < m ? j0 + r : m - 1;
+        As[r * AQ_P + k] = A[ia * d + k0 + k];
+        Bs[r * AQ_P + k] = B[jb * d + k0 + k];
+      }
+    }
+    __syncthreads();
+    for (int k = 0; k < kt; ++k)
+#pragma unroll
+      for (int r = 0; r < 8; ++r)
+#pragma unroll
+        for (int c = 0; c < 8; ++c) {
+          const SKL_TOUT z = SKL_ZFUNC(As[(ty + 16 * r) * AQ_P + k], Bs[(tx + 16 * c) * AQ_P + k]);
+          acc[r][c] = (nfull == 0 && k == 0) ? z : SKL_RFUNC(acc[r][c], z);
+        }
+  }
+#pragma unroll
+  for (int r = 0; r < 8; ++r) {
+    const long i = i0 + ty + 16 * r;
+    if (i >= n) continue;
+#pragma unroll
+    for (int c = 0; c < 8; ++c) {
+      const long j = j0 + tx + 16 * c;
+      if (j < m) Cm[i * m + j] = acc[r][c];
+    }
+  }
+}
+#endif
 #else
 extern "C" __global__ void __launch_bounds__(256)
 skl_ap_gen(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,

@@ -120,7 +120,8 @@ struct Ctx {
   int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
-  int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
+  int halo_push = 1;
+  int ap_fast = 1;             // Allpairs zip-reduce: 128 x 128 tiles (4-byte inputs, d % 4 == 0)           // MapOverlap stores its border rows into the neighbours' halos
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 6 = one block per tile, tile kept in shared memory, low
   // register count so 5 tiles fit per SM (default, fastest measured: 5.8 TB/s

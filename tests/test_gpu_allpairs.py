@@ -13,7 +13,10 @@ from paper_conf_pact_steuwerg13_b200 import skl as S
 
 pytestmark = pytest.mark.gpu
 
-SHAPES = [(1, 1, 1), (2, 3, 3), (70, 33, 13), (130, 200, 64), (257, 129, 100), (64, 64, 16)]
+# d % 4 == 0 (4-byte inputs) takes the 128 x 128 kernel (d = 4: tail slice only;
+# d = 20, 36, 100: full slices + tail); other d the 64 x 64 one
+SHAPES = [(1, 1, 1), (2, 3, 3), (70, 33, 13), (130, 200, 64), (257, 129, 100), (64, 64, 16), (5, 300, 4),
+          (129, 257, 20), (300, 130, 36), (256, 384, 32)]
 
 
 @pytest.fixture(scope="module", params=[1, 3])

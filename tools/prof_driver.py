@@ -55,6 +55,14 @@ def main(which: str, reps: int = 3):
         s = sm(mult(a, b))
         for _ in range(reps):
             sm(mult(a, b), out=s)   # fused Zip -> Reduce (one kernel)
+    elif which in ("allpairs_dot", "allpairs_manhattan"):
+        d = 4096 if which == "allpairs_dot" else 128
+        ap = S.Allpairs(ctx, A.MULT if which == "allpairs_dot" else A.ABSDIFF, S.F32, S.F32, reduce=A.ADD)
+        a = S.Matrix.from_numpy(ctx, I.uniform_f32(81, 4096 * d).reshape(4096, d)).set_distribution(S.BLOCK)
+        b = S.Matrix.from_numpy(ctx, I.uniform_f32(82, 4096 * d).reshape(4096, d)).set_distribution(S.COPY)
+        c = ap(a, b)
+        for _ in range(reps):
+            ap(a, b, out=c)
     elif which == "lmosem":
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
