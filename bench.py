@@ -500,6 +500,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                          "ms": round(ms, 4), "pairs_per_s": nn * mm / (ms / 1e3),
                          "roofline": {"bound": "alu", "achieved": flops / (ms / 1e3) / 1e12, "peak": peak / 1e12,
                                       "unit": "TFLOP/s", "frac": flops / (ms / 1e3) / peak,
+                                      "traffic": ncu_traffic(name),
                                       "note": f"{ops} fp32 ops per (i,j,k), no FMA (-fmad=false)"},
                          "check": "ok" if ok else "FAIL"}
             for x in (ma, mb, c):
