@@ -371,7 +371,11 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                 bpp, okind = 2, O.OS_SOBEL
             else:
                 img = I.image_f32(I.SEED_GAUSS, R, C)
+                # 128-thread blocks (8 rows x 4 columns per thread, <= 128 registers):
+                # the fastest swept configuration (profiles/sweeps/sweep16-17)
+                ctx.set_option("block_threads", 128)
                 mo = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+                ctx.set_option("block_threads", 256)
                 bpp, okind = 8, O.OS_GAUSS5
             mi = S.Matrix.from_numpy(ctx, img)
             o = mo(mi)
@@ -392,6 +396,15 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                                      f"MapOverlap {R}x{C}, overlap distribution",
                          "ms": round(ms, 4), "elements_per_s": R * C / (ms / 1e3),
                          "roofline": roof_hbm(bpp * R * C, ms, P, name), "check": "ok" if ok else "FAIL"}
+            if name == "gauss":
+                # the binding roof: 25 FMUL + 25 FADD per pixel (no FMA under -fmad=false)
+                import torch as _t
+                sms = _t.cuda.get_device_properties(D.local).multi_processor_count
+                peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
+                fl = 50.0 * R * C / (ms / 1e3)
+                res[name]["roofline_alu"] = {"bound": "alu", "achieved": fl / 1e12, "peak": peak / 1e12,
+                                             "unit": "TFLOP/s", "frac": fl / peak,
+                                             "note": "50 fp32 ops/pixel (25 mul + 25 add)"}
             mi.destroy()
             o.destroy()
 

@@ -36,12 +36,32 @@ __device__ __forceinline__ long skl_clampl(long v, long lo, long hi) {
   return v < lo ? lo : (v > hi ? hi : v);
 }
 
+union SklMoRes {
+  SKL_TOUT e[SKL_CW];
+  typename SklRaw<SKL_OUTB>::type raw;
+};
+// store one thread's SKL_CW outputs of a row at o (ncols columns remain in the row)
+__device__ __forceinline__ void skl_mo_store(SKL_TOUT* o, const SklMoRes& v, bool full, long ncols) {
+#if SKL_OUT_PACK
+  if (full) {
+    *(typename SklRaw<SKL_OUTB>::type*)o = v.raw;
+    return;
+  }
+#endif
+#pragma unroll
+  for (int j = 0; j < SKL_CW; ++j)
+    if (j < ncols) o[j] = v.e[j];
+}
+
 #if !SKL_MO1D
 // ------------------------------------------------------------------ 2-D
 #define SKL_SROWS (SKL_TH + 2 * SKL_D)
 #define SKL_CPR (SKL_PITCH / SKL_EPC)  // 16-byte chunks per smem row
 
-extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+#ifndef SKL_MO_MINB
+#define SKL_MO_MINB 1
+#endif
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
 skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
          long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
          SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
@@ -49,6 +69,27 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
   const long r0 = r_begin + (long)blockIdx.y * SKL_TH;
   const long c0 = (long)blockIdx.x * SKL_TW;
   // ---- stage rows r0-d .. r0+TH+d-1, columns c0-A .. c0+TW+A-1
+  const bool interior = vec_ok && c0 - SKL_A >= 0 && c0 + SKL_TW + SKL_A <= C && r0 - SKL_D >= 0 &&
+                        r0 + SKL_TH + SKL_D <= R && r0 + SKL_TH <= r_end;
+  if (interior) {
+    // block-uniform fast path: every staged chunk is an in-range 16-byte copy;
+    // incremental (row, chunk) walk, no per-chunk bounds or boundary logic
+    const SKL_TIN* src = in + (r0 - SKL_D - in_row0) * C + (c0 - SKL_A);
+    const unsigned sbase = (unsigned)__cvta_generic_to_shared(tile);
+    int i = threadIdx.x / SKL_CPR, jc = threadIdx.x % SKL_CPR;
+#pragma unroll 4
+    for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
+      const unsigned sa = sbase + (unsigned)((i * SKL_PITCH + jc * SKL_EPC) * (int)sizeof(SKL_TIN));
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa),
+                   "l"(src + (long)i * C + jc * SKL_EPC) : "memory");
+      i += SKL_BLOCK / SKL_CPR;
+      jc += SKL_BLOCK % SKL_CPR;
+      if (jc >= SKL_CPR) {
+        jc -= SKL_CPR;
+        ++i;
+      }
+    }
+  } else
   for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
     const int i = q / SKL_CPR, jc = q - i * SKL_CPR;
     long gr = r0 - SKL_D + i;
@@ -90,39 +131,37 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
   // ---- apply f to a SKL_RH x SKL_CW block per thread
   const int ty = threadIdx.x / (SKL_TW / SKL_CW), tx = threadIdx.x % (SKL_TW / SKL_CW);
   const long cc = c0 + (long)tx * SKL_CW;
+  const bool full = vec_ok && cc + SKL_CW <= C;  // whole packed store in range
+  // fused halo push: the first / last hd rows of this device's
+  // block also go into the neighbours' halo rows (peer memory), so the next
+  // overlap read needs no exchange.  Block-uniform; the common path below
+  // carries none of it (live registers matter: f may call the IEEE sqrt
+  // subroutine).
+  if ((push_up && r0 < r_begin + hd) || (push_down && r0 + SKL_TH > r_end - hd)) {
+#pragma unroll
+    for (int i = 0; i < SKL_RH; ++i) {
+      const long r = r0 + (long)ty * SKL_RH + i;
+      const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
+      SklMoRes res;
+#pragma unroll
+      for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
+      if (r >= r_end) continue;
+      skl_mo_store(out + (r - out_row0) * C + cc, res, full, C - cc);
+      if (push_up && r < r_begin + hd) skl_mo_store(push_up + (r - r_begin) * C + cc, res, full, C - cc);
+      if (push_down && r >= r_end - hd)
+        skl_mo_store(push_down + (r - (r_end - hd)) * C + cc, res, full, C - cc);
+    }
+    return;
+  }
 #pragma unroll
   for (int i = 0; i < SKL_RH; ++i) {
     const long r = r0 + (long)ty * SKL_RH + i;
     const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
-    union {
-      SKL_TOUT e[SKL_CW];
-      typename SklRaw<SKL_OUTB>::type raw;
-    } res;
+    SklMoRes res;
 #pragma unroll
     // f may declare a non-const pointer (Listing 1.2: "float func(float* m_in)")
     for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
-    if (r < r_end) {
-      // fused halo push: the first / last hd rows of this device's block are
-      // also stored into the neighbours' halo rows (peer memory), so the next
-      // overlap read needs no exchange
-      SKL_TOUT* dst[3] = {out + (r - out_row0) * C + cc, nullptr, nullptr};
-      if (push_up && r < r_begin + hd) dst[1] = push_up + (r - r_begin) * C + cc;
-      if (push_down && r >= r_end - hd) dst[2] = push_down + (r - (r_end - hd)) * C + cc;
-#pragma unroll
-      for (int k = 0; k < 3; ++k) {
-        SKL_TOUT* o = dst[k];
-        if (!o) continue;
-#if SKL_OUT_PACK
-        if (cc + SKL_CW <= C && vec_ok) {
-          *(typename SklRaw<SKL_OUTB>::type*)o = res.raw;
-          continue;
-        }
-#endif
-#pragma unroll
-        for (int j = 0; j < SKL_CW; ++j)
-          if (cc + j < C) o[j] = res.e[j];
-      }
-    }
+    if (r < r_end) skl_mo_store(out + (r - out_row0) * C + cc, res, full, C - cc);
   }
   (void)in_rows;
 }

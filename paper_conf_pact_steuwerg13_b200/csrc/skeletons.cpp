@@ -165,11 +165,12 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       const int epc = (int)(16 / si);
       const int A = (int)ceil_div((size_t)d, (size_t)epc) * epc;
       int cw, rh, tw, th;
-      // default register block: one 16-byte-wide run of outputs per row, 2 rows
-      // (swept on B200, tools/sweep.py mo: Gaussian f32 0.224 -> 0.182 ms,
-      // Sobel u8 0.092 -> 0.088 ms at 256 threads)
+      // default register block: one 16-byte-wide run of outputs per row; 2 rows
+      // for byte images, 8 rows for wider elements (swept on B200, tools/sweep.py
+      // mo, profiles/sweeps/sweep15-17: Sobel u8 0.090 ms at 2 rows / 64
+      // registers; Gaussian f32 0.19 -> 0.146-0.159 ms at 8 rows / <= 128 registers)
       cw = (int)(16 / std::min<size_t>(so, 16) > 0 ? 16 / std::min<size_t>(so, 16) : 1);
-      rh = 2;
+      rh = si >= 4 ? 8 : 2;
       if (ctx->mo_cw > 0) cw = ctx->mo_cw;  // register block per thread (tuning knobs)
       if (ctx->mo_rh > 0) rh = ctx->mo_rh;
       if ((cw * (int)si) % 16 != 0 && (16 % (cw * (int)si)) != 0)
@@ -194,6 +195,11 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       defs += "#define SKL_CW " + std::to_string(cw) + "\n#define SKL_RH " + std::to_string(rh) + "\n";
       defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n";
       defs += "#define SKL_MO1D 0\n";
+      // resident blocks per SM the register allocation must allow (default: 64
+      // registers per thread for byte images - 87 registers halved the Sobel
+      // occupancy and cost 30 % - and 128 for wider elements)
+      const int minb = ctx->mo_minb > 0 ? ctx->mo_minb : std::max(1, 65536 / (nthr * (si >= 4 ? 128 : 64)));
+      defs += "#define SKL_MO_MINB " + std::to_string(minb) + "\n";
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;

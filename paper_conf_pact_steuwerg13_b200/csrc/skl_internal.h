@@ -119,6 +119,7 @@ struct Ctx {
   int scan_minb_pipe = 2;      // Scan pipelined kernel: min resident blocks
   int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
+  int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
   int ap_fast = 1;             // Allpairs zip-reduce: 128 x 128 tiles (4-byte inputs, d % 4 == 0)           // MapOverlap stores its border rows into the neighbours' halos
