@@ -219,7 +219,10 @@ void skel_destroy(Skel* s) {
   // deferred results of this skeleton must exist before it goes away
   for (Cont* c : std::vector<Cont*>(ctx->conts.begin(), ctx->conts.end()))
     if (c->lazy.s == s) materialize(c);
-  for (Skel* k : ctx->skels) k->fused.erase(s);
+  for (Skel* k : ctx->skels) {
+    k->fused.erase(s);
+    k->composed.erase(s);
+  }
   for (auto* m : {&s->scratch_red, &s->scratch_scan, &s->scratch_stage})
     for (auto& kv : *m)
       if (kv.second.ptr && ctx->is_local(kv.first)) device_free(ctx, kv.first, kv.second.ptr);
@@ -299,6 +302,36 @@ void finish_extras(Ctx* ctx, ExtraArgs& ea, int ndev_exec) {
 }  // namespace
 
 // ------------------------------------------------------------------ Map / Zip
+// Lazy fusion of chains: a Map g applied to the deferred
+// result of a Map/Zip f becomes one elementwise skeleton computing g(f(x[, y]))
+// (both sources renamed by macros: both may be called `func`).  Compiled once
+// per (g, f) pair; nullptr if it cannot be composed (types differ, or the two
+// sources clash), and the call then runs eagerly.
+static Skel* composed_skel(Skel* g, Skel* f) {
+  auto it = g->composed.find(f);
+  if (it != g->composed.end()) return it->second;
+  Ctx* ctx = g->ctx;
+  Skel* c = nullptr;
+  if (g->kind == K_MAP && g->extra.empty() && f->extra.empty() && g->tin == f->tout &&
+      (f->kind == K_MAP || f->kind == K_ZIP) && f->tout != SKL_VOID && g->tout != SKL_VOID) {
+    const std::string id = "skl_c" + std::to_string(++ctx->composed_id);
+    const bool zip = f->kind == K_ZIP;
+    std::string src = "#define " + f->entry + " " + id + "_f\n" + f->user_src + "\n#undef " + f->entry + "\n";
+    src += "#define " + g->entry + " " + id + "_g\n" + g->user_src + "\n#undef " + g->entry + "\n";
+    src += tname(ctx, g->tout) + " " + id + "(" + tname(ctx, f->tin) + " x" +
+           (zip ? ", " + tname(ctx, f->tin2) + " y" : std::string()) + ") { return " + id + "_g(" + id +
+           "_f(x" + (zip ? ", y" : "") + ")); }\n";
+    try {
+      c = skel_create(ctx, f->kind, src.c_str(), id.c_str(), f->tin, f->tin2, g->tout, nullptr, 0, 0, 0,
+                      nullptr);
+    } catch (const Error&) {
+      c = nullptr;  // e.g. a helper function defined in both sources
+    }
+  }
+  g->composed[f] = c;
+  return c;
+}
+
 static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_arg* extra,
                             int nextra) {
   Ctx* ctx = s->ctx;
@@ -308,6 +341,24 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     if (in2->elt != ctx->type(s->tin2).size) fail(SKL_ERR_TYPE, "right input type mismatch");
     if (in2->rows * in2->cols != in->rows * in->cols || in2->rows != in->rows)
       fail(SKL_ERR_SIZE_MISMATCH, "zip inputs differ in size (P:L257-259)");
+  }
+  if (!in2 && nextra == 0 && in->lazy.s && ctx->lazy_fusion && s->kind == K_MAP) {
+    if (Skel* c = composed_skel(s, in->lazy.s)) {
+      const Lazy L = in->lazy;
+      if (*out == nullptr) {
+        // stays deferred: g(f(...)) of f's inputs
+        Cont* o = cont_create(ctx, s->tout, in->rows, in->cols, in->matrix);
+        o->lazy = Lazy{c, L.l, L.r, L.d};
+        o->dist = L.d;
+        L.l->dependents.push_back(o);
+        if (L.r && L.r != L.l) L.r->dependents.push_back(o);
+        *out = o;
+        return;
+      }
+      // an explicit output: one kernel from f's inputs, no intermediate
+      run_elementwise(c, L.l, L.r, out, nullptr, 0);
+      return;
+    }
   }
   const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));  // A6
   ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);

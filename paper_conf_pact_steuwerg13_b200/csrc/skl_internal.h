@@ -133,6 +133,7 @@ struct Ctx {
   int scan_variant = 6;
   // counters
   std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0};
+  int composed_id = 0;  // names of composed Map chains (lazy fusion)
   // NVRTC cache: source hash -> program
   std::map<std::string, std::unique_ptr<Program>> programs;
   // builtin kernels (fill) per element size
@@ -264,6 +265,7 @@ struct Skel {
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
   std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
+  std::map<Skel*, Skel*> composed;  // Map g: g∘f per producing Zip/Map f (nullptr: not composable)
 };
 Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int tin, int tin2,
                   int tout, const int* extra, int nextra, int d, int boundary, const void* neutral);
