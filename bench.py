@@ -3,7 +3,7 @@
 task statement; DESIGN.md §"Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,sobel,gauss,scan_i32,scan_f32,lmosem]
+                    [--skeletons all|none|dot,sobel,gauss,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
 block-distributed Matrix<float2> of pixel coordinates (MAX_ITER 1000, window
@@ -570,6 +570,38 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                          "rel_l2_c_sample": e, "check": "ok" if e <= 1e-4 else "FAIL"}
         for x in (ev, f, c, fn, evs):
             x.destroy()
+
+    if "lmosem_osem" in which:
+        # one pass over 10 subsets of the same 10^7 events; f
+        # block->copy and c copy(+)->block at every subset (lmosem.py)
+        from paper_conf_pact_steuwerg13_b200.lmosem import ListModeOSEM
+        N, nev, nsub = 150, 10_000_000, 10
+        events = I.lmosem_events(I.SEED_LMOSEM, nev, N)
+        osem = ListModeOSEM(ctx, N)
+        osem.load_events(events, nsub)
+        f0 = np.ones(N ** 3, np.float32)
+        osem.set_image(f0)
+
+        def step(_):
+            osem.iterate(1)
+
+        ms, _ = timer.run(step, max(3, K // 4), 2, D)
+        ms = D.max(ms)
+        # parity: the same program on every 100th event (10 subsets) vs the oracle
+        sub = events[::100].copy()
+        osem.load_events(sub, nsub)
+        osem.set_image(f0)
+        osem.iterate(1)
+        fo = f0.copy()
+        for lo, hi in ListModeOSEM.subset_bounds(sub.shape[0], nsub):
+            fo = O.lmosem(sub[lo:hi], N, fo)[1].astype(np.float32)
+        fg = osem.image().astype(np.float64)
+        e = float(np.linalg.norm(fg - fo) / np.linalg.norm(fo))
+        res["lmosem_osem"] = {"workload": f"LM OSEM pass: {nsub} subsets x 10^6 events, 150^3 image; per subset "
+                                          "f block->copy, Map (block events), c copy(+)->block, Zip f*c",
+                              "ms": round(ms, 4), "events_per_s": nev / (ms / 1e3),
+                              "rel_l2_f_sample": e, "check": "ok" if e <= 1e-4 else "FAIL"}
+        osem.destroy()
     ctx.finalize()
     return res
 
@@ -620,7 +652,8 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, D, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "sobel", "gauss", "scan_i32", "scan_f32", "lmosem", "allpairs"] if args.skeletons == "all"
+        ["dot", "sobel", "gauss", "scan_i32", "scan_f32", "lmosem", "lmosem_osem", "allpairs"]
+        if args.skeletons == "all"
         else args.skeletons.split(","))
     sk = bench_skeletons(args, D, P, which) if which else {}
     if D.rank != 0:
