@@ -219,13 +219,17 @@ def bench_mandelbrot(args, D: Dist, P: dict):
     from paper_conf_pact_steuwerg13_b200 import skl as S
     ctx, g = make_context(D)
     # user-side tuning (the paper's optional work-group size):
-    # 512-thread blocks, 2 chunks per thread; the customising function checks the
-    # escape once per 4 iterations and replays the block (bit-identical counts)
-    ctx.set_option("block_threads", 512)
-    ctx.set_option("map_unroll", 2)
-    m = S.Map(ctx, A.mandelbrot_unrolled(MAX_ITER), S.F32X2, S.U32)
+    # 1024-thread blocks, one 4-pixel chunk per thread, warp-interleaved pixels
+    # (lanes of a warp iterate neighbouring pixels: less idle-lane time); the
+    # customising function checks the escape once per 8 iterations and replays
+    # the block (bit-identical counts).  Swept: profiles/sweeps/sweep18-19.
+    ctx.set_option("block_threads", 1024)
+    ctx.set_option("map_unroll", 1)
+    ctx.set_option("map_interleave", 1)
+    m = S.Map(ctx, A.mandelbrot_unrolled(MAX_ITER, 8), S.F32X2, S.U32)
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
+    ctx.set_option("map_interleave", 0)
     grid = I.mandel_grid(ROWS, COLS)
     cin = S.Matrix(ctx, S.F32X2, ROWS, COLS).set_distribution(S.BLOCK)
     cin.copy_in(grid)

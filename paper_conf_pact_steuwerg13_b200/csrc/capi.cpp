@@ -194,6 +194,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       (k == "mo_rh" ? c->mo_rh : c->mo_cw) = (int)value;
     } else if (k == "lazy_fusion") {
       c->lazy_fusion = value ? 1 : 0;
+    } else if (k == "map_interleave") {
+      c->map_interleave = value ? 1 : 0;
     } else if (k == "ap_fast") {
       c->ap_fast = value ? 1 : 0;
     } else if (k == "halo_push") {

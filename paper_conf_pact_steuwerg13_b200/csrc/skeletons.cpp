@@ -83,6 +83,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
   // launch geometry is fixed at creation (compiled into the program)
   s->block = ctx->block_threads;
   s->unroll = ctx->map_unroll;
+  s->interleave = ctx->map_interleave != 0;
   std::string defs = defs_common(ctx, s->entry, s->block);
   std::string body;
   switch (kind) {
@@ -415,7 +416,10 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     }
     size_t grid;
     const char* kname;
-    if (vec_ok) {
+    if (s->interleave) {
+      grid = std::max<size_t>(1, ceil_div(n, per_block * vec));
+      kname = "skl_map_il";
+    } else if (vec_ok) {
       grid = std::max<size_t>(1, ceil_div(n / vec, per_block));
       kname = "skl_map_vec";
     } else {

@@ -122,6 +122,7 @@ struct Ctx {
   int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
+  int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
   int ap_fast = 1;             // Allpairs zip-reduce: 128 x 128 tiles (4-byte inputs, d % 4 == 0)           // MapOverlap stores its border rows into the neighbours' halos
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 6 = one block per tile, tile kept in shared memory, low
@@ -264,6 +265,7 @@ struct Skel {
   bool ap_zr = false;     // Allpairs: zip-reduce form
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
+  bool interleave = false;  // Map/Zip: launch the warp-interleaved kernel
   std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
   std::map<Skel*, Skel*> composed;  // Map g: g∘f per producing Zip/Map f (nullptr: not composable)
 };

@@ -21,9 +21,10 @@ def main(which: str, reps: int = 3):
     ctx = S.Context(1)
     if which == "mandel":
         # the bench's configuration
-        ctx.set_option("block_threads", 512)
-        ctx.set_option("map_unroll", 2)
-        m = S.Map(ctx, A.mandelbrot_unrolled(1000), S.F32X2, S.U32)
+        ctx.set_option("block_threads", 1024)
+        ctx.set_option("map_unroll", 1)
+        ctx.set_option("map_interleave", 1)
+        m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
         x = S.Matrix(ctx, S.F32X2, 3072, 4096).copy_in(I.mandel_grid(3072, 4096))
         o = m(x)
         for _ in range(reps):

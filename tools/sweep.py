@@ -51,23 +51,25 @@ def timeit(fn, reps=10, warm=3):
 
 
 def mandel():
+    """MANDEL_CFGS="fn,block,unroll,interleave;..." (fn: plain | unroll4)"""
     grid = I.mandel_grid(3072, 4096)
     ref = None
-    for name, src in (("plain", A.mandelbrot(1000)), ("unroll4", A.mandelbrot_unrolled(1000))):
-        for bt in (128, 256, 512):
-            for un in (1, 2, 4):
-                c = ctx_with({"block_threads": bt, "map_unroll": un})
-                m = S.Map(c, src, S.F32X2, S.U32)
-                x = S.Matrix(c, S.F32X2, 3072, 4096).copy_in(grid)
-                o = m(x)
-                ms = timeit(lambda: m(x, out=o))
-                out = o.to_numpy()
-                if ref is None:
-                    ref, tot = O.mandelbrot(grid, 1000)
-                ok = np.array_equal(out, ref)
-                print(f"mandel {name:8s} block={bt:4d} unroll={un}: {ms:.4f} ms  "
-                      f"{8 * tot / (ms / 1e3) / 1e12:.2f} TFLOP/s  bitexact={ok}", flush=True)
-                c.finalize()
+    cfgs = [t.split(",") for t in os.environ.get("MANDEL_CFGS", "unroll4,512,2,0").split(";")]
+    for name, bt, un, il in cfgs:
+        bt, un, il = int(bt), int(un), int(il)
+        src = A.mandelbrot(1000) if name == "plain" else A.mandelbrot_unrolled(1000, int(name[6:] or 4))
+        c = ctx_with({"block_threads": bt, "map_unroll": un, "map_interleave": il})
+        m = S.Map(c, src, S.F32X2, S.U32)
+        x = S.Matrix(c, S.F32X2, 3072, 4096).copy_in(grid)
+        o = m(x)
+        ms = timeit(lambda: m(x, out=o))
+        out = o.to_numpy()
+        if ref is None:
+            ref, tot = O.mandelbrot(grid, 1000)
+        ok = np.array_equal(out, ref)
+        print(f"mandel {name:8s} block={bt:4d} unroll={un} interleave={il}: {ms:.4f} ms  "
+              f"{8 * tot / (ms / 1e3) / 1e12:.2f} TFLOP/s  bitexact={ok}", flush=True)
+        c.finalize()
 
 
 def lmosem():
