@@ -188,7 +188,7 @@ class Timer:
         self.flush.zero_()
         self.sink.copy_(self.sweep.sum())
 
-    def run(self, step, K: int, W: int, D: Dist, marks: int = 0):
+    def run(self, step, K: int, W: int, D: Dist, marks: int = 0, flush: bool = True):
         torch = self.torch
         for _ in range(W):
             step(None)
@@ -197,7 +197,8 @@ class Timer:
         torch.cuda.synchronize()
         evs = []
         for _ in range(K):
-            self.flush_l2()
+            if flush:
+                self.flush_l2()
             e = [torch.cuda.Event(enable_timing=True) for _ in range(2 + marks)]
             e[0].record()
             step(e[1:-1] if marks else None)
@@ -273,14 +274,36 @@ def bench_mandelbrot(args, D: Dist, P: dict):
                      "h2d_bytes_per_step": int(h2d), "d2h_bytes_per_step": int(d2h)})
 
 
+def cpu_info() -> dict:
+    """host CPU of this box (record nproc and the model)"""
+    model = "unknown"
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                model = line.split(":", 1)[1].strip()
+                break
+    except OSError:
+        pass
+    return {"cpu_model": model, "nproc": os.cpu_count()}
+
+
 def mandel_oracle(sample_every: int = 1):
     """CPU oracle on rows 0, s, 2s, ... (bounded sample); returns counts, sum iters, seconds"""
     import oracle as O
     from paper_conf_pact_steuwerg13_b200 import inputs as I
     grid = I.mandel_grid(ROWS, COLS)[::sample_every].copy()
-    t0 = time.perf_counter()
-    counts, tot = O.mandelbrot(grid, MAX_ITER)
-    return counts, tot, time.perf_counter() - t0
+    # one thread pinned to one core (SURVEY 8(d)), the affinity restored afterwards
+    allowed = os.sched_getaffinity(0) if hasattr(os, "sched_getaffinity") else None
+    if allowed:
+        os.sched_setaffinity(0, {min(allowed)})
+    try:
+        t0 = time.perf_counter()
+        counts, tot = O.mandelbrot(grid, MAX_ITER)
+        sec = time.perf_counter() - t0
+    finally:
+        if allowed:
+            os.sched_setaffinity(0, allowed)
+    return counts, tot, sec
 
 
 # ---------------------------------------------------------------- per-skeleton lines
@@ -329,11 +352,14 @@ def bench_skeletons(args, D: Dist, P: dict, which):
 
             ms_eager, _ = timer.run(step, K, W, D)
             ms_eager = D.max(ms_eager)
+            ms_warm = None
             # the same step recorded once as a CUDA graph and replayed (removes the
             # host enqueue time that dominates at 2^20 elements)
             graph = ctx.capture(lambda: step(None)) if D.world == 1 else None
             if graph is not None:
                 ms, _ = timer.run(lambda _: graph.launch(), K, W, D)
+                if n == 1 << 20:   # 8 MiB fits L2: also the warm number (no flush)
+                    ms_warm, _ = timer.run(lambda _: graph.launch(), K, W, D, flush=False)
             else:
                 ms = ms_eager
             # the same composition with the intermediate materialised (Zip then Reduce)
@@ -355,6 +381,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                                     "Zip fused into Reduce (lazy)",
                         "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3),
                         "ms_without_graph": round(ms_eager, 4), "cuda_graph": graph is not None,
+                        "ms_warm_l2": round(ms_warm, 4) if ms_warm else None,
                         "roofline": roof_hbm(8 * n, ms, P, "dot_2^28_fused" if n == 1 << 28 else None),
                         "unfused": {"ms": round(ms_u, 4), "zip_ms": round(seg[0], 4), "reduce_ms": round(seg[1], 4),
                                     "roofline_zip": roof_hbm(12 * n, seg[0], P), "roofline_reduce": roof_hbm(4 * n, seg[1], P)},
@@ -363,6 +390,68 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                 graph.destroy()
             for x in (va, vb, c):
                 x.destroy()
+
+    if "dot_sweep" in which:
+        # the fused dot product from 2^20 to 2^30 elements
+        # (cold L2), where the HBM gate applies at the large end; inputs filled on
+        # the device (a = 1, b = 2^-10: every partial sum is exact in fp32)
+        mult, sm = S.Zip(ctx, A.MULT, S.F32, S.F32, S.F32), S.Reduce(ctx, A.SUM, S.F32)
+        sweep = {}
+        for lg in (20, 22, 24, 26, 28, 30):
+            n = 1 << lg
+            va = S.Vector(ctx, S.F32, n).set_distribution(S.BLOCK).fill(1.0)
+            vb = S.Vector(ctx, S.F32, n).set_distribution(S.BLOCK).fill(2.0 ** -10)
+            s = sm(mult(va, vb))
+
+            def step(_):
+                sm(mult(va, vb), out=s)
+
+            ms, _ = timer.run(step, max(3, K // 2), W, D)
+            ms = D.max(ms)
+            ok = float(s.scalar()) == n * 2.0 ** -10
+            gbs = 8 * n / (ms / 1e3) / 1e9
+            sweep[f"2^{lg}"] = {"ms": round(ms, 4), "GB_s": round(gbs, 1), "frac": round(gbs / P["hbm_gbs"], 4),
+                                "check": "ok" if ok else "FAIL"}
+            va.destroy()
+            vb.destroy()
+        res["dot_sweep"] = {"workload": "fused sum(mult(A,B)) sweep 2^20..2^30 fp32 (no graph), cold L2, "
+                                        "8 B/element", "points": sweep,
+                            "check": "ok" if all(v["check"] == "ok" for v in sweep.values()) else "FAIL"}
+
+    if "gauss_iter" in which:
+        # K=10 iterated Gaussian (ping-pong); on several GPUs the halo
+        # rows move between iterations (NCCL, one process per GPU)
+        R = C = 8192
+        img = I.image_f32(I.SEED_GAUSS, R, C)
+        ctx.set_option("block_threads", 128)
+        gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+        ctx.set_option("block_threads", 256)
+        a = S.Matrix.from_numpy(ctx, img)
+        b = S.Matrix(ctx, S.F32, R, C)
+        t = S.Matrix(ctx, S.F32, R, C)
+        ITER = 10
+
+        def step(_):
+            gau(a, out=b)
+            for k in range(ITER - 1):
+                gau(b, out=t) if k % 2 == 0 else gau(t, out=b)
+
+        ms, _ = timer.run(step, max(3, K // 4), W, D)
+        ms = D.max(ms)
+        # parity: rows 4000..4063 after 10 iterations (the oracle iterates a band wide
+        # enough that its edges do not reach the checked rows: 10 x d = 20 rows)
+        sub = img[3970:4094]
+        r = sub
+        for _ in range(ITER):
+            r = O.mapoverlap2d(O.OS_GAUSS5, r, 2, O.OB_NEAREST, 0.0)
+        fin = (t if (ITER - 1) % 2 == 1 else b)
+        ok = bool(np.array_equal(fin.to_numpy()[4000:4064], r[30:94]))
+        res["gauss_iter10"] = {"workload": f"10 x Gaussian 5x5 f32 MapOverlap {R}x{C}, ping-pong (halo refresh "
+                                           "between iterations on >1 GPU)",
+                               "ms": round(ms, 4), "ms_per_iteration": round(ms / ITER, 4),
+                               "elements_per_s": ITER * R * C / (ms / 1e3), "check": "ok" if ok else "FAIL"}
+        for x in (a, b, t):
+            x.destroy()
 
     if "sobel" in which or "gauss" in which:
         R = C = 8192
@@ -629,7 +718,7 @@ def run_reference(args, D: Dist):
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": sec * 1e3, "higher_is_better": True,
             "scaling": "strong", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
             "config": {"workload": f"mandelbrot {COLS}x{ROWS} Map, MAX_ITER={MAX_ITER} (oracle on every {every}th row)"},
-            "cpu_baseline": {"value": v, "unit": "elements/s", "cores": 1, "kind": "oracle",
+            "cpu_baseline": {"value": v, "unit": "elements/s", "cores": 1, "kind": "oracle", **cpu_info(),
                              "sample": f"rows 0,{every},{2 * every},... ({pix} pixels) per step"},
             "e2e": {"value": v, "unit": "elements/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
@@ -656,7 +745,8 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, D, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "sobel", "gauss", "scan_i32", "scan_f32", "lmosem", "lmosem_osem", "allpairs"]
+        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "scan_i32", "scan_f32", "lmosem", "lmosem_osem",
+         "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
     sk = bench_skeletons(args, D, P, which) if which else {}
@@ -687,7 +777,7 @@ def main():
                      "frac": achieved / alu_peak, "traffic": ncu_traffic("mandelbrot"),
                      "note": f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count); peak = {sms} SMs x 128 "
                              f"FP32 lanes x {P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false)"},
-        "cpu_baseline": {"value": ROWS * COLS / cpu_s, "unit": "elements/s", "cores": 1, "kind": "oracle",
+        "cpu_baseline": {"value": ROWS * COLS / cpu_s, "unit": "elements/s", "cores": 1, "kind": "oracle", **cpu_info(),
                          "sample": f"whole {COLS}x{ROWS} image, single thread ({cpu_s:.2f} s)"},
         "e2e": r["e2e"], "gpu_launches": int(r["launches"]), "clocks": r["clocks"],
         "parity": {"mandelbrot_full_image_bitexact": parity, "sum_iterations": int(sum_iter)},

@@ -104,6 +104,17 @@ skl_status skl_num_devices(skl_ctx* ctx, int* ndev, int* first_local, int* nloca
 skl_status skl_set_stream(skl_ctx* ctx, int g, void* cuda_stream);
 skl_status skl_get_stream(skl_ctx* ctx, int g, void** cuda_stream);
 skl_status skl_sync(skl_ctx* ctx);
+/* Device memory from the caller's allocator instead of the library's
+ * cudaMallocAsync pool (e.g. torch's caching allocator, so that
+ * PyTorch owns device memory).  alloc(bytes, cuda_device, cuda_stream, user)
+ * returns a device pointer usable in stream order on cuda_stream (NULL ->
+ * SKL_ERR_OOM); release(ptr, cuda_device, cuda_stream, user) returns it.  Every
+ * container part and skeleton scratch buffer goes through them.  Only before
+ * any container or skeleton exists (else SKL_ERR_INVALID_ARG); both NULL
+ * restores the default.                                                        */
+typedef void* (*skl_alloc_fn)(size_t bytes, int cuda_device, void* cuda_stream, void* user);
+typedef void (*skl_free_fn)(void* ptr, int cuda_device, void* cuda_stream, void* user);
+skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn release, void* user);
 /* Options: "block_threads" (work-group size; default 256),
  * "debug_bounds" (1 = get() range-checked, A21), "map_unroll" (chunks per
  * thread, default 4), "lazy_fusion" (1 = a Map/Zip without an output is

@@ -137,6 +137,17 @@ skl_status skl_set_stream(skl_ctx* ctx, int g, void* stream) {
     d.stream = ns;
   });
 }
+skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn release, void* user) {
+  return guard([&] {
+    Ctx* c = C(ctx);
+    if ((alloc == nullptr) != (release == nullptr)) fail(SKL_ERR_INVALID_ARG, "give both functions or neither");
+    if (!c->conts.empty() || !c->skels.empty())
+      fail(SKL_ERR_INVALID_ARG, "set the allocator before creating containers or skeletons");
+    c->user_alloc = alloc;
+    c->user_free = release;
+    c->alloc_user = user;
+  });
+}
 skl_status skl_get_stream(skl_ctx* ctx, int g, void** stream) {
   return guard([&] {
     Ctx* c = C(ctx);

@@ -179,12 +179,26 @@ void* device_alloc(Ctx* ctx, int g, size_t bytes) {
   if (bytes == 0) bytes = 16;
   ctx->set_device(g);
   void* p = nullptr;
+  if (ctx->user_alloc) {
+    // caller's allocator (e.g. torch's caching allocator), stream-ordered on
+    // this device's stream
+    p = ctx->user_alloc(bytes, ctx->D(g).phys, (void*)ctx->D(g).stream, ctx->alloc_user);
+    if (!p) fail(SKL_ERR_OOM, "user allocator returned NULL for " + std::to_string(bytes) + " bytes");
+    return p;
+  }
   SKL_CUDA(cudaMallocAsync(&p, bytes, ctx->D(g).stream));
   return p;
 }
 void device_free(Ctx* ctx, int g, void* p) {
   if (!p) return;
   ctx->set_device(g);
+  if (ctx->user_free) {
+    // the block may be reused at once on this stream: work other devices'
+    // streams queued on it (peer copies) must be ordered before that reuse
+    if (ctx->nlocal > 1) barrier_streams(ctx);
+    ctx->user_free(p, ctx->D(g).phys, (void*)ctx->D(g).stream, ctx->alloc_user);
+    return;
+  }
   SKL_CUDA(cudaFreeAsync(p, ctx->D(g).stream));
 }
 

@@ -135,6 +135,10 @@ struct Ctx {
   // counters
   std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0};
   int composed_id = 0;  // names of composed Map chains (lazy fusion)
+  // optional caller-provided device allocator (skl_set_allocator)
+  void* (*user_alloc)(size_t, int, void*, void*) = nullptr;
+  void (*user_free)(void*, int, void*, void*) = nullptr;
+  void* alloc_user = nullptr;
   // NVRTC cache: source hash -> program
   std::map<std::string, std::unique_ptr<Program>> programs;
   // builtin kernels (fill) per element size

@@ -67,6 +67,7 @@ def lib():
         "skl_nccl_unique_id": [vp], "skl_finalize": [vp],
         "skl_num_devices": [vp, C.POINTER(i), C.POINTER(i), C.POINTER(i)],
         "skl_set_stream": [vp, i, vp], "skl_get_stream": [vp, i, pp], "skl_sync": [vp],
+        "skl_set_allocator": [vp, vp, vp, vp],
         "skl_set_option": [vp, C.c_char_p, C.c_longlong],
         "skl_get_counter": [vp, C.c_char_p, C.POINTER(C.c_longlong)],
         "skl_type_struct": [vp, C.c_char_p, C.c_char_p, sz, sz, C.POINTER(i)],
@@ -116,6 +117,10 @@ def check(rc: int):
 
 def exported_symbols() -> list:
     return [n for n in dir(lib()) if n.startswith("skl_")]
+
+
+_ALLOC_FN = C.CFUNCTYPE(C.c_void_p, C.c_size_t, C.c_int, C.c_void_p, C.c_void_p)
+_FREE_FN = C.CFUNCTYPE(None, C.c_void_p, C.c_int, C.c_void_p, C.c_void_p)
 
 
 # ---------------------------------------------------------------- context
@@ -176,6 +181,25 @@ class Context:
 
     def sync(self):
         check(lib().skl_sync(self._h))
+
+    def use_torch_allocator(self):
+        """Route the library's device memory through torch's caching allocator
+        (skl_set_allocator; PyTorch as the device-memory plumbing).  Call before
+        creating containers or skeletons."""
+        import torch
+
+        def _alloc(nbytes, dev, stream, _user):
+            try:
+                return torch.cuda.caching_allocator_alloc(nbytes, dev, stream or 0)
+            except Exception:   # noqa: BLE001 - the library reports SKL_ERR_OOM
+                return None
+
+        def _free(ptr, _dev, _stream, _user):
+            torch.cuda.caching_allocator_delete(ptr)
+
+        self._alloc_cb = (_ALLOC_FN(_alloc), _FREE_FN(_free))   # kept alive with the context
+        check(lib().skl_set_allocator(self._h, C.cast(self._alloc_cb[0], C.c_void_p),
+                                      C.cast(self._alloc_cb[1], C.c_void_p), None))
 
     def set_option(self, key: str, value: int):
         check(lib().skl_set_option(self._h, key.encode(), value))
