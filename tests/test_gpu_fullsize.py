@@ -25,11 +25,14 @@ def ctx():
 
 
 def test_mandelbrot_full_image_bitexact(ctx):
-    ctx.set_option("block_threads", 512)
-    ctx.set_option("map_unroll", 2)
-    m = S.Map(ctx, A.mandelbrot_unrolled(1000), S.F32X2, S.U32)
+    # bench.py's configuration: 1024 threads, 1 chunk, warp-interleaved, 8-iteration blocks
+    ctx.set_option("block_threads", 1024)
+    ctx.set_option("map_unroll", 1)
+    ctx.set_option("map_interleave", 1)
+    m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
+    ctx.set_option("map_interleave", 0)
     grid = I.mandel_grid(3072, 4096)
     x = S.Matrix(ctx, S.F32X2, 3072, 4096).set_distribution(S.BLOCK)
     x.copy_in(grid)
@@ -57,7 +60,9 @@ def test_stencils_8192_bands(ctx, name):
         mo = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
     else:
         img = I.image_f32(I.SEED_GAUSS, R, C)
+        ctx.set_option("block_threads", 128)   # bench.py's Gaussian configuration
         mo = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+        ctx.set_option("block_threads", 256)
     out = mo(S.Matrix.from_numpy(ctx, img)).to_numpy()
     for r0 in (0, 4000, R - 64):  # top edge, interior, bottom edge
         lo, hi = max(0, r0 - 8), min(R, r0 + 72)
