@@ -115,7 +115,11 @@ class Dist:
         self.rank = int(os.environ.get("RANK", "0"))
         self.local = int(os.environ.get("LOCAL_RANK", "0"))
         self.pg = None
-        if self.world > 1:
+        # SKL_BENCH_FORCE_DIST=1: the one-process-per-GPU path (NCCL communicator,
+        # collective host reads, max over ranks) even at world size 1, so that it
+        # can be exercised on a single GPU
+        self.force = os.environ.get("SKL_BENCH_FORCE_DIST", "0") == "1"
+        if self.world > 1 or self.force:
             import torch
             import torch.distributed as dist
             torch.cuda.set_device(self.local)
@@ -154,7 +158,7 @@ def make_context(D: Dist):
     import torch
     from paper_conf_pact_steuwerg13_b200 import skl as S
     torch.cuda.set_device(D.local)
-    if D.world > 1:
+    if D.world > 1 or D.force:
         nid = S.Context.nccl_unique_id() if D.rank == 0 else b"\0" * 128
         nid = D.bcast_bytes(nid)
         ctx = S.Context.dist(D.rank, D.world, D.local, nid)
@@ -794,5 +798,17 @@ def S_block(n, G, g):
     return min(n, g * chunk), min(n, (g + 1) * chunk)
 
 
+def _main_and_shutdown():
+    try:
+        return main()
+    finally:
+        try:
+            import torch.distributed as dist
+            if dist.is_available() and dist.is_initialized():
+                dist.destroy_process_group()
+        except Exception:   # noqa: BLE001 - shutdown only
+            pass
+
+
 if __name__ == "__main__":
-    sys.exit(main())
+    sys.exit(_main_and_shutdown())
