@@ -34,18 +34,58 @@ class ListModeOSEM:
         self.subsets: list[S.Vector] = []
 
     @staticmethod
+    def path_order(events: np.ndarray, N: int) -> np.ndarray:
+        """A permutation of the events, longest ray walk first (application-level
+        load balancing; within a subset the order of events does not change the
+        result beyond fp32 atomic rounding).  The walk length is estimated on the
+        host in float64 from the ray's entry and exit voxels (the number of voxel
+        boundaries crossed + 1; 0 for rays that miss the volume).  Warps then hold
+        rays of similar length, so fewer lanes idle while the longest ray of the
+        warp finishes, and the block scheduler runs the long rays first."""
+        ev = np.asarray(events, dtype=np.float64)
+        p0, d = ev[:, 0:3], ev[:, 3:6] - ev[:, 0:3]
+        amin = np.zeros(len(ev))
+        amax = np.ones(len(ev))
+        hit = np.ones(len(ev), dtype=bool)
+        with np.errstate(divide="ignore", invalid="ignore"):
+            for a in range(3):
+                flat = d[:, a] == 0.0
+                hit &= ~(flat & ((p0[:, a] < 0.0) | (p0[:, a] > N)))
+                a0 = np.where(flat, -np.inf, (0.0 - p0[:, a]) / d[:, a])
+                aN = np.where(flat, np.inf, (N - p0[:, a]) / d[:, a])
+                amin = np.maximum(amin, np.minimum(a0, aN))
+                amax = np.minimum(amax, np.maximum(a0, aN))
+        hit &= amax > amin
+        top = np.nextafter(float(N), 0.0)
+        ent = np.clip(p0 + amin[:, None] * d, 0.0, top)
+        ext = np.clip(p0 + amax[:, None] * d, 0.0, top)
+        steps = np.abs(np.floor(ext) - np.floor(ent)).sum(axis=1) + 1.0
+        key = np.where(hit, steps, 0.0)
+        return np.argsort(-key, kind="stable")
+
+    @staticmethod
     def subset_bounds(nev: int, nsub: int):
         """contiguous slices [lo, hi) of the event stream, sizes differing by <= 1"""
         return [(nev * i // nsub, nev * (i + 1) // nsub) for i in range(nsub)]
 
-    def load_events(self, events: np.ndarray, nsub: int):
-        """upload the list-mode events once, one block-distributed Vector per subset"""
+    def load_events(self, events: np.ndarray, nsub: int, balance: bool = True):
+        """upload the list-mode events once, one block-distributed Vector per
+        subset (each subset's events ordered longest walk first if `balance`)"""
         for v in self.subsets:
             v.destroy()
         self.subsets = []
         for lo, hi in self.subset_bounds(events.shape[0], nsub):
+            sub = events[lo:hi]
+            if balance:
+                order = self.path_order(sub, self.N)
+                G = self.ctx.ndev
+                if G > 1:
+                    # deal the sorted rays round-robin so that every device's
+                    # block holds an equal share of long and short rays
+                    order = np.concatenate([order[g::G] for g in range(G)])
+                sub = sub[order]
             v = S.Vector(self.ctx, self.evd, hi - lo).set_distribution(S.BLOCK)
-            v.copy_in(np.ascontiguousarray(events[lo:hi]))
+            v.copy_in(np.ascontiguousarray(sub))
             self.subsets.append(v)
 
     def set_image(self, f0: np.ndarray):

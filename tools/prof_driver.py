@@ -70,7 +70,9 @@ def main(which: str, reps: int = 3):
         ctx.set_option("map_unroll", 1)
         lm = S.Map(ctx, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
         ev = S.Vector(ctx, evd, nev).set_distribution(S.BLOCK)
-        ev.copy_in(I.lmosem_events(7, nev, N))
+        from paper_conf_pact_steuwerg13_b200.lmosem import ListModeOSEM
+        events = I.lmosem_events(7, nev, N)
+        ev.copy_in(np.ascontiguousarray(events[ListModeOSEM.path_order(events, N)]))   # bench.py's order
         f = S.Vector(ctx, S.F32, N ** 3).set_distribution(S.COPY).fill(1.0)
         c = S.Vector(ctx, S.F32, N ** 3).set_distribution(S.COPY).fill(0.0)
         for _ in range(reps):
