@@ -43,7 +43,9 @@ def main(which: str, reps: int = 3):
             mo = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
             x = S.Matrix.from_numpy(ctx, I.image_u8(5, 8192, 8192))
         else:
+            ctx.set_option("block_threads", 128)   # bench.py's Gaussian configuration
             mo = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+            ctx.set_option("block_threads", 256)
             x = S.Matrix.from_numpy(ctx, I.image_f32(6, 8192, 8192))
         o = mo(x)
         for _ in range(reps):
