@@ -66,22 +66,26 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
          long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
          SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
   __shared__ __align__(16) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
-  const long r0 = r_begin + (long)blockIdx.y * SKL_TH;
-  const long c0 = (long)blockIdx.x * SKL_TW;
+  // 32-bit row / column arithmetic (the host guarantees R, C < 2^31); 64-bit
+  // only where a row index is scaled to an element offset
+  const int Ri = (int)R, Ci = (int)C, rb = (int)r_begin, re = (int)r_end;
+  const int irow0 = (int)in_row0, orow0 = (int)out_row0;
+  const int r0 = rb + (int)blockIdx.y * SKL_TH;
+  const int c0 = (int)blockIdx.x * SKL_TW;
   // ---- stage rows r0-d .. r0+TH+d-1, columns c0-A .. c0+TW+A-1
-  const bool interior = vec_ok && c0 - SKL_A >= 0 && c0 + SKL_TW + SKL_A <= C && r0 - SKL_D >= 0 &&
-                        r0 + SKL_TH + SKL_D <= R && r0 + SKL_TH <= r_end;
+  const bool interior = vec_ok && c0 - SKL_A >= 0 && c0 + SKL_TW + SKL_A <= Ci && r0 - SKL_D >= 0 &&
+                        r0 + SKL_TH + SKL_D <= Ri && r0 + SKL_TH <= re;
   if (interior) {
     // block-uniform fast path: every staged chunk is an in-range 16-byte copy;
     // incremental (row, chunk) walk, no per-chunk bounds or boundary logic
-    const SKL_TIN* src = in + (r0 - SKL_D - in_row0) * C + (c0 - SKL_A);
+    const SKL_TIN* src = in + (long)(r0 - SKL_D - irow0) * Ci + (c0 - SKL_A);
     const unsigned sbase = (unsigned)__cvta_generic_to_shared(tile);
     int i = threadIdx.x / SKL_CPR, jc = threadIdx.x % SKL_CPR;
 #pragma unroll 4
     for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
       const unsigned sa = sbase + (unsigned)((i * SKL_PITCH + jc * SKL_EPC) * (int)sizeof(SKL_TIN));
       asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa),
-                   "l"(src + (long)i * C + jc * SKL_EPC) : "memory");
+                   "l"(src + (long)i * Ci + jc * SKL_EPC) : "memory");
       i += SKL_BLOCK / SKL_CPR;
       jc += SKL_BLOCK % SKL_CPR;
       if (jc >= SKL_CPR) {
@@ -92,34 +96,33 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
   } else
   for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
     const int i = q / SKL_CPR, jc = q - i * SKL_CPR;
-    long gr = r0 - SKL_D + i;
-    const long gc0 = c0 - SKL_A + (long)jc * SKL_EPC;
-    const bool row_in = gr >= 0 && gr < R;
+    int gr = r0 - SKL_D + i;
+    const int gc0 = c0 - SKL_A + jc * SKL_EPC;
+    const bool row_in = gr >= 0 && gr < Ri;
 #if SKL_BOUNDARY == 1
-    gr = skl_clampl(gr, 0, R - 1);
+    gr = gr < 0 ? 0 : (gr > Ri - 1 ? Ri - 1 : gr);
 #endif
     SKL_TIN* dst = tile + i * SKL_PITCH + jc * SKL_EPC;
-    if (r0 - SKL_D + i >= r_end + SKL_D) {  // below the last output row's window: unused
+    if (r0 - SKL_D + i >= re + SKL_D) {  // below the last output row's window: unused
 #pragma unroll
       for (int e = 0; e < SKL_EPC; ++e) dst[e] = neutral;
       continue;
     }
-    if (vec_ok && (SKL_BOUNDARY == 1 || row_in) && gc0 >= 0 && gc0 + SKL_EPC <= C) {
-      // interior: asynchronous 16-byte global->shared copy (LDGSTS), no register
-      // round trip, all of a thread's chunks in flight at once
+    const SKL_TIN* row = in + (long)(gr - irow0) * Ci;
+    if (vec_ok && (SKL_BOUNDARY == 1 || row_in) && gc0 >= 0 && gc0 + SKL_EPC <= Ci) {
+      // asynchronous 16-byte global->shared copy (LDGSTS), no register round trip
       const unsigned sa = (unsigned)__cvta_generic_to_shared(dst);
-      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa),
-                   "l"(in + (gr - in_row0) * C + gc0) : "memory");
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(row + gc0) : "memory");
     } else {
 #pragma unroll
       for (int e = 0; e < SKL_EPC; ++e) {
-        long gc = gc0 + e;
+        int gc = gc0 + e;
         SKL_TIN v;
 #if SKL_BOUNDARY == 1
-        gc = skl_clampl(gc, 0, C - 1);
-        v = in[(gr - in_row0) * C + gc];
+        gc = gc < 0 ? 0 : (gc > Ci - 1 ? Ci - 1 : gc);
+        v = row[gc];
 #else
-        if (row_in && gc >= 0 && gc < C) v = in[(gr - in_row0) * C + gc];
+        if (row_in && gc >= 0 && gc < Ci) v = row[gc];
         else v = neutral;
 #endif
         dst[e] = v;
@@ -130,38 +133,41 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
   __syncthreads();
   // ---- apply f to a SKL_RH x SKL_CW block per thread
   const int ty = threadIdx.x / (SKL_TW / SKL_CW), tx = threadIdx.x % (SKL_TW / SKL_CW);
-  const long cc = c0 + (long)tx * SKL_CW;
-  const bool full = vec_ok && cc + SKL_CW <= C;  // whole packed store in range
+  const int cc = c0 + tx * SKL_CW;
+  const int ncols = Ci - cc;                        // columns left in the row from cc
+  const bool full = vec_ok && ncols >= SKL_CW;      // whole packed store in range
+  const int rt = r0 + ty * SKL_RH;                  // this thread's first row
+  SKL_TOUT* o = out + (long)(rt - orow0) * Ci + cc;
   // fused halo push: the first / last hd rows of this device's
   // block also go into the neighbours' halo rows (peer memory), so the next
   // overlap read needs no exchange.  Block-uniform; the common path below
   // carries none of it (live registers matter: f may call the IEEE sqrt
   // subroutine).
-  if ((push_up && r0 < r_begin + hd) || (push_down && r0 + SKL_TH > r_end - hd)) {
+  const int hdi = (int)hd;
+  if ((push_up && r0 < rb + hdi) || (push_down && r0 + SKL_TH > re - hdi)) {
 #pragma unroll
     for (int i = 0; i < SKL_RH; ++i) {
-      const long r = r0 + (long)ty * SKL_RH + i;
+      const int r = rt + i;
       const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
       SklMoRes res;
 #pragma unroll
       for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
-      if (r >= r_end) continue;
-      skl_mo_store(out + (r - out_row0) * C + cc, res, full, C - cc);
-      if (push_up && r < r_begin + hd) skl_mo_store(push_up + (r - r_begin) * C + cc, res, full, C - cc);
-      if (push_down && r >= r_end - hd)
-        skl_mo_store(push_down + (r - (r_end - hd)) * C + cc, res, full, C - cc);
+      if (r >= re) continue;
+      skl_mo_store(o + (long)i * Ci, res, full, ncols);
+      if (push_up && r < rb + hdi) skl_mo_store(push_up + (long)(r - rb) * Ci + cc, res, full, ncols);
+      if (push_down && r >= re - hdi)
+        skl_mo_store(push_down + (long)(r - (re - hdi)) * Ci + cc, res, full, ncols);
     }
     return;
   }
 #pragma unroll
   for (int i = 0; i < SKL_RH; ++i) {
-    const long r = r0 + (long)ty * SKL_RH + i;
     const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
     SklMoRes res;
 #pragma unroll
     // f may declare a non-const pointer (Listing 1.2: "float func(float* m_in)")
     for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
-    if (r < r_end) skl_mo_store(out + (r - out_row0) * C + cc, res, full, C - cc);
+    if (rt + i < re) skl_mo_store(o + (long)i * Ci, res, full, ncols);
   }
   (void)in_rows;
 }

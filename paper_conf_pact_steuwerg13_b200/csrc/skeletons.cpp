@@ -807,6 +807,8 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   const Dist dout = (din.kind == DOVERLAP) ? Dist{DBLOCK, 0} : din;
   Cont* o = output_for(ctx, out, s->tout, in->rows, in->cols, in->matrix);
   if (o == in) fail(SKL_ERR_INVALID_ARG, "MapOverlap cannot run in place");
+  if (in->rows >= (1ull << 31) || in->cols >= (1ull << 31))
+    fail(SKL_ERR_INVALID_ARG, "MapOverlap: rows and columns must be < 2^31");
   prepare_output(o, dout, dout.kind == DBLOCK ? (size_t)d : 0);
   const size_t si = in->elt, so = o->elt;
   std::vector<void*> push_up, push_down;
