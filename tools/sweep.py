@@ -50,6 +50,58 @@ def timeit(fn, reps=10, warm=3):
     return float(np.median([a.elapsed_time(b) for a, b in ts]))
 
 
+def dot20():
+    """fused dot product at 2^20 (BASELINE config 0) in a CUDA graph, cold and warm,
+    DOT_CFGS="block,..." """
+    n = 1 << 20
+    a, b = I.uniform_f32(1, n), I.uniform_f32(2, n)
+    for bt in (int(x) for x in os.environ.get("DOT_CFGS", "256").split(",")):
+        c = ctx_with({"block_threads": bt})
+        va = S.Vector.from_numpy(c, a).set_distribution(S.BLOCK)
+        vb = S.Vector.from_numpy(c, b).set_distribution(S.BLOCK)
+        mult, sm = S.Zip(c, A.MULT, S.F32, S.F32, S.F32), S.Reduce(c, A.SUM, S.F32)
+        s = sm(mult(va, vb))
+        g = c.capture(lambda: sm(mult(va, vb), out=s))
+        cold = timeit(g.launch, reps=30)
+        ts = []
+        for _ in range(30):
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record()
+            g.launch()
+            e1.record()
+            ts.append((e0, e1))
+        torch.cuda.synchronize()
+        warm = float(np.median([x.elapsed_time(y) for x, y in ts]))
+        ref = O.reduce_(O.OP_ADD_F32, O.zip_(O.OZ_MULT_F32, a, b))
+        ok = abs(float(s.scalar()) - ref) <= 1e-5 * abs(ref)
+        print(f"dot20 block={bt}: cold {cold * 1e3:.2f} us  warm {warm * 1e3:.2f} us  ok={ok}", flush=True)
+        g.destroy()
+        # floor of this measurement: a graph with one tiny kernel (fill of 4 floats)
+        tiny = S.Vector(c, S.F32, 4).set_distribution(S.BLOCK).fill(0.0)
+        g0 = c.capture(lambda: tiny.fill(1.0))
+        ts = []
+        for _ in range(30):
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record()
+            g0.launch()
+            e1.record()
+            ts.append((e0, e1))
+        torch.cuda.synchronize()
+        print(f"   one-kernel graph floor: {float(np.median([x.elapsed_time(y) for x, y in ts])) * 1e3:.2f} us", flush=True)
+        # and a plain torch kernel between the same events
+        t = torch.zeros(4, device="cuda")
+        ts = []
+        for _ in range(30):
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record()
+            t.add_(1.0)
+            e1.record()
+            ts.append((e0, e1))
+        torch.cuda.synchronize()
+        print(f"   one torch kernel: {float(np.median([x.elapsed_time(y) for x, y in ts])) * 1e3:.2f} us", flush=True)
+        c.finalize()
+
+
 def mandel():
     """MANDEL_CFGS="fn,block,unroll,interleave;..." (fn: plain | unroll4)"""
     grid = I.mandel_grid(3072, 4096)
