@@ -235,6 +235,7 @@ skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value) {
     else if (k == "d2h_bytes") *value = c->d2h;
     else if (k == "p2p_bytes") *value = c->p2p;
     else if (k == "halo_push_bytes") *value = c->pushed;
+    else if (k == "disk_cache_hits") *value = c->n_disk_hit;
     else fail(SKL_ERR_INVALID_ARG, "unknown counter " + k);
   });
 }
@@ -346,6 +347,7 @@ skl_status skl_fill(skl_cont* c, const void* value) {
   });
 }
 skl_status skl_set_distribution(skl_cont* c, int kind, int arg, skl_skel* combine) {
+  NvtxRange nr("skl_set_distribution");
   return guard([&] {
     Cont* k = K(c);
     Ctx* ctx = k->ctx;
@@ -457,6 +459,7 @@ skl_status skl_allpairs_zr_create(skl_ctx* ctx, const char* zip_src, const char*
   });
 }
 skl_status skl_allpairs_run(skl_skel* sk, skl_cont* a, skl_cont* b, skl_cont** c) {
+  NvtxRange nr("skl_allpairs_run");
   return run_out(c, [&](Cont** o) { run_allpairs(S(sk), K(a), K(b), o); });
 }
 skl_status skl_mapoverlap_bounds(skl_skel* sk, int* proven) {
@@ -476,6 +479,7 @@ skl_status skl_skel_destroy(skl_skel* sk) {
   });
 }
 skl_status skl_map_run(skl_skel* sk, skl_cont* in, skl_cont** out, const skl_arg* extra, int nextra) {
+  NvtxRange nr("skl_map_run");
   Skel* s = nullptr;
   skl_status st = guard([&] { s = S(sk); K(in); });
   if (st) return st;
@@ -490,6 +494,7 @@ skl_status skl_map_run(skl_skel* sk, skl_cont* in, skl_cont** out, const skl_arg
 }
 skl_status skl_zip_run(skl_skel* sk, skl_cont* left, skl_cont* right, skl_cont** out,
                        const skl_arg* extra, int nextra) {
+  NvtxRange nr("skl_zip_run");
   Skel* s = nullptr;
   skl_status st = guard([&] { s = S(sk); K(left); K(right); });
   if (st) return st;
@@ -503,12 +508,15 @@ skl_status skl_zip_run(skl_skel* sk, skl_cont* left, skl_cont* right, skl_cont**
   return run_out(out, [&](Cont** o) { run_zip(s, K(left), K(right), o, extra, nextra); });
 }
 skl_status skl_reduce_run(skl_skel* sk, skl_cont* in, skl_cont** scalar) {
+  NvtxRange nr("skl_reduce_run");
   return run_out(scalar, [&](Cont** o) { run_reduce(S(sk), K(in), o); });
 }
 skl_status skl_scan_run(skl_skel* sk, skl_cont* in, skl_cont** out) {
+  NvtxRange nr("skl_scan_run");
   return run_out(out, [&](Cont** o) { run_scan(S(sk), K(in), o); });
 }
 skl_status skl_mapoverlap_run(skl_skel* sk, skl_cont* in, skl_cont** out) {
+  NvtxRange nr("skl_mapoverlap_run");
   return run_out(out, [&](Cont** o) { run_mapoverlap(S(sk), K(in), o); });
 }
 skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes) {

@@ -27,6 +27,7 @@ struct NcclApi {
   decltype(&ncclSend) send = nullptr;
   decltype(&ncclRecv) recv = nullptr;
   decltype(&ncclGetErrorString) errstr = nullptr;
+  decltype(&ncclCommGetAsyncError) asyncError = nullptr;
 };
 NcclApi* nccl() {
   static NcclApi a;
@@ -46,6 +47,7 @@ NcclApi* nccl() {
     a.send = (decltype(a.send))dlsym(a.h, "ncclSend");
     a.recv = (decltype(a.recv))dlsym(a.h, "ncclRecv");
     a.errstr = (decltype(a.errstr))dlsym(a.h, "ncclGetErrorString");
+    a.asyncError = (decltype(a.asyncError))dlsym(a.h, "ncclCommGetAsyncError");
   });
   if (!a.h || !a.commInitRank || !a.send || !a.recv)
     fail(SKL_ERR_UNSUPPORTED, "NCCL (libnccl.so.2) could not be loaded");
@@ -120,6 +122,12 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
     }
   }
   nccl_check(a->groupEnd(), "ncclGroupEnd");
+  // errors of communication already in flight (peer failure, transport errors)
+  if (a->asyncError) {
+    ncclResult_t ar = ncclSuccess;
+    nccl_check(a->asyncError(comm, &ar), "ncclCommGetAsyncError");
+    if (ar != ncclSuccess && ar != ncclInProgress) nccl_check(ar, "NCCL asynchronous error");
+  }
 }
 
 }  // namespace skl

@@ -41,6 +41,7 @@ struct Nvrtc {
   nvrtcResult_t (*cubin)(void*, char*);
   nvrtcResult_t (*destroy)(void**);
   const char* (*errstr)(nvrtcResult_t);
+  nvrtcResult_t (*version)(int*, int*);
 };
 Nvrtc* nvrtc() {
   static Nvrtc n;
@@ -61,6 +62,7 @@ Nvrtc* nvrtc() {
     n.cubin = (decltype(n.cubin))dlsym(n.h, "nvrtcGetCUBIN");
     n.destroy = (decltype(n.destroy))dlsym(n.h, "nvrtcDestroyProgram");
     n.errstr = (decltype(n.errstr))dlsym(n.h, "nvrtcGetErrorString");
+    n.version = (decltype(n.version))dlsym(n.h, "nvrtcVersion");
   });
   if (!n.h || !n.create || !n.compile || !n.cubin)
     fail(SKL_ERR_UNSUPPORTED, "NVRTC (libnvrtc.so.12) could not be loaded");
@@ -79,6 +81,53 @@ std::string program_source(Ctx* ctx, const std::string& body) {
   return s;
 }
 
+// ---- optional on-disk cubin cache (SKL_CACHE_DIR): a process that creates the
+// same skeletons again skips NVRTC.  Key = two independent 64-bit hashes of the
+// options, the NVRTC version and the full program source.
+static const char* const kNvrtcOpts[] = {"--gpu-architecture=sm_100a", "-fmad=false", "--prec-div=true",
+                                         "--prec-sqrt=true", "--ftz=false", "-default-device", "-std=c++17",
+                                         "-lineinfo", "--extra-device-vectorization"};
+static std::string cache_path(const std::string& source, int nvrtc_version) {
+  const char* dir = std::getenv("SKL_CACHE_DIR");
+  if (!dir || !*dir) return std::string();
+  std::string text = std::to_string(nvrtc_version) + "\n";
+  for (const char* o : kNvrtcOpts) text += std::string(o) + "\n";
+  text += source;
+  unsigned long long h1 = 1469598103934665603ull, h2 = 0x9e3779b97f4a7c15ull;
+  for (unsigned char ch : text) {
+    h1 = (h1 ^ ch) * 1099511628211ull;                          // FNV-1a
+    h2 = (h2 ^ (ch + 0x9e3779b97f4a7c15ull + (h2 << 6) + (h2 >> 2))) * 0xff51afd7ed558ccdull;
+  }
+  char name[64];
+  std::snprintf(name, sizeof(name), "/skl_%016llx%016llx.cubin", h1, h2);
+  return std::string(dir) + name;
+}
+static bool cache_read(const std::string& path, std::vector<char>& out) {
+  if (path.empty()) return false;
+  FILE* f = std::fopen(path.c_str(), "rb");
+  if (!f) return false;
+  std::fseek(f, 0, SEEK_END);
+  const long n = std::ftell(f);
+  std::fseek(f, 0, SEEK_SET);
+  bool ok = n > 0;
+  if (ok) {
+    out.resize((size_t)n);
+    ok = std::fread(out.data(), 1, (size_t)n, f) == (size_t)n;
+  }
+  std::fclose(f);
+  return ok;
+}
+static void cache_write(const std::string& path, const std::vector<char>& cubin) {
+  if (path.empty()) return;
+  const std::string tmp = path + ".tmp" + std::to_string((long long)getpid());
+  FILE* f = std::fopen(tmp.c_str(), "wb");
+  if (!f) return;  // the cache is an optimisation only
+  const bool ok = std::fwrite(cubin.data(), 1, cubin.size(), f) == cubin.size();
+  std::fclose(f);
+  if (ok) std::rename(tmp.c_str(), path.c_str());  // atomic publish
+  else std::remove(tmp.c_str());
+}
+
 Program* compile(Ctx* ctx, const std::string& source, std::string* log_out) {
   auto it = ctx->programs.find(source);
   if (it != ctx->programs.end()) {
@@ -86,13 +135,27 @@ Program* compile(Ctx* ctx, const std::string& source, std::string* log_out) {
     return it->second.get();
   }
   Nvrtc* N = nvrtc();
+  int vmaj = 0, vmin = 0;
+  if (N->version) N->version(&vmaj, &vmin);
+  const std::string cpath = cache_path(source, vmaj * 100 + vmin);
+  {
+    auto P = std::make_unique<Program>();
+    if (cache_read(cpath, P->cubin)) {
+      P->source = source;
+      if (!ctx->offline) {
+        ctx->set_device(ctx->first_local);
+        SKL_CUDA(cudaLibraryLoadData(&P->lib, P->cubin.data(), nullptr, nullptr, 0, nullptr, nullptr, 0));
+      }
+      ctx->n_disk_hit++;
+      Program* raw = P.get();
+      ctx->programs[source] = std::move(P);
+      return raw;
+    }
+  }
   void* prog = nullptr;
   if (N->create(&prog, source.c_str(), "skl_program.cu", 0, nullptr, nullptr) != 0)
     fail(SKL_ERR_COMPILE, "nvrtcCreateProgram failed");
-  const char* opts[] = {"--gpu-architecture=sm_100a", "-fmad=false", "--prec-div=true",
-                        "--prec-sqrt=true", "--ftz=false", "-default-device", "-std=c++17",
-                        "-lineinfo", "--extra-device-vectorization"};
-  const int rc = N->compile(prog, (int)(sizeof(opts) / sizeof(opts[0])), opts);
+  const int rc = N->compile(prog, (int)(sizeof(kNvrtcOpts) / sizeof(kNvrtcOpts[0])), kNvrtcOpts);
   size_t ls = 0;
   N->logsize(prog, &ls);
   std::string log(ls, '\0');
@@ -114,6 +177,7 @@ Program* compile(Ctx* ctx, const std::string& source, std::string* log_out) {
     SKL_CUDA(cudaLibraryLoadData(&P->lib, P->cubin.data(), nullptr, nullptr, 0, nullptr, nullptr, 0));
   }
   ctx->n_compile++;
+  cache_write(cpath, P->cubin);
   Program* raw = P.get();
   ctx->programs[source] = std::move(P);
   return raw;

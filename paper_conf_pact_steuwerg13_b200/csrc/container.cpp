@@ -354,6 +354,7 @@ static void combine_to_block(Cont* c) {
 }
 
 static void redistribute(Cont* c, const Dist& to) {
+  NvtxRange nr("skl_redistribute");
   Ctx* ctx = c->ctx;
   const size_t U = c->units(), ub = c->unit_bytes();
   const Dist from = c->dist;
@@ -434,6 +435,7 @@ void ensure(Cont* c, const Dist& d, bool halo) {
   if (c->dist == d && c->dev_valid) {
     if (d.kind == DOVERLAP && halo && !c->halo_valid) {
       // halo refresh: only the border units move
+      NvtxRange nr("skl_halo_refresh");
       const std::vector<Transfer> tr = plan_transfers(c->units(), c->ctx->G, d, false, d, true);
       set_layout(c, d);  // buffers already cover the halo (need_range)
       std::vector<Part> cur = c->parts;

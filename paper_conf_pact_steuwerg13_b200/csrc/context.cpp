@@ -15,6 +15,8 @@
 
 #include <cstdio>
 
+#include <cstdlib>
+
 #include "skl_internal.h"
 
 namespace skl {
@@ -42,7 +44,19 @@ void Ctx::set_device(int g) {
   SKL_CUDA(cudaSetDevice(D(g).phys));
 }
 
+// Environment defaults: SKL_BLOCK_THREADS (work-group size,
+// P:L470), SKL_DEBUG_BOUNDS (A21); skl_set_option overrides both.  SKL_CACHE_DIR
+// is read by the compiler (on-disk cubin cache).
+static void apply_env(Ctx* c) {
+  if (const char* v = std::getenv("SKL_BLOCK_THREADS")) {
+    const long b = std::strtol(v, nullptr, 10);
+    if (b >= 64 && b <= 1024 && b % 32 == 0) c->block_threads = (int)b;
+  }
+  if (const char* v = std::getenv("SKL_DEBUG_BOUNDS")) c->debug_bounds = std::strtol(v, nullptr, 10) != 0;
+}
+
 static void init_types(Ctx* c) {
+  apply_env(c);
   c->types.resize(12);
   c->types[SKL_VOID] = {"void", 0, 1, ""};
   c->types[SKL_U8] = {"unsigned char", 1, 1, ""};

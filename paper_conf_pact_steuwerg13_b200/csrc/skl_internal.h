@@ -7,6 +7,7 @@
 #pragma once
 
 #include <cuda_runtime.h>
+#include <nvtx3/nvToolsExt.h>
 
 #include <atomic>
 #include <cstdint>
@@ -24,6 +25,16 @@
 namespace skl {
 
 // ------------------------------------------------------------------ errors
+// NVTX ranges (SURVEY §5 tracing): one per skeleton call and redistribution,
+// visible in nsys / ncu timelines; no-ops unless a tool is attached (NVTX v3 is
+// header-only and loads the tool's injection library on first use).
+struct NvtxRange {
+  explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+  ~NvtxRange() { nvtxRangePop(); }
+  NvtxRange(const NvtxRange&) = delete;
+  NvtxRange& operator=(const NvtxRange&) = delete;
+};
+
 struct Error : std::runtime_error {
   int code;
   Error(int c, const std::string& m) : std::runtime_error(m), code(c) {}
@@ -133,7 +144,7 @@ struct Ctx {
   // only: 3 / 4 / 6 without look-back (wrong results, the pipeline's ceiling)
   int scan_variant = 6;
   // counters
-  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0};
+  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0}, n_disk_hit{0};
   int composed_id = 0;  // names of composed Map chains (lazy fusion)
   // optional caller-provided device allocator (skl_set_allocator)
   void* (*user_alloc)(size_t, int, void*, void*) = nullptr;

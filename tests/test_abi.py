@@ -197,3 +197,25 @@ def test_static_get_bounds(offline):
     # comments do not count
     assert S.MapOverlap(c, "float f(const float* p){ /* get(p, 9, 9) */ return get(p, 1, 1); }",
                         S.F32, S.F32, 1).bounds_proven
+
+
+def test_disk_cache_and_env_defaults(tmp_path, monkeypatch):
+    """SKL_CACHE_DIR: a second context loads the cubin from disk instead of
+    running NVRTC; SKL_BLOCK_THREADS / SKL_DEBUG_BOUNDS set context defaults
+    (SURVEY §5 config).  Offline contexts: no GPU needed."""
+    monkeypatch.setenv("SKL_CACHE_DIR", str(tmp_path))
+    src = "float twice(float x){ return x + x; }"
+    c1 = S.Context.offline()
+    S.Map(c1, src, S.F32, S.F32)
+    assert c1.counter("compiles") == 1 and c1.counter("disk_cache_hits") == 0
+    c1.finalize()
+    assert len(list(tmp_path.glob("skl_*.cubin"))) == 1
+    c2 = S.Context.offline()
+    m = S.Map(c2, src, S.F32, S.F32)
+    assert c2.counter("compiles") == 0 and c2.counter("disk_cache_hits") == 1
+    assert len(m.cubin()) > 0
+    c2.finalize()
+    monkeypatch.setenv("SKL_BLOCK_THREADS", "128")
+    c3 = S.Context.offline()
+    assert "#define SKL_BLOCK 128" in S.Map(c3, src, S.F32, S.F32).source()
+    c3.finalize()

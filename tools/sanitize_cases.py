@@ -1,0 +1,114 @@
+"""Small cases of every kernel for compute-sanitizer, each checked
+against the oracle so a sanitizer run is also a parity run:
+
+  compute-sanitizer --tool memcheck  --error-exitcode 3 python tools/sanitize_cases.py
+  compute-sanitizer --tool racecheck --error-exitcode 3 python tools/sanitize_cases.py
+  compute-sanitizer --tool synccheck --error-exitcode 3 python tools/sanitize_cases.py
+"""
+import os
+import sys
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+sys.path.insert(0, os.path.join(ROOT, "tests"))
+
+import oracle as O  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import apps as A  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import inputs as I  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
+from paper_conf_pact_steuwerg13_b200.lmosem import ListModeOSEM  # noqa: E402
+
+
+def rel(a, b):
+    a, b = np.asarray(a, np.float64), np.asarray(b, np.float64)
+    return float(np.linalg.norm(a - b) / max(np.linalg.norm(b), 1e-300))
+
+
+def one_device(opts):
+    ctx = S.Context(1)
+    for k, v in opts.items():
+        ctx.set_option(k, v)
+    n = 70001
+    x = I.uniform_f32(1, n) - np.float32(0.5)
+    y = I.uniform_f32(2, n)
+    vx, vy = S.Vector.from_numpy(ctx, x), S.Vector.from_numpy(ctx, y)
+    assert np.array_equal(S.Map(ctx, A.SQP1, S.F32, S.F32)(vx).to_numpy(), O.map_(O.OM_SQP1_F32, x))
+    assert np.array_equal(S.Zip(ctx, A.ADD, S.F32, S.F32, S.F32)(vx, vy).to_numpy(), O.zip_(O.OZ_ADD_F32, x, y))
+    u = I.uniform_int(3, n, 0, 255, np.int64).astype(np.uint8)
+    assert np.array_equal(S.Map(ctx, A.INV_U8, S.U8, S.U8)(S.Vector.from_numpy(ctx, u)).to_numpy(),
+                          O.map_(O.OM_INV_U8, u))
+    red = S.Reduce(ctx, A.SUM, S.F32)
+    ref = O.reduce_(O.OP_ADD_F32, x)
+    assert abs(float(red(vx).scalar()) - ref) <= 1e-5 * max(1.0, abs(ref))
+    d = float(red(S.Zip(ctx, A.MULT, S.F32, S.F32, S.F32)(vx, vy)).scalar())   # fused
+    dref = O.reduce_(O.OP_ADD_F32, O.zip_(O.OZ_MULT_F32, x, y))
+    assert abs(d - dref) <= 1e-5 * max(1.0, abs(dref))
+    xi = I.uniform_int(4, n, -1000, 1000)
+    sc = S.Scan(ctx, A.ADD_I32, S.I32)
+    assert np.array_equal(sc(S.Vector.from_numpy(ctx, xi)).to_numpy(), O.scan(O.OP_ADD_I32, xi))
+    aff = ctx.struct_type("Aff", A.AFFINE_DECL, 8, 4)
+    p = I.uniform_int(5, 2 * 5003, 0, 2**32 - 1, np.uint64).astype(np.uint32).reshape(5003, 2)
+    got = S.Scan(ctx, A.AFFINE_COMPOSE, aff)(S.Vector(ctx, aff, 5003).copy_in(p)).to_numpy(np.uint32)
+    assert np.array_equal(got.reshape(5003, 2), O.scan(O.OP_AFFINE_U32, p))
+    img8 = I.image_u8(5, 70, 133)
+    sob = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+    assert np.array_equal(sob(S.Matrix.from_numpy(ctx, img8)).to_numpy(),
+                          O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0))
+    imgf = I.image_f32(6, 150, 270)
+    gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    assert np.array_equal(gau(S.Matrix.from_numpy(ctx, imgf)).to_numpy(),
+                          O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0))
+    v1 = I.uniform_f32(7, 9001)
+    box1 = S.MapOverlap(ctx, A.BOX1D, S.F32, S.F32, 1, S.NEAREST, 0.0)
+    assert np.array_equal(box1(S.Vector.from_numpy(ctx, v1)).to_numpy(),
+                          O.mapoverlap1d(O.OS_BOX3, v1, 1, O.OB_NEAREST, 0.0))
+    a = I.uniform_f32(8, 130 * 36).reshape(130, 36)
+    b = I.uniform_f32(9, 70 * 36).reshape(70, 36)
+    for src, red_src, fn in ((A.MULT, A.ADD, O.AP_DOT), (A.MANHATTAN_ROWS, None, O.AP_MANHATTAN)):
+        ap = S.Allpairs(ctx, src, S.F32, S.F32, reduce=red_src) if red_src else S.Allpairs(ctx, src, S.F32, S.F32)
+        assert np.array_equal(ap(S.Matrix.from_numpy(ctx, a), S.Matrix.from_numpy(ctx, b)).to_numpy(),
+                              O.allpairs(fn, a, b))
+    grid = I.mandel_grid(24, 32)
+    m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
+    assert np.array_equal(m(S.Matrix(ctx, S.F32X2, 24, 32).copy_in(grid)).to_numpy(), O.mandelbrot(grid, 1000)[0])
+    ctx.finalize()
+
+
+def logical_devices(G):
+    ctx = S.Context(G, devices=[0] * G)
+    x = I.uniform_f32(11, 10007)
+    v = S.Vector.from_numpy(ctx, x).set_distribution(S.BLOCK)
+    v.set_distribution(S.COPY)
+    v.set_distribution(S.SINGLE, G - 1)
+    v.set_distribution(S.OVERLAP, 3)
+    v.set_distribution(S.BLOCK)
+    assert np.array_equal(v.to_numpy(), x)
+    sc = S.Scan(ctx, A.ADD, S.F32)
+    assert rel(sc(v).to_numpy(), O.scan(O.OP_ADD_F32, x)) <= 1e-5
+    imgf = I.image_f32(12, 61, 40)
+    gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    g2 = gau(gau(S.Matrix.from_numpy(ctx, imgf)))       # fused halo push between the two
+    r1 = O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0)
+    assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
+    N, nev = 8, 3000
+    osem = ListModeOSEM(ctx, N)
+    ev = I.lmosem_events(13, nev, N)
+    f0 = np.ones(N ** 3, np.float32)
+    osem.load_events(ev, 2)
+    osem.set_image(f0)
+    osem.iterate(1)
+    f = f0
+    for lo, hi in ListModeOSEM.subset_bounds(nev, 2):
+        f = O.lmosem(ev[lo:hi], N, f)[1].astype(np.float32)
+    assert rel(osem.image(), f) <= 1e-4
+    osem.destroy()
+    ctx.finalize()
+
+
+if __name__ == "__main__":
+    one_device({})
+    one_device({"scan_variant": 3, "map_interleave": 1, "block_threads": 128})
+    logical_devices(3)
+    print("sanitize cases ok", flush=True)
