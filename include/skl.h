@@ -121,13 +121,19 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * deferred and fused into the Reduce that consumes it; default 1),
  * "halo_push" (1 = a MapOverlap on several devices of this process stores its
  * border units into the neighbours' halo units, so the next overlap read
- * exchanges nothing; default 1), plus the Scan/MapOverlap tuning
- * keys listed in DESIGN.md 6.                                                  */
+ * exchanges nothing; default 1), "map_interleave" (1 = lane l of a
+ * warp handles elements base + 32 j + l: for customising functions whose cost
+ * varies per element, e.g. Mandelbrot; default 0), "ap_fast" (Allpairs
+ * zip-reduce 128 x 128 tiles for 4-byte inputs with d % 4 == 0; default 1),
+ * and the tuning keys "scan_variant", "scan_chunks", "scan_minb", "mo_rh",
+ * "mo_cw", "mo_minb".  Environment defaults: SKL_BLOCK_THREADS,
+ * SKL_DEBUG_BOUNDS; SKL_CACHE_DIR keeps compiled cubins on disk.              */
 skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
 /* Counters: "launches" (kernels this library launched), "compiles" (NVRTC runs),
  * "cache_hits", "h2d_bytes", "d2h_bytes", "p2p_bytes" (device-to-device copy
  * bytes), "halo_push_bytes" (halo bytes stored by MapOverlap kernels directly
- * into neighbour devices' memory).                                             */
+ * into neighbour devices' memory), "disk_cache_hits" (cubins loaded from
+ * SKL_CACHE_DIR instead of compiled).                                          */
 skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value);
 const char* skl_last_error(void);
 
