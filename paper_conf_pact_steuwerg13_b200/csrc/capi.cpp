@@ -205,6 +205,9 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       (k == "mo_rh" ? c->mo_rh : c->mo_cw) = (int)value;
     } else if (k == "lazy_fusion") {
       c->lazy_fusion = value ? 1 : 0;
+    } else if (k == "xfer_chunks") {
+      if (value < 1 || value > 64) fail(SKL_ERR_INVALID_ARG, "xfer_chunks in [1,64]");
+      c->xfer_chunks = (int)value;
     } else if (k == "map_interleave") {
       c->map_interleave = value ? 1 : 0;
     } else if (k == "ap_fast") {
@@ -400,6 +403,7 @@ skl_status skl_local_part(skl_cont* c, int g, void** dptr, size_t* first_unit, s
     materialize(k);
     // a distribution set on host data becomes resident here (implicit upload)
     if (k->dist.kind != DNONE && !k->dev_valid && k->host_valid) ensure(k, k->dist, k->dist.kind == DOVERLAP);
+    sync_ready(k);  // the caller reads the buffer on its own terms: pending chunks first
     Part& p = k->parts[(size_t)g];
     if (!p.ptr || p.valid.empty() || !k->dev_valid) return;
     *dptr = part_ptr(k, g, p.valid.lo);

@@ -35,7 +35,44 @@ Cont* cont_create(Ctx* ctx, int type, size_t rows, size_t cols, bool matrix) {
   return c;
 }
 
+// device stream of g waits for the pending chunks of one part
+static void sync_part(Cont* c, int g) {
+  Part& p = c->parts[(size_t)g];
+  if (p.ready.empty()) return;
+  Ctx* ctx = c->ctx;
+  ctx->set_device(g);
+  for (const Ready& rd : p.ready) {
+    SKL_CUDA(cudaStreamWaitEvent(ctx->D(g).stream, rd.ev, 0));
+    event_put(ctx, g, rd.ev);
+  }
+  p.ready.clear();
+}
+
+void sync_ready(Cont* c) {
+  Ctx* ctx = c->ctx;
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g)
+    if ((size_t)g < c->parts.size()) sync_part(c, g);
+}
+
+// number of chunks for a host<->device transfer of `bytes` (1 = one copy on the
+// device stream): chunks let a Map start on the first rows while the rest is in
+// flight, and stream its output back while later rows compute
+static int xfer_chunks(Ctx* ctx, size_t bytes) {
+  if (ctx->capturing || ctx->xfer_chunks <= 1 || bytes < (size_t)(4u << 20)) return 1;
+  return (int)std::min<size_t>((size_t)ctx->xfer_chunks, bytes / (1u << 20));
+}
+// chunk k of K of the unit range r (boundaries on multiples of 64 units, so
+// that chunk pointers keep the buffer's 16-byte alignment)
+static Range chunk_of(const Range& r, int k, int K) {
+  auto cut = [&](int i) -> size_t {
+    if (i >= K) return r.hi;
+    return r.lo + (r.size() * (size_t)i / (size_t)K) / 64 * 64;
+  };
+  return Range{cut(k), cut(k + 1)};
+}
+
 static void free_part(Cont* c, int g) {
+  sync_part(c, g);  // pending copies into the buffer complete before it is freed
   Part& p = c->parts[(size_t)g];
   if (p.ptr) device_free(c->ctx, g, p.ptr);
   p = Part();
@@ -74,6 +111,7 @@ static Range alloc_range(Cont* c, const Dist& d, int g) {
 // (Re)allocate device parts for layout d; data in reused buffers is kept.
 static void set_layout(Cont* c, const Dist& d) {
   Ctx* ctx = c->ctx;
+  sync_ready(c);
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
     const Range ar = alloc_range(c, d, g);
     Part& p = c->parts[(size_t)g];
@@ -138,8 +176,28 @@ void host_upload(Cont* c, const void* host) {
     const Range r = need_range(c->units(), ctx->G, d, g);
     if (r.empty()) continue;
     ctx->set_device(g);
-    SKL_CUDA(cudaMemcpyAsync(part_ptr(c, g, r.lo), (const char*)host + r.lo * ub, r.size() * ub,
-                             cudaMemcpyHostToDevice, ctx->D(g).stream));
+    Device& D = ctx->D(g);
+    const int K = xfer_chunks(ctx, r.size() * ub);
+    if (K == 1) {
+      SKL_CUDA(cudaMemcpyAsync(part_ptr(c, g, r.lo), (const char*)host + r.lo * ub, r.size() * ub,
+                               cudaMemcpyHostToDevice, D.stream));
+    } else {
+      // chunked upload on the copy stream, after whatever the device stream
+      // queued on this buffer (its allocation, earlier readers); each chunk's
+      // event lets a consumer start on it while later chunks are in flight
+      SKL_CUDA(cudaEventRecord(D.ev, D.stream));
+      SKL_CUDA(cudaStreamWaitEvent(D.h2d, D.ev, 0));
+      Part& p = c->parts[(size_t)g];
+      for (int k = 0; k < K; ++k) {
+        const Range q = chunk_of(r, k, K);
+        if (q.empty()) continue;
+        SKL_CUDA(cudaMemcpyAsync(part_ptr(c, g, q.lo), (const char*)host + q.lo * ub, q.size() * ub,
+                                 cudaMemcpyHostToDevice, D.h2d));
+        cudaEvent_t e = event_get(ctx, g);
+        SKL_CUDA(cudaEventRecord(e, D.h2d));
+        p.ready.push_back(Ready{q, e});
+      }
+    }
     ctx->h2d += (long long)(r.size() * ub);
   }
   set_valid(c, d, true);
@@ -154,7 +212,39 @@ static void sync_local(Ctx* ctx) {
   for (auto& d : ctx->dev) {
     SKL_CUDA(cudaSetDevice(d.phys));
     SKL_CUDA(cudaStreamSynchronize(d.stream));
+    SKL_CUDA(cudaStreamSynchronize(d.d2h));
   }
+}
+
+// Chunked download of units r of part g to `host` (which receives unit r.lo
+// first) on the copy stream, each chunk as soon as its producer finished, when
+// the part's pending chunks cover r; returns false (nothing done) otherwise.
+static bool stream_out(Cont* c, int g, const Range& r, void* host) {
+  Ctx* ctx = c->ctx;
+  Part& p = c->parts[(size_t)g];
+  if (p.ready.empty() || ctx->capturing) return false;
+  size_t covered = 0;
+  for (const Ready& rd : p.ready) {
+    const size_t lo = std::max(rd.r.lo, r.lo), hi = std::min(rd.r.hi, r.hi);
+    if (hi > lo) covered += hi - lo;
+  }
+  if (covered != r.size()) return false;  // chunks overlap or leave gaps: plain path
+  ctx->set_device(g);
+  Device& D = ctx->D(g);
+  const size_t ub = c->unit_bytes();
+  for (const Ready& rd : p.ready) {
+    const size_t lo = std::max(rd.r.lo, r.lo), hi = std::min(rd.r.hi, r.hi);
+    SKL_CUDA(cudaStreamWaitEvent(D.d2h, rd.ev, 0));
+    if (hi > lo)
+      SKL_CUDA(cudaMemcpyAsync((char*)host + (lo - r.lo) * ub, part_ptr(c, g, lo), (hi - lo) * ub,
+                               cudaMemcpyDeviceToHost, D.d2h));
+    event_put(ctx, g, rd.ev);
+  }
+  p.ready.clear();
+  // later writers of this buffer on the device stream come after the reads
+  SKL_CUDA(cudaEventRecord(D.ev, D.d2h));
+  SKL_CUDA(cudaStreamWaitEvent(D.stream, D.ev, 0));
+  return true;
 }
 
 namespace {
@@ -194,14 +284,17 @@ void host_download(Cont* c, void* host) {
       Range r = c->dist.kind == DCOPY ? block_range(c->units(), ctx->G, g)
                                       : core_range(c->units(), ctx->G, c->dist, g);
       if (r.empty()) continue;
-      ctx->set_device(g);
-      SKL_CUDA(cudaMemcpyAsync((char*)host + r.lo * ub, part_ptr(c, g, r.lo), r.size() * ub,
-                               cudaMemcpyDeviceToHost, ctx->D(g).stream));
+      if (!stream_out(c, g, r, (char*)host + r.lo * ub)) {
+        ctx->set_device(g);
+        SKL_CUDA(cudaMemcpyAsync((char*)host + r.lo * ub, part_ptr(c, g, r.lo), r.size() * ub,
+                                 cudaMemcpyDeviceToHost, ctx->D(g).stream));
+      }
       ctx->d2h += (long long)(r.size() * ub);
     }
     sync_local(ctx);
     return;
   }
+  sync_ready(c);
   // one process per GPU: every rank assembles the whole container (collective)
   const int g = ctx->first_local;
   const Range have = core_range(c->units(), ctx->G, c->dist, g);
@@ -242,8 +335,12 @@ void download_part(Cont* c, int g, void* host, size_t* first, size_t* n) {
   *n = r.size();
   if (r.empty()) return;
   ctx->set_device(g);
-  SKL_CUDA(cudaMemcpyAsync(host, part_ptr(c, g, r.lo), r.size() * c->unit_bytes(),
-                           cudaMemcpyDeviceToHost, ctx->D(g).stream));
+  if (stream_out(c, g, r, host)) {
+    SKL_CUDA(cudaStreamSynchronize(ctx->D(g).d2h));
+  } else {
+    SKL_CUDA(cudaMemcpyAsync(host, part_ptr(c, g, r.lo), r.size() * c->unit_bytes(),
+                             cudaMemcpyDeviceToHost, ctx->D(g).stream));
+  }
   ctx->d2h += (long long)(r.size() * c->unit_bytes());
   SKL_CUDA(cudaStreamSynchronize(ctx->D(g).stream));
 }
@@ -295,6 +392,7 @@ void fill(Cont* c, const void* value) {
 // canonical all-to-all), then the ordered-combine kernel folds them.
 static void combine_to_block(Cont* c) {
   Ctx* ctx = c->ctx;
+  sync_ready(c);
   const int G = ctx->G;
   const size_t U = c->units(), ub = c->unit_bytes();
   const Dist blk{DBLOCK, 0};
@@ -413,7 +511,19 @@ static bool halos_allocated(Cont* c, const Dist& d) {
   return true;
 }
 
-void ensure(Cont* c, const Dist& d, bool halo) {
+static void ensure_impl(Cont* c, const Dist& d, bool halo);
+
+void ensure(Cont* c, const Dist& d, bool halo, bool keep_ready) {
+  // nothing to move: pending upload chunks may stay pending for the caller
+  const bool noop = !c->lazy.s && c->dev_valid && c->dist == d &&
+                    !(d.kind == DOVERLAP && halo && !c->halo_valid) &&
+                    !(c->dist.kind == DCOPY && c->diverged && c->combine);
+  if (!noop) sync_ready(c);
+  ensure_impl(c, d, halo);
+  if (!keep_ready) sync_ready(c);
+}
+
+static void ensure_impl(Cont* c, const Dist& d, bool halo) {
   if (d.kind == DNONE) fail(SKL_ERR_DISTRIBUTION, "no distribution");
   materialize(c);  // a deferred Zip/Map result is computed before it is used
   if (c->dev_valid && c->dist.kind == DCOPY && c->diverged && c->combine && !(d == c->dist)) {

@@ -29,6 +29,10 @@ void fail(int code, const std::string& msg) { throw Error(code, msg); }
 
 void cuda_check(cudaError_t e, const char* what) {
   if (e == cudaSuccess) return;
+  // the runtime also keeps the error as its per-thread "last error": clear it,
+  // or a later cudaGetLastError() (after a launch) would report this failure
+  // again (non-sticky errors such as a failed allocation leave the context usable)
+  (void)cudaGetLastError();
   const int code = (e == cudaErrorMemoryAllocation) ? SKL_ERR_OOM : SKL_ERR_CUDA;
   fail(code, std::string(what) + ": " + cudaGetErrorName(e) + " (" + cudaGetErrorString(e) + ")");
 }
@@ -77,6 +81,8 @@ static void init_device(Ctx* c, Device& d) {
   SKL_CUDA(cudaStreamCreateWithFlags(&d.own, cudaStreamNonBlocking));
   d.stream = d.own;
   SKL_CUDA(cudaEventCreateWithFlags(&d.ev, cudaEventDisableTiming));
+  SKL_CUDA(cudaStreamCreateWithFlags(&d.h2d, cudaStreamNonBlocking));
+  SKL_CUDA(cudaStreamCreateWithFlags(&d.d2h, cudaStreamNonBlocking));
   SKL_CUDA(cudaDeviceGetAttribute(&d.sm_count, cudaDevAttrMultiProcessorCount, d.phys));
   cudaMemPool_t pool;
   SKL_CUDA(cudaDeviceGetDefaultMemPool(&pool, d.phys));
@@ -171,6 +177,8 @@ void ctx_destroy(Ctx* c) {
     cudaSetDevice(d.phys);
     cudaStreamSynchronize(d.stream);
     cudaStreamSynchronize(d.own);
+    if (d.h2d) cudaStreamSynchronize(d.h2d);
+    if (d.d2h) cudaStreamSynchronize(d.d2h);
   }
   while (!c->skels.empty()) skel_destroy(*c->skels.begin());
   while (!c->conts.empty()) cont_destroy(*c->conts.begin());
@@ -184,6 +192,9 @@ void ctx_destroy(Ctx* c) {
   for (auto& d : c->dev) {
     cudaSetDevice(d.phys);
     if (d.ev) cudaEventDestroy(d.ev);
+    for (cudaEvent_t e : d.ev_pool) cudaEventDestroy(e);
+    if (d.h2d) cudaStreamDestroy(d.h2d);
+    if (d.d2h) cudaStreamDestroy(d.d2h);
     if (d.own) cudaStreamDestroy(d.own);
   }
   delete c;
@@ -214,6 +225,24 @@ void device_free(Ctx* ctx, int g, void* p) {
     return;
   }
   SKL_CUDA(cudaFreeAsync(p, ctx->D(g).stream));
+}
+
+// Reusable events (a stream wait captures the event's state when it is issued,
+// so an event can be re-recorded as soon as the waits on it are enqueued).
+cudaEvent_t event_get(Ctx* ctx, int g) {
+  Device& d = ctx->D(g);
+  if (!d.ev_pool.empty()) {
+    cudaEvent_t e = d.ev_pool.back();
+    d.ev_pool.pop_back();
+    return e;
+  }
+  ctx->set_device(g);
+  cudaEvent_t e = nullptr;
+  SKL_CUDA(cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
+  return e;
+}
+void event_put(Ctx* ctx, int g, cudaEvent_t e) {
+  if (e) ctx->D(g).ev_pool.push_back(e);
 }
 
 // Every local stream waits for the work already queued on every other local

@@ -362,7 +362,8 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     }
   }
   const Dist din = elementwise(default_dist(in, Dist{DBLOCK, 0}));  // A6
-  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false);
+  // keep_ready: chunks of an upload still in flight are consumed one by one below
+  ensure(in, in->dist.kind == DOVERLAP ? in->dist : din, false, /*keep_ready=*/true);
   if (in2) {
     // A7: the right input follows the left input's distribution
     if (!(elementwise(in2->dist) == din && in2->dev_valid)) ensure(in2, din, false);
@@ -380,6 +381,14 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     return;
   }
   ExtraArgs ea = prepare_extras(s, extra, nextra);
+  // the input's pending upload chunks (chunked copy_in / upload on first use):
+  // one launch per chunk, each waiting only for its own chunk
+  std::vector<std::vector<Ready>> chunks((size_t)ctx->G);
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    chunks[(size_t)g].swap(in->parts[(size_t)g].ready);
+    std::sort(chunks[(size_t)g].begin(), chunks[(size_t)g].end(),
+              [](const Ready& a, const Ready& b) { return a.r.lo < b.r.lo; });
+  }
   Cont* o = nullptr;
   if (s->tout != SKL_VOID) {
     o = output_for(ctx, out, s->tout, in->rows, in->cols, in->matrix);
@@ -391,10 +400,7 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
                s->tout == SKL_VOID ? 0 : ctx->type(s->tout).size}), 64);
   const size_t per_block = (size_t)s->block * (size_t)s->unroll;
   int ndev = 0;
-  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
-    const Range r = core_range(in->units(), ctx->G, din, g);
-    if (r.empty()) continue;
-    ++ndev;
+  auto launch_range = [&](int g, const Range& r) {
     const void* pin = part_ptr(in, g, r.lo);
     const void* pin2 = in2 ? part_ptr(in2, g, r.lo) : nullptr;
     void* pout = o ? part_ptr(o, g, r.lo) : nullptr;
@@ -427,6 +433,48 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
       kname = "skl_map_sc";
     }
     launch(ctx, g, s->prog, kname, dim3((unsigned)grid), dim3(s->block), 0, args.data());
+  };
+  for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
+    const Range r = core_range(in->units(), ctx->G, din, g);
+    std::vector<Ready>& ch = chunks[(size_t)g];
+    if (r.empty()) {
+      ctx->set_device(g);
+      for (const Ready& rd : ch) {  // nothing to compute here: just order the stream
+        SKL_CUDA(cudaStreamWaitEvent(ctx->D(g).stream, rd.ev, 0));
+        event_put(ctx, g, rd.ev);
+      }
+      continue;
+    }
+    ++ndev;
+    size_t covered = 0;
+    for (const Ready& rd : ch) {
+      const size_t lo = std::max(rd.r.lo, r.lo), hi = std::min(rd.r.hi, r.hi);
+      if (hi > lo) covered += hi - lo;
+    }
+    if (ch.empty() || covered != r.size()) {
+      ctx->set_device(g);
+      for (const Ready& rd : ch) {
+        SKL_CUDA(cudaStreamWaitEvent(ctx->D(g).stream, rd.ev, 0));
+        event_put(ctx, g, rd.ev);
+      }
+      launch_range(g, r);
+      continue;
+    }
+    // pipelined: chunk k computes while chunk k+1 uploads; each output chunk
+    // gets an event so that a download can stream it out while later chunks run
+    for (const Ready& rd : ch) {
+      const Range q{std::max(rd.r.lo, r.lo), std::min(rd.r.hi, r.hi)};
+      ctx->set_device(g);
+      SKL_CUDA(cudaStreamWaitEvent(ctx->D(g).stream, rd.ev, 0));
+      event_put(ctx, g, rd.ev);
+      if (q.empty()) continue;
+      launch_range(g, q);
+      if (o) {
+        cudaEvent_t e = event_get(ctx, g);
+        SKL_CUDA(cudaEventRecord(e, ctx->D(g).stream));
+        o->parts[(size_t)g].ready.push_back(Ready{q, e});
+      }
+    }
   }
   if (o) mark_written(o);
   finish_extras(ctx, ea, ndev);

@@ -100,6 +100,10 @@ struct Device {
   cudaStream_t own = nullptr, stream = nullptr;  // library stream, current stream
   cudaEvent_t ev = nullptr;                      // scratch event for cross-stream sync
   int sm_count = 148;
+  // copy-engine streams for chunked host<->device transfers that overlap with
+  // kernels on `stream`, and a pool of reusable events
+  cudaStream_t h2d = nullptr, d2h = nullptr;
+  std::vector<cudaEvent_t> ev_pool;
 };
 
 struct Cont;
@@ -134,6 +138,7 @@ struct Ctx {
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
+  int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
   int ap_fast = 1;             // Allpairs zip-reduce: 128 x 128 tiles (4-byte inputs, d % 4 == 0)           // MapOverlap stores its border rows into the neighbours' halos
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 6 = one block per tile, tile kept in shared memory, low
@@ -160,11 +165,19 @@ struct Ctx {
 };
 
 // ------------------------------------------------------------------ containers
+// A unit range of a part that becomes valid when `ev` completes (chunked
+// upload on the copy stream, or a chunk of a Map's output); consumers on the
+// device stream wait for it, or stream it out chunk by chunk.
+struct Ready {
+  Range r;
+  cudaEvent_t ev = nullptr;
+};
 struct Part {
   void* ptr = nullptr;  // device buffer; addresses unit buf.lo
   Range buf;            // units the buffer covers
   Range valid;          // units holding valid data (subset of buf)
   size_t cap_bytes = 0;
+  std::vector<Ready> ready;  // pending chunks (empty: everything is ordered on the stream)
 };
 
 // A Zip/Map called without an output container is deferred (lazy fusion,
@@ -208,7 +221,11 @@ void cont_destroy(Cont* c);
 // Make `c` hold valid data in distribution `d` on the devices (upload from the
 // host mirror or redistribute device-to-device as needed).  `halo` = overlap
 // halos must be valid too.
-void ensure(Cont* c, const Dist& d, bool halo);
+// keep_ready: leave chunk events of an upload pending for the caller (a Map/Zip
+// consumes the chunks as they arrive); otherwise every pending chunk is ordered
+// before later work on the device stream.
+void ensure(Cont* c, const Dist& d, bool halo, bool keep_ready = false);
+void sync_ready(Cont* c);  // device streams wait for every pending chunk of c
 // Prepare `c` as an output in distribution `d` (contents will be overwritten on
 // the core ranges); allocates parts with `spare` halo units of room.
 void prepare_output(Cont* c, const Dist& d, size_t spare);
@@ -234,6 +251,8 @@ struct PtrFn {
 };
 void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes, PtrFn& p);
 void barrier_streams(Ctx* ctx);  // every local stream waits for every other
+cudaEvent_t event_get(Ctx* ctx, int g);
+void event_put(Ctx* ctx, int g, cudaEvent_t e);
 // NCCL (dlopen)
 void nccl_get_unique_id(void* out128);
 void nccl_init(Ctx* ctx, const void* id);

@@ -36,6 +36,10 @@ def test_out_of_memory_is_reported(ctx):
     assert e.value.name == "OOM"
     v.destroy()
     _still_works(ctx)
+    # the failed allocation must not resurface in a later launch check
+    w = S.Vector(ctx, S.F32, 1 << 20).set_distribution(S.BLOCK)
+    w.fill(1.0)
+    assert float(S.Reduce(ctx, A.SUM, S.F32)(w).scalar()) == float(1 << 20)
 
 
 def test_compile_error_carries_the_nvrtc_log(ctx):
