@@ -322,6 +322,28 @@ def ncu_traffic(workload: str):
         return None
 
 
+def ncu_field(workload: str, key: str):
+    f = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    try:
+        return float(json.load(open(f))[workload][key])
+    except Exception:
+        return None
+
+
+def roof_issue(workload: str, ms: float, P: dict, sms: int):
+    """issue-slot roofline for ALU/issue-bound kernels: the warp instructions one
+    launch executes (ncu smsp__inst_executed.sum of the committed capture) per
+    second of the measured step, against SMs x 4 schedulers x 1 instruction/clock"""
+    inst = ncu_field(workload, "inst_executed")
+    if inst is None:
+        return None
+    peak = sms * 4 * P["sm_max_mhz"] * 1e6
+    ach = inst / (ms / 1e3)
+    return {"bound": "issue", "achieved": ach / 1e12, "peak": peak / 1e12, "unit": "Twarp-inst/s",
+            "frac": ach / peak, "inst_per_launch": inst,
+            "threads_per_inst": ncu_field(workload, "threads_per_inst")}
+
+
 def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None):
     gbs = bytes_per_step / (ms / 1e3) / 1e9
     return {"bound": "hbm", "achieved": round(gbs, 1), "peak": P["hbm_gbs"], "unit": "GB/s",
@@ -493,10 +515,11 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                                      f"MapOverlap {R}x{C}, overlap distribution",
                          "ms": round(ms, 4), "elements_per_s": R * C / (ms / 1e3),
                          "roofline": roof_hbm(bpp * R * C, ms, P, name), "check": "ok" if ok else "FAIL"}
+            import torch as _t
+            sms = _t.cuda.get_device_properties(D.local).multi_processor_count
+            res[name]["roofline_issue"] = roof_issue(name, ms, P, sms)
             if name == "gauss":
                 # the binding roof: 25 FMUL + 25 FADD per pixel (no FMA under -fmad=false)
-                import torch as _t
-                sms = _t.cuda.get_device_properties(D.local).multi_processor_count
                 peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
                 fl = 50.0 * R * C / (ms / 1e3)
                 res[name]["roofline_alu"] = {"bound": "alu", "achieved": fl / 1e12, "peak": peak / 1e12,
