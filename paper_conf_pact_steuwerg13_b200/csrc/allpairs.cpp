@@ -86,12 +86,24 @@ void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out) {
       void* args[] = {(void*)&pa, (void*)&pb, &pc, &nn, &mm, &dd};
       const bool fast = si == 4 && d % 4 == 0 && ((uintptr_t)pa % 16) == 0 && ((uintptr_t)pb % 16) == 0 &&
                         ctx->ap_fast;
-      if (fast)
-        launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)cdiv(r.size(), 128)),
-               dim3(256), 0, args);
-      else
+      if (fast) {
+        // 128 x 128 tiles (2 blocks/SM) or 128 x 64 (3 blocks/SM): the one whose
+        // tile count fills the last wave better (option ap_tile forces 8 / 4)
+        const size_t sms = (size_t)ctx->D(g).sm_count, rows = cdiv(r.size(), 128);
+        const size_t t8 = cdiv(m, 128) * rows, t4 = cdiv(m, 64) * rows;
+        auto eff = [](size_t t, size_t slots) { return (double)t / (double)(cdiv(t, slots) * slots); };
+        // 128 x 64 measured ~17 % slower per FLOP (4096^3: 5.42 vs 4.98 ms): only for poor wave fill
+        bool narrow = eff(t4, 3 * sms) * 0.82 > eff(t8, 2 * sms);
+        if (ctx->ap_tile == 8) narrow = false;
+        if (ctx->ap_tile == 4) narrow = true;
+        if (narrow)
+          launch(ctx, g, s->prog, "skl_ap_zr4", dim3((unsigned)cdiv(m, 64), (unsigned)rows), dim3(256), 0, args);
+        else
+          launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)rows), dim3(256), 0, args);
+      } else {
         launch(ctx, g, s->prog, "skl_ap_zr", dim3((unsigned)cdiv(m, 64), (unsigned)cdiv(r.size(), 64)),
                dim3(256), 0, args);
+      }
     } else {
       const size_t smem = 32 * (d + 1) * si;
       int use_smem = smem <= 96 * 1024;

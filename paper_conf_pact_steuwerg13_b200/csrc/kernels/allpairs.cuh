@@ -89,7 +89,6 @@ skl_ap_zr(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT
 #define AQ_BM 128
 #define AQ_BK 16
 #define AQ_P (AQ_BK + 4)
-#define AQ_STAGE (2 * AQ_BM * AQ_P)
 union SklAp4 {
   uint4 q;
   SKL_TIN e[4];
@@ -98,8 +97,8 @@ __device__ __forceinline__ void skl_ap_cp16(void* smem, const void* g) {
   const unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
   asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(g) : "memory");
 }
-template <bool FIRST>
-__device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][8], const SKL_TIN* As, const SKL_TIN* Bs,
+template <bool FIRST, int TC>
+__device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][TC], const SKL_TIN* As, const SKL_TIN* Bs,
                                              int tx, int ty) {
 #pragma unroll
   for (int kq = 0; kq < AQ_BK; kq += 4) {
@@ -107,7 +106,7 @@ __device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][8], const SKL_TI
 #pragma unroll
     for (int r = 0; r < 8; ++r) a[r].q = *(const uint4*)&As[(ty + 16 * r) * AQ_P + kq];
 #pragma unroll
-    for (int c = 0; c < 8; ++c) {
+    for (int c = 0; c < TC; ++c) {
       SklAp4 b;
       b.q = *(const uint4*)&Bs[(tx + 16 * c) * AQ_P + kq];
 #pragma unroll
@@ -120,33 +119,45 @@ __device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][8], const SKL_TI
     }
   }
 }
-extern "C" __global__ void __launch_bounds__(256, 2)
-skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
-           long n, long m, long d) {
-  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE];
+// One 128 x (16 TC) tile of C per block of 256 threads, 8 x TC per thread.
+template <int TC>
+__device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B,
+                                            SKL_TOUT* __restrict__ Cm, long n, long m, long d) {
+  constexpr int BN = 16 * TC;                      // tile columns (rows of B)
+  constexpr int STAGE = (AQ_BM + BN) * AQ_P;
+  __shared__ __align__(16) SKL_TIN sm[2 * STAGE];
   const int tx = threadIdx.x & 15, ty = threadIdx.x >> 4;
-  const long i0 = (long)blockIdx.y * AQ_BM, j0 = (long)blockIdx.x * AQ_BM;
+  const long i0 = (long)blockIdx.y * AQ_BM, j0 = (long)blockIdx.x * BN;
   const long nfull = d / AQ_BK;
-  // chunk q of a 128 x 16 slab: row q / 4, k-quad q % 4 (rows beyond n / m are
-  // clamped to the last one: loaded, never stored)
-  long ra[2], rb[2];
+  // chunk q of a (rows x 16) slab: row q / 4, k-quad q % 4 (rows beyond n / m
+  // are clamped to the last one: loaded, never stored)
+  constexpr int HA = AQ_BM * 4 / 256, HB = BN * 4 / 256;   // chunks per thread
+  long ra[HA], rb[HB];
 #pragma unroll
-  for (int h = 0; h < 2; ++h) {
+  for (int h = 0; h < HA; ++h) {
     const int r = (threadIdx.x + h * 256) >> 2;
     ra[h] = (i0 + r < n ? i0 + r : n - 1) * d;
+  }
+#pragma unroll
+  for (int h = 0; h < HB; ++h) {
+    const int r = (threadIdx.x + h * 256) >> 2;
     rb[h] = (j0 + r < m ? j0 + r : m - 1) * d;
   }
   auto stage = [&](int st, long k0) {
-    SKL_TIN* As = sm + st * AQ_STAGE;
+    SKL_TIN* As = sm + st * STAGE;
     SKL_TIN* Bs = As + AQ_BM * AQ_P;
 #pragma unroll
-    for (int h = 0; h < 2; ++h) {
+    for (int h = 0; h < HA; ++h) {
       const int q = threadIdx.x + h * 256, r = q >> 2, kq = (q & 3) * 4;
       skl_ap_cp16(&As[r * AQ_P + kq], A + ra[h] + k0 + kq);
+    }
+#pragma unroll
+    for (int h = 0; h < HB; ++h) {
+      const int q = threadIdx.x + h * 256, r = q >> 2, kq = (q & 3) * 4;
       skl_ap_cp16(&Bs[r * AQ_P + kq], B + rb[h] + k0 + kq);
     }
   };
-  SKL_TOUT acc[8][8];
+  SKL_TOUT acc[8][TC];
   if (nfull > 0) stage(0, 0);
   asm volatile("cp.async.commit_group;" ::: "memory");
   for (long s = 0; s < nfull; ++s) {
@@ -154,9 +165,9 @@ skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOU
     asm volatile("cp.async.commit_group;" ::: "memory");
     asm volatile("cp.async.wait_group 1;" ::: "memory");
     __syncthreads();
-    const SKL_TIN* As = sm + (s & 1) * AQ_STAGE;
-    if (s == 0) skl_ap_slice<true>(acc, As, As + AQ_BM * AQ_P, tx, ty);
-    else skl_ap_slice<false>(acc, As, As + AQ_BM * AQ_P, tx, ty);
+    const SKL_TIN* As = sm + (s & 1) * STAGE;
+    if (s == 0) skl_ap_slice<true, TC>(acc, As, As + AQ_BM * AQ_P, tx, ty);
+    else skl_ap_slice<false, TC>(acc, As, As + AQ_BM * AQ_P, tx, ty);
     __syncthreads();  // the next stage() overwrites this buffer
   }
   // tail k-slice (d % 16 elements): scalar, guarded
@@ -166,12 +177,15 @@ skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOU
     SKL_TIN* As = sm;
     SKL_TIN* Bs = As + AQ_BM * AQ_P;
     const long k0 = nfull * AQ_BK;
-    for (int e = threadIdx.x; e < AQ_BM * AQ_BK; e += 256) {
+    for (int e = threadIdx.x; e < (AQ_BM + BN) * AQ_BK; e += 256) {
       const int r = e / AQ_BK, k = e % AQ_BK;
-      if (k < kt) {
-        const long ia = i0 + r < n ? i0 + r : n - 1, jb = j0 + r < m ? j0 + r : m - 1;
+      if (k >= kt) continue;
+      if (r < AQ_BM) {
+        const long ia = i0 + r < n ? i0 + r : n - 1;
         As[r * AQ_P + k] = A[ia * d + k0 + k];
-        Bs[r * AQ_P + k] = B[jb * d + k0 + k];
+      } else {
+        const long jb = j0 + (r - AQ_BM) < m ? j0 + (r - AQ_BM) : m - 1;
+        Bs[(r - AQ_BM) * AQ_P + k] = B[jb * d + k0 + k];
       }
     }
     __syncthreads();
@@ -179,7 +193,7 @@ skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOU
 #pragma unroll
       for (int r = 0; r < 8; ++r)
 #pragma unroll
-        for (int c = 0; c < 8; ++c) {
+        for (int c = 0; c < TC; ++c) {
           const SKL_TOUT z = SKL_ZFUNC(As[(ty + 16 * r) * AQ_P + k], Bs[(tx + 16 * c) * AQ_P + k]);
           acc[r][c] = (nfull == 0 && k == 0) ? z : SKL_RFUNC(acc[r][c], z);
         }
@@ -189,11 +203,23 @@ skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOU
     const long i = i0 + ty + 16 * r;
     if (i >= n) continue;
 #pragma unroll
-    for (int c = 0; c < 8; ++c) {
+    for (int c = 0; c < TC; ++c) {
       const long j = j0 + tx + 16 * c;
       if (j < m) Cm[i * m + j] = acc[r][c];
     }
   }
+}
+// 128 x 128 tiles (2 blocks per SM) and 128 x 64 tiles (3 blocks per SM, twice
+// the tiles: the host picks the one whose tile count fills the waves better)
+extern "C" __global__ void __launch_bounds__(256, 2)
+skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
+           long n, long m, long d) {
+  skl_ap_tile<8>(A, B, Cm, n, m, d);
+}
+extern "C" __global__ void __launch_bounds__(256, 3)
+skl_ap_zr4(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
+           long n, long m, long d) {
+  skl_ap_tile<4>(A, B, Cm, n, m, d);
 }
 #endif
 #else

@@ -102,6 +102,25 @@ def dot20():
         c.finalize()
 
 
+def allpairs():
+    """AP_CFGS="tile,...": 4096^3 dot and 4096x4096x128 Manhattan, zip-reduce form"""
+    for tile in (int(x) for x in os.environ.get("AP_CFGS", "0").split(",")):
+        c = ctx_with({"ap_tile": tile})
+        for name, z, dd in (("dot", A.MULT, 4096), ("manhattan", A.ABSDIFF, 128)):
+            a = I.uniform_f32(81, 4096 * dd).reshape(4096, dd)
+            b = I.uniform_f32(82, 4096 * dd).reshape(4096, dd)
+            ap = S.Allpairs(c, z, S.F32, S.F32, reduce=A.ADD)
+            ma, mb = S.Matrix.from_numpy(c, a), S.Matrix.from_numpy(c, b)
+            o = ap(ma, mb)
+            ms = timeit(lambda: ap(ma, mb, out=o), reps=5)
+            cg = o.to_numpy()
+            fn = O.AP_DOT if z == A.MULT else O.AP_MANHATTAN
+            ok = np.array_equal(cg[:16, :40], O.allpairs(fn, a[:16], b[:40]))
+            tf = 2.0 * 4096 * 4096 * dd / (ms / 1e3) / 1e12
+            print(f"allpairs {name:9s} tile={tile}: {ms:.4f} ms  {tf:.2f} TFLOP/s  bitexact={ok}", flush=True)
+        c.finalize()
+
+
 def mandel():
     """MANDEL_CFGS="fn,block,unroll,interleave;..." (fn: plain | unroll4)"""
     grid = I.mandel_grid(3072, 4096)
