@@ -73,3 +73,18 @@ def test_size_mismatch(ctx, sk):
         sk["man"](S.Matrix.from_numpy(ctx, np.zeros((3, 4), np.float32)),
                   S.Matrix.from_numpy(ctx, np.zeros((3, 5), np.float32)))
     assert e.value.name == "SIZE_MISMATCH"
+
+
+@pytest.mark.parametrize("tile", [4, 8])
+def test_forced_tile_widths_bitexact(ctx, sk, tile):
+    """both 128-row kernels (128 x 64 and 128 x 128 tiles of C) agree with the oracle"""
+    ctx.set_option("ap_tile", tile)
+    try:
+        for n, m, d in ((130, 200, 64), (257, 129, 100), (5, 300, 4)):
+            a = I.uniform_f32(85, n * d).reshape(n, d)
+            b = I.uniform_f32(86, m * d).reshape(m, d)
+            ma, mb = S.Matrix.from_numpy(ctx, a), S.Matrix.from_numpy(ctx, b)
+            assert np.array_equal(sk["dot_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_DOT, a, b))
+            assert np.array_equal(sk["man_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_MANHATTAN, a, b))
+    finally:
+        ctx.set_option("ap_tile", 0)
