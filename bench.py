@@ -226,12 +226,14 @@ def bench_mandelbrot(args, D: Dist, P: dict):
     # user-side tuning (the paper's optional work-group size):
     # 1024-thread blocks, one 4-pixel chunk per thread, warp-interleaved pixels
     # (lanes of a warp iterate neighbouring pixels: less idle-lane time); the
-    # customising function checks the escape once per 8 iterations and replays
-    # the block (bit-identical counts).  Swept: profiles/sweeps/sweep18-19.
+    # customising function tests the escape on the end state of each block of 12
+    # iterations (the orbit grows monotonically after an escape) and replays a
+    # suspicious block exactly (bit-identical counts; apps.mandelbrot_blocktest).
+    # Swept: profiles/sweeps/sweep18-19, sweep24.
     ctx.set_option("block_threads", 1024)
     ctx.set_option("map_unroll", 1)
     ctx.set_option("map_interleave", 1)
-    m = S.Map(ctx, A.mandelbrot_unrolled(MAX_ITER, 8), S.F32X2, S.U32)
+    m = S.Map(ctx, A.mandelbrot_blocktest(MAX_ITER, 12), S.F32X2, S.U32)
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
     ctx.set_option("map_interleave", 0)

@@ -29,7 +29,7 @@ def test_mandelbrot_full_image_bitexact(ctx):
     ctx.set_option("block_threads", 1024)
     ctx.set_option("map_unroll", 1)
     ctx.set_option("map_interleave", 1)
-    m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
+    m = S.Map(ctx, A.mandelbrot_blocktest(1000, 12), S.F32X2, S.U32)
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
     ctx.set_option("map_interleave", 0)

@@ -41,10 +41,30 @@ def test_map_zip_interleaved(ctx, n):
     assert np.array_equal(z.to_numpy(), O.zip_(O.OZ_ADD_F32, x, y))
 
 
+@pytest.mark.parametrize("block", [1, 7, 12, 16])
+def test_mandelbrot_blocktest_exact(ctx, block, golden):
+    """the amortised escape test (apps.mandelbrot_blocktest) gives the oracle's
+    counts: a coarse grid of the A22 window, the hand-derived golden points
+    (including c = -2, whose orbit stays at |z| = 2 exactly), points just outside
+    |c| = 2 in the window's corners, and MAX values that are not multiples of the
+    block"""
+    gp = np.array(golden("mandelbrot_points.txt")[None], np.float64)   # re, im, count (MAX 1000)
+    pts = gp[:, :2].astype(np.float32)
+    grid = I.mandel_grid(48, 64)
+    extra = np.array([[-2.0, 1.125], [-2.0, -1.125], [0.99, 1.12], [-0.75, 0.1], [0.2501, 0.0]], np.float32)
+    cs = np.concatenate([pts, extra, grid.reshape(-1, 2)])
+    for mx in (1000, 37):
+        m = S.Map(ctx, A.mandelbrot_blocktest(mx, block), S.F32X2, S.U32)
+        got = m(S.Matrix(ctx, S.F32X2, 1, cs.shape[0]).copy_in(cs[None])).to_numpy().ravel()
+        assert np.array_equal(got, O.mandelbrot(cs[None], mx)[0].ravel()), (block, mx)
+        if mx == 1000:
+            assert np.array_equal(got[:len(gp)], gp[:, 2].astype(np.uint32))
+
+
 def test_mandelbrot_interleaved(ctx):
     R, C = 96, 128
     grid = I.mandel_grid(R, C)      # a coarse 96 x 128 view of the A22 window
-    m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
+    m = S.Map(ctx, A.mandelbrot_blocktest(1000, 12), S.F32X2, S.U32)
     got = m(S.Matrix(ctx, S.F32X2, R, C).copy_in(grid)).to_numpy()
     ref, _ = O.mandelbrot(grid, 1000)
     assert np.array_equal(got, ref)

@@ -19,12 +19,13 @@ from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
 
 def main(which: str, reps: int = 3):
     ctx = S.Context(1)
+    ctx.set_option("xfer_chunks", 1)   # one launch per call: the captured kernel is the bench step's
     if which == "mandel":
         # the bench's configuration
         ctx.set_option("block_threads", 1024)
         ctx.set_option("map_unroll", 1)
         ctx.set_option("map_interleave", 1)
-        m = S.Map(ctx, A.mandelbrot_unrolled(1000, 8), S.F32X2, S.U32)
+        m = S.Map(ctx, A.mandelbrot_blocktest(1000, 12), S.F32X2, S.U32)
         x = S.Matrix(ctx, S.F32X2, 3072, 4096).copy_in(I.mandel_grid(3072, 4096))
         o = m(x)
         for _ in range(reps):

@@ -128,7 +128,12 @@ def mandel():
     cfgs = [t.split(",") for t in os.environ.get("MANDEL_CFGS", "unroll4,512,2,0").split(";")]
     for name, bt, un, il in cfgs:
         bt, un, il = int(bt), int(un), int(il)
-        src = A.mandelbrot(1000) if name == "plain" else A.mandelbrot_unrolled(1000, int(name[6:] or 4))
+        if name == "plain":
+            src = A.mandelbrot(1000)
+        elif name.startswith("btest"):
+            src = A.mandelbrot_blocktest(1000, int(name[5:] or 8))
+        else:
+            src = A.mandelbrot_unrolled(1000, int(name[6:] or 4))
         c = ctx_with({"block_threads": bt, "map_unroll": un, "map_interleave": il})
         m = S.Map(c, src, S.F32X2, S.U32)
         x = S.Matrix(c, S.F32X2, 3072, 4096).copy_in(grid)
