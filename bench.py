@@ -119,11 +119,20 @@ class Dist:
         # collective host reads, max over ranks) even at world size 1, so that it
         # can be exercised on a single GPU
         self.force = os.environ.get("SKL_BENCH_FORCE_DIST", "0") == "1"
+        # SKL_COMM=shm (several ranks on one GPU, testing only): the library's
+        # shared-memory transport and a gloo process group for the bench plumbing
+        self.gloo = os.environ.get("SKL_COMM", "") == "shm"
+        if self.gloo:
+            import torch
+            self.local %= max(1, torch.cuda.device_count())   # ranks may share a GPU
         if self.world > 1 or self.force:
             import torch
             import torch.distributed as dist
             torch.cuda.set_device(self.local)
-            dist.init_process_group("nccl", device_id=torch.device("cuda", self.local))
+            if self.gloo:
+                dist.init_process_group("gloo")
+            else:
+                dist.init_process_group("nccl", device_id=torch.device("cuda", self.local))
             self.pg = dist
 
     def barrier(self):
@@ -134,7 +143,7 @@ class Dist:
         if not self.pg:
             return v
         import torch
-        t = torch.tensor([v], dtype=torch.float64, device="cuda")
+        t = torch.tensor([v], dtype=torch.float64, device="cpu" if self.gloo else "cuda")
         self.pg.all_reduce(t, op=self.pg.ReduceOp.MAX)
         return float(t.item())
 
@@ -142,7 +151,7 @@ class Dist:
         if not self.pg:
             return v
         import torch
-        t = torch.tensor([v], dtype=torch.float64, device="cuda")
+        t = torch.tensor([v], dtype=torch.float64, device="cpu" if self.gloo else "cuda")
         self.pg.all_reduce(t)
         return float(t.item())
 

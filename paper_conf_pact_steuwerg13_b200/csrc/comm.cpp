@@ -8,9 +8,17 @@
 // ncclSend / ncclRecv halves that touch it, so matching pairs are issued in the
 // same order on both sides (NCCL matches p2p operations per peer in order).
 #include <dlfcn.h>
+#include <fcntl.h>
 #include <nccl.h>
+#include <sys/mman.h>
+#include <unistd.h>
 
+#include <atomic>
+#include <chrono>
+#include <cstdlib>
 #include <mutex>
+#include <random>
+#include <thread>
 
 #include "skl_internal.h"
 
@@ -60,7 +68,116 @@ void nccl_check(ncclResult_t r, const char* what) {
 }
 }  // namespace
 
+// ---- host shared-memory loopback transport (SKL_COMM=shm) ------------------
+// Test transport for the one-process-per-GPU mode with several processes on ONE
+// GPU (NCCL refuses two ranks on one device; SURVEY §4 T3 "loopback backend").
+// Every rank walks the same canonical transfer list in the same order: a send
+// copies the units device -> a POSIX shared-memory object and publishes a
+// per-(src, dst) sequence number; the matching receive waits for it and copies
+// shared memory -> device.  Sends never block, so the list order cannot
+// deadlock.  Slow (two host copies), correct, and never used unless asked for.
+namespace {
+struct ShmComm {
+  std::string name;
+  int rank = 0, world = 1;
+  std::atomic<unsigned long long>* seq = nullptr;  // world x world published counters
+  size_t ctl_bytes = 0;
+  std::vector<unsigned long long> sent, recvd;     // this rank's counters per pair
+};
+bool shm_mode() {
+  const char* v = std::getenv("SKL_COMM");
+  return v && std::string(v) == "shm";
+}
+std::string shm_data_name(const ShmComm& c, int src, int dst, unsigned long long k) {
+  return c.name + "_" + std::to_string(src) + "_" + std::to_string(dst) + "_" + std::to_string(k);
+}
+void shm_send(Ctx* ctx, ShmComm& c, const void* dptr, size_t bytes, int dst) {
+  Device& L = ctx->D(ctx->first_local);
+  const size_t pair = (size_t)c.rank * c.world + dst;
+  const unsigned long long k = c.sent[pair]++;
+  const std::string nm = shm_data_name(c, c.rank, dst, k);
+  const int fd = shm_open(nm.c_str(), O_CREAT | O_RDWR | O_TRUNC, 0600);
+  if (fd < 0) fail(SKL_ERR_NCCL, "shm transport: shm_open failed for " + nm);
+  if (ftruncate(fd, (off_t)std::max<size_t>(bytes, 1)) != 0) {
+    close(fd);
+    fail(SKL_ERR_NCCL, "shm transport: ftruncate failed");
+  }
+  void* h = mmap(nullptr, std::max<size_t>(bytes, 1), PROT_READ | PROT_WRITE, MAP_SHARED, fd, 0);
+  close(fd);
+  if (h == MAP_FAILED) fail(SKL_ERR_NCCL, "shm transport: mmap failed");
+  SKL_CUDA(cudaMemcpyAsync(h, dptr, bytes, cudaMemcpyDeviceToHost, L.stream));  // after its producers
+  SKL_CUDA(cudaStreamSynchronize(L.stream));
+  munmap(h, std::max<size_t>(bytes, 1));
+  c.seq[pair].store(k + 1, std::memory_order_release);
+}
+void shm_recv(Ctx* ctx, ShmComm& c, void* dptr, size_t bytes, int src) {
+  Device& L = ctx->D(ctx->first_local);
+  const size_t pair = (size_t)src * c.world + c.rank;
+  const unsigned long long k = c.recvd[pair]++;
+  const auto t0 = std::chrono::steady_clock::now();
+  while (c.seq[pair].load(std::memory_order_acquire) <= k) {
+    if (std::chrono::steady_clock::now() - t0 > std::chrono::seconds(300))
+      fail(SKL_ERR_NCCL, "shm transport: timed out waiting for rank " + std::to_string(src));
+    std::this_thread::sleep_for(std::chrono::microseconds(50));
+  }
+  const std::string nm = shm_data_name(c, src, c.rank, k);
+  const int fd = shm_open(nm.c_str(), O_RDONLY, 0600);
+  if (fd < 0) fail(SKL_ERR_NCCL, "shm transport: missing " + nm);
+  void* h = mmap(nullptr, std::max<size_t>(bytes, 1), PROT_READ, MAP_SHARED, fd, 0);
+  close(fd);
+  if (h == MAP_FAILED) fail(SKL_ERR_NCCL, "shm transport: mmap failed");
+  SKL_CUDA(cudaMemcpyAsync(dptr, h, bytes, cudaMemcpyHostToDevice, L.stream));
+  SKL_CUDA(cudaStreamSynchronize(L.stream));
+  munmap(h, std::max<size_t>(bytes, 1));
+  shm_unlink(nm.c_str());
+}
+void shm_init(Ctx* ctx, const void* id128) {
+  auto* c = new ShmComm();
+  c->name = std::string((const char*)id128, strnlen((const char*)id128, 127));
+  c->rank = ctx->rank;
+  c->world = ctx->world;
+  c->ctl_bytes = (size_t)c->world * c->world * sizeof(unsigned long long);
+  const std::string ctl = c->name + "_ctl";
+  const int fd = shm_open(ctl.c_str(), O_CREAT | O_RDWR, 0600);
+  if (fd < 0) {
+    delete c;
+    fail(SKL_ERR_NCCL, "shm transport: cannot open " + ctl);
+  }
+  if (ftruncate(fd, (off_t)c->ctl_bytes) != 0) {  // same size on every rank: idempotent
+    close(fd);
+    delete c;
+    fail(SKL_ERR_NCCL, "shm transport: ftruncate failed");
+  }
+  void* h = mmap(nullptr, c->ctl_bytes, PROT_READ | PROT_WRITE, MAP_SHARED, fd, 0);
+  close(fd);
+  if (h == MAP_FAILED) {
+    delete c;
+    fail(SKL_ERR_NCCL, "shm transport: mmap failed");
+  }
+  c->seq = (std::atomic<unsigned long long>*)h;
+  c->sent.assign((size_t)c->world * c->world, 0);
+  c->recvd.assign((size_t)c->world * c->world, 0);
+  ctx->shm_comm = c;
+}
+void shm_destroy(Ctx* ctx) {
+  auto* c = (ShmComm*)ctx->shm_comm;
+  if (!c) return;
+  munmap((void*)c->seq, c->ctl_bytes);
+  if (c->rank == 0) shm_unlink((c->name + "_ctl").c_str());
+  delete c;
+  ctx->shm_comm = nullptr;
+}
+}  // namespace
+
 void nccl_get_unique_id(void* out128) {
+  if (shm_mode()) {
+    std::random_device rd;
+    const std::string nm = "/skl_" + std::to_string((long long)getpid()) + "_" + std::to_string(rd()) +
+                           std::to_string(rd());
+    std::memset(out128, 0, 128);
+    std::memcpy(out128, nm.c_str(), std::min<size_t>(nm.size(), 127));
+    return;
+  }
   ncclUniqueId id;
   nccl_check(nccl()->getUniqueId(&id), "ncclGetUniqueId");
   std::memcpy(out128, &id, sizeof(id));
@@ -68,6 +185,10 @@ void nccl_get_unique_id(void* out128) {
 
 void nccl_init(Ctx* ctx, const void* id128) {
   if (!id128) fail(SKL_ERR_INVALID_ARG, "multi-process mode needs the NCCL unique id");
+  if (shm_mode()) {
+    shm_init(ctx, id128);
+    return;
+  }
   ncclUniqueId id;
   std::memcpy(&id, id128, sizeof(id));
   ctx->set_device(ctx->first_local);
@@ -77,6 +198,7 @@ void nccl_init(Ctx* ctx, const void* id128) {
 }
 
 void nccl_destroy(Ctx* ctx) {
+  shm_destroy(ctx);
   if (ctx->nccl_comm) nccl()->commDestroy((ncclComm_t)ctx->nccl_comm);
   ctx->nccl_comm = nullptr;
 }
@@ -100,6 +222,25 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
       ctx->p2p += (long long)bytes;
     }
     barrier_streams(ctx);
+    return;
+  }
+  if (ctx->shm_comm) {
+    auto* sc = (ShmComm*)ctx->shm_comm;
+    Device& L = ctx->D(ctx->first_local);
+    ctx->set_device(ctx->first_local);
+    for (const Transfer& t : tr) {
+      const size_t bytes = t.n * unit_bytes;
+      if (bytes == 0) continue;
+      const bool src_here = ctx->is_local(t.src), dst_here = ctx->is_local(t.dst);
+      if (src_here && dst_here) {
+        SKL_CUDA(cudaMemcpyAsync(p.dst(t), p.src(t), bytes, cudaMemcpyDeviceToDevice, L.stream));
+      } else if (src_here) {
+        shm_send(ctx, *sc, p.src(t), bytes, t.dst);
+        ctx->p2p += (long long)bytes;
+      } else if (dst_here) {
+        shm_recv(ctx, *sc, p.dst(t), bytes, t.src);
+      }
+    }
     return;
   }
   NcclApi* a = nccl();

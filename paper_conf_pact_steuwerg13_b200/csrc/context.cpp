@@ -188,7 +188,7 @@ void ctx_destroy(Ctx* c) {
       extern void program_unload(Program*);
       program_unload(kv.second.get());
     }
-  if (c->nccl_comm) nccl_destroy(c);
+  if (c->nccl_comm || c->shm_comm) nccl_destroy(c);
   for (auto& d : c->dev) {
     cudaSetDevice(d.phys);
     if (d.ev) cudaEventDestroy(d.ev);

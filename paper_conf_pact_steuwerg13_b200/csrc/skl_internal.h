@@ -117,6 +117,7 @@ struct Ctx {
   bool capturing = false;      // a CUDA graph capture is open on the device stream
   int rank = 0, world = 1;
   void* nccl_comm = nullptr;   // ncclComm_t
+  void* shm_comm = nullptr;    // host shared-memory loopback transport (SKL_COMM=shm, tests)
   std::vector<Device> dev;     // local devices, index g - first_local
   std::vector<TypeInfo> types; // index = skl_type (builtins first)
   std::set<Cont*> conts;
