@@ -197,6 +197,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "scan_minb") {
       if (value < 1 || value > 32) fail(SKL_ERR_INVALID_ARG, "scan_minb in [1,32]");
       c->scan_minb = (int)value;
+    } else if (k == "mo_persist") {
+      c->mo_persist = value ? 1 : 0;
     } else if (k == "mo_minb") {
       if (value < 0 || value > 32) fail(SKL_ERR_INVALID_ARG, "mo_minb in [0,32]");
       c->mo_minb = (int)value;

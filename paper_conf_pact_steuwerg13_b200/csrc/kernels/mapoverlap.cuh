@@ -61,39 +61,47 @@ __device__ __forceinline__ void skl_mo_store(SKL_TOUT* o, const SklMoRes& v, boo
 #ifndef SKL_MO_MINB
 #define SKL_MO_MINB 1
 #endif
-extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
-skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
-         long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
-         SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
-  __shared__ __align__(16) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
-  // 32-bit row / column arithmetic (the host guarantees R, C < 2^31); 64-bit
-  // only where a row index is scaled to an element offset
-  const int Ri = (int)R, Ci = (int)C, rb = (int)r_begin, re = (int)r_end;
-  const int irow0 = (int)in_row0, orow0 = (int)out_row0;
-  const int r0 = rb + (int)blockIdx.y * SKL_TH;
-  const int c0 = (int)blockIdx.x * SKL_TW;
-  // ---- stage rows r0-d .. r0+TH+d-1, columns c0-A .. c0+TW+A-1
+
+// Geometry of one launch: 32-bit row / column arithmetic (the host guarantees
+// R, C < 2^31); 64-bit only where a row index is scaled to an element offset.
+struct SklMoGeo {
+  int Ri, Ci, rb, re, irow0, orow0, hd;
+};
+
+// Stage the input window of the tile at (r0, c0) into `tile`: rows r0-d ..
+// r0+TH+d-1, columns c0-A .. c0+TW+A-1.  Issues cp.async copies (the caller
+// commits / waits) and plain stores for border chunks.
+__device__ __forceinline__ void skl_mo_stage(SKL_TIN* tile, const SKL_TIN* __restrict__ in, const SklMoGeo& G,
+                                             int r0, int c0, SKL_TIN neutral, int vec_ok) {
+  const int Ri = G.Ri, Ci = G.Ci;
   const bool interior = vec_ok && c0 - SKL_A >= 0 && c0 + SKL_TW + SKL_A <= Ci && r0 - SKL_D >= 0 &&
-                        r0 + SKL_TH + SKL_D <= Ri && r0 + SKL_TH <= re;
+                        r0 + SKL_TH + SKL_D <= Ri && r0 + SKL_TH <= G.re;
   if (interior) {
-    // block-uniform fast path: every staged chunk is an in-range 16-byte copy;
-    // incremental (row, chunk) walk, no per-chunk bounds or boundary logic
-    const SKL_TIN* src = in + (long)(r0 - SKL_D - irow0) * Ci + (c0 - SKL_A);
-    const unsigned sbase = (unsigned)__cvta_generic_to_shared(tile);
-    int i = threadIdx.x / SKL_CPR, jc = threadIdx.x % SKL_CPR;
+    // block-uniform fast path: every staged chunk is an in-range 16-byte copy.
+    // The tile is dense in shared memory (SKL_PITCH = SKL_CPR chunks), so chunk
+    // q lands at byte 16 q; its global address advances by a constant per step
+    // (plus one row's remainder when the column wraps)
+    const int jc0 = threadIdx.x % SKL_CPR;
+    const char* gp = (const char*)(in + (long)(r0 - SKL_D - G.irow0 + (int)threadIdx.x / SKL_CPR) * Ci +
+                                   (c0 - SKL_A) + jc0 * SKL_EPC);
+    unsigned sa = (unsigned)__cvta_generic_to_shared(tile) + 16u * threadIdx.x;
+    const long rowb = (long)Ci * (long)sizeof(SKL_TIN);
+    const long step = (long)(SKL_BLOCK / SKL_CPR) * rowb + (long)(SKL_BLOCK % SKL_CPR) * 16;
+    const long wrap = rowb - (long)SKL_CPR * 16;
+    int jc = jc0;
 #pragma unroll 4
     for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
-      const unsigned sa = sbase + (unsigned)((i * SKL_PITCH + jc * SKL_EPC) * (int)sizeof(SKL_TIN));
-      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa),
-                   "l"(src + (long)i * Ci + jc * SKL_EPC) : "memory");
-      i += SKL_BLOCK / SKL_CPR;
+      asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(gp) : "memory");
+      sa += 16u * SKL_BLOCK;
+      gp += step;
       jc += SKL_BLOCK % SKL_CPR;
       if (jc >= SKL_CPR) {
         jc -= SKL_CPR;
-        ++i;
+        gp += wrap;
       }
     }
-  } else
+    return;
+  }
   for (int q = threadIdx.x; q < SKL_SROWS * SKL_CPR; q += SKL_BLOCK) {
     const int i = q / SKL_CPR, jc = q - i * SKL_CPR;
     int gr = r0 - SKL_D + i;
@@ -103,12 +111,12 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
     gr = gr < 0 ? 0 : (gr > Ri - 1 ? Ri - 1 : gr);
 #endif
     SKL_TIN* dst = tile + i * SKL_PITCH + jc * SKL_EPC;
-    if (r0 - SKL_D + i >= re + SKL_D) {  // below the last output row's window: unused
+    if (r0 - SKL_D + i >= G.re + SKL_D) {  // below the last output row's window: unused
 #pragma unroll
       for (int e = 0; e < SKL_EPC; ++e) dst[e] = neutral;
       continue;
     }
-    const SKL_TIN* row = in + (long)(gr - irow0) * Ci;
+    const SKL_TIN* row = in + (long)(gr - G.irow0) * Ci;
     if (vec_ok && (SKL_BOUNDARY == 1 || row_in) && gc0 >= 0 && gc0 + SKL_EPC <= Ci) {
       // asynchronous 16-byte global->shared copy (LDGSTS), no register round trip
       const unsigned sa = (unsigned)__cvta_generic_to_shared(dst);
@@ -129,21 +137,24 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
       }
     }
   }
-  asm volatile("cp.async.wait_all;" ::: "memory");
-  __syncthreads();
-  // ---- apply f to a SKL_RH x SKL_CW block per thread
+}
+
+// Apply f to the staged tile: a SKL_RH x SKL_CW block of outputs per thread.
+__device__ __forceinline__ void skl_mo_apply(const SKL_TIN* tile, SKL_TOUT* __restrict__ out, const SklMoGeo& G,
+                                             int r0, int c0, int vec_ok, SKL_TOUT* __restrict__ push_up,
+                                             SKL_TOUT* __restrict__ push_down) {
+  const int Ci = G.Ci, rb = G.rb, re = G.re, hdi = G.hd;
   const int ty = threadIdx.x / (SKL_TW / SKL_CW), tx = threadIdx.x % (SKL_TW / SKL_CW);
   const int cc = c0 + tx * SKL_CW;
   const int ncols = Ci - cc;                        // columns left in the row from cc
   const bool full = vec_ok && ncols >= SKL_CW;      // whole packed store in range
   const int rt = r0 + ty * SKL_RH;                  // this thread's first row
-  SKL_TOUT* o = out + (long)(rt - orow0) * Ci + cc;
+  SKL_TOUT* o = out + (long)(rt - G.orow0) * Ci + cc;
   // fused halo push: the first / last hd rows of this device's
   // block also go into the neighbours' halo rows (peer memory), so the next
   // overlap read needs no exchange.  Block-uniform; the common path below
   // carries none of it (live registers matter: f may call the IEEE sqrt
   // subroutine).
-  const int hdi = (int)hd;
   if ((push_up && r0 < rb + hdi) || (push_down && r0 + SKL_TH > re - hdi)) {
 #pragma unroll
     for (int i = 0; i < SKL_RH; ++i) {
@@ -168,6 +179,52 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
     // f may declare a non-const pointer (Listing 1.2: "float func(float* m_in)")
     for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
     if (rt + i < re) skl_mo_store(o + (long)i * Ci, res, full, ncols);
+  }
+}
+
+// One block per tile (grid = tiles_x x tiles_y).
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
+skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
+         long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
+         SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd) {
+  __shared__ __align__(16) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
+  const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
+  const int r0 = G.rb + (int)blockIdx.y * SKL_TH;
+  const int c0 = (int)blockIdx.x * SKL_TW;
+  skl_mo_stage(tile, in, G, r0, c0, neutral, vec_ok);
+  asm volatile("cp.async.wait_all;" ::: "memory");
+  __syncthreads();
+  skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
+  (void)in_rows;
+}
+
+// Persistent variant: a grid of resident blocks walks the tiles (t = blockIdx.x,
+// + gridDim.x, ...) with two shared-memory buffers, staging tile k+1 while
+// applying f to tile k, so the load latency of a tile hides behind the
+// computation of the previous one (ncu of the one-tile-per-block kernel: the
+// top stall was the wait for the tile, with only 4 blocks resident per SM).
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
+skl_mo2d_p(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* __restrict__ out,
+           long out_row0, long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok,
+           SKL_TOUT* __restrict__ push_up, SKL_TOUT* __restrict__ push_down, long hd, int tiles_x, int ntiles) {
+  extern __shared__ __align__(16) unsigned char skl_mo_dyn[];
+  SKL_TIN* buf[2] = {(SKL_TIN*)skl_mo_dyn, (SKL_TIN*)skl_mo_dyn + SKL_SROWS * SKL_PITCH};
+  const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
+  int t = blockIdx.x;
+  if (t >= ntiles) return;
+  skl_mo_stage(buf[0], in, G, G.rb + (t / tiles_x) * SKL_TH, (t % tiles_x) * SKL_TW, neutral, vec_ok);
+  asm volatile("cp.async.commit_group;" ::: "memory");
+  for (int k = 0; t < ntiles; ++k, t += gridDim.x) {
+    const int tn = t + gridDim.x;
+    if (tn < ntiles)
+      skl_mo_stage(buf[(k + 1) & 1], in, G, G.rb + (tn / tiles_x) * SKL_TH, (tn % tiles_x) * SKL_TW, neutral,
+                   vec_ok);
+    asm volatile("cp.async.commit_group;" ::: "memory");
+    asm volatile("cp.async.wait_group 1;" ::: "memory");  // tile t has landed
+    __syncthreads();
+    skl_mo_apply(buf[k & 1], out, G, G.rb + (t / tiles_x) * SKL_TH, (t % tiles_x) * SKL_TW, vec_ok, push_up,
+                 push_down);
+    __syncthreads();  // buf[k & 1] is restaged two tiles later
   }
   (void)in_rows;
 }

@@ -890,7 +890,20 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                       s->neutral.data(), &vec_ok, &pu, &pd, &hd};
       const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
                       (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
-      launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(s->block), 0, args);
+      if (ctx->mo_persist) {
+        // resident blocks walk the tiles with two staging buffers (load of tile
+        // k+1 overlaps f on tile k)
+        const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;
+        const size_t smem = 2 * tile_bytes;
+        int tiles_x = (int)grid.x, ntiles = (int)(grid.x * grid.y);
+        const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_mo2d_p", s->block, smem));
+        const size_t pgrid = std::min((size_t)ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
+        void* pargs[] = {(void*)&pin, &in_row0, &in_rows, &pout, &out_row0, &R, &C, &rb, &re,
+                         s->neutral.data(), &vec_ok, &pu, &pd, &hd, &tiles_x, &ntiles};
+        launch(ctx, g, s->prog, "skl_mo2d_p", dim3((unsigned)pgrid), dim3(s->block), smem, pargs);
+      } else {
+        launch(ctx, g, s->prog, "skl_mo2d", grid, dim3(s->block), 0, args);
+      }
     }
   } else {
     // vector form: compile the 1-D variant once

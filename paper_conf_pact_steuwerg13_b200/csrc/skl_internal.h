@@ -136,6 +136,7 @@ struct Ctx {
   int scan_lbw = 1;            // Scan look-back: predecessors watched per thread (2-6 measured slower)
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
+  int mo_persist = 0;          // MapOverlap 2-D: persistent blocks, double-buffered tiles
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)

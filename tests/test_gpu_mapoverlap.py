@@ -117,3 +117,23 @@ def test_debug_bounds_flags_access_beyond_d():
         x = np.ones((8, 8), np.float32)
         assert np.array_equal(ok(S.Matrix.from_numpy(c, x)).to_numpy(),
                               O.mapoverlap2d(O.OS_BOX3, x, 1, O.OB_NEUTRAL, 0.0))
+
+
+@pytest.mark.parametrize("shape", [(5, 9), (131, 257), (600, 1030)])
+def test_persistent_variant_bitexact(shape):
+    """mo_persist=1 (resident blocks walking the tiles with two staging buffers;
+    measured slower on B200, kept selectable) gives the oracle's results"""
+    require_gpu()
+    c = S.Context(1)
+    try:
+        c.set_option("mo_persist", 1)
+        img8 = I.image_u8(I.SEED_SOBEL, *shape)
+        sob = S.MapOverlap(c, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+        assert np.array_equal(sob(S.Matrix.from_numpy(c, img8)).to_numpy(),
+                              O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0))
+        imgf = I.image_f32(I.SEED_GAUSS, *shape)
+        gau = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+        assert np.array_equal(gau(S.Matrix.from_numpy(c, imgf)).to_numpy(),
+                              O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0))
+    finally:
+        c.finalize()

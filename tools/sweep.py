@@ -214,7 +214,8 @@ def mo():
     cfgs = [tuple(int(x) for x in t.split(",")) for t in os.environ.get("MO_CFGS", "256,0,0,0").split(";")]
     for cfg in cfgs:
         bt, rh, cw8, cw32 = cfg[:4]
-        c = ctx_with({"block_threads": bt, "mo_minb": cfg[4] if len(cfg) > 4 else 0})
+        c = ctx_with({"block_threads": bt, "mo_minb": cfg[4] if len(cfg) > 4 else 0,
+                      "mo_persist": cfg[5] if len(cfg) > 5 else 0})
         for name, src, t, d, bnd, img in (("ident_u8", A.IDENT2D_U8, S.U8, 1, S.NEUTRAL, img8),
                                           ("sobel", A.SOBEL, S.U8, 1, S.NEUTRAL, img8),
                                           ("ident_f32", A.IDENT2D, S.F32, 2, S.NEAREST, imgf),
@@ -232,7 +233,7 @@ def mo():
                 ref = (O.mapoverlap2d(O.OS_SOBEL, sub, 1, O.OB_NEUTRAL, 0) if name == "sobel"
                        else O.mapoverlap2d(O.OS_GAUSS5, sub, 2, O.OB_NEAREST, 0.0))[10:74]
                 ok = f" bitexact={np.array_equal(o.to_numpy()[4000:4064], ref)}"
-            print(f"mo {name:9s} block={bt} rh={rh} cw={cw8 if t == S.U8 else cw32} minb={cfg[4] if len(cfg) > 4 else 0}: {ms:.4f} ms  "
+            print(f"mo {name:9s} block={bt} rh={rh} cw={cw8 if t == S.U8 else cw32} minb={cfg[4] if len(cfg) > 4 else 0} persist={cfg[5] if len(cfg) > 5 else 0}: {ms:.4f} ms  "
                   f"{bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s{ok}", flush=True)
             x.destroy()
             o.destroy()
