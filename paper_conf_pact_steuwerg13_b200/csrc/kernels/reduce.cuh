@@ -80,6 +80,9 @@ template <int RVEC, class Loader>
 __device__ __forceinline__ void skl_reduce_body(const Loader& ld, skl_u64 n, skl_u64 wseg,
                                                 SKL_T* partials, unsigned* counter, SKL_T* result) {
   SklOp op;
+  // a warp-tile is 32 lanes x RVEC elements of THIS instantiation (the scalar
+  // kernel, RVEC = 1, serves unaligned views)
+  constexpr skl_u64 RT = 32 * RVEC;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const skl_u64 w = (skl_u64)blockIdx.x * SKL_NW + warp;
   const skl_u64 lo = w * wseg;
@@ -89,11 +92,11 @@ __device__ __forceinline__ void skl_reduce_body(const Loader& ld, skl_u64 n, skl
   skl_u64 t = lo;
   // fast path: SKL_RU full warp-tiles, no per-tile branches, so all loads of the
   // iteration are issued before the first use (memory-level parallelism)
-  for (; t + (skl_u64)SKL_RTILE * SKL_RU <= hi; t += (skl_u64)SKL_RTILE * SKL_RU) {
+  for (; t + RT * SKL_RU <= hi; t += RT * SKL_RU) {
     SKL_T x[SKL_RU][RVEC];
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u)
-      ld.template load<RVEC>(t + (skl_u64)u * SKL_RTILE + (skl_u64)lane * RVEC, RVEC, x[u]);
+      ld.template load<RVEC>(t + (skl_u64)u * RT + (skl_u64)lane * RVEC, RVEC, x[u]);
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u) {
       SKL_T v = x[u][0];
@@ -106,25 +109,25 @@ __device__ __forceinline__ void skl_reduce_body(const Loader& ld, skl_u64 n, skl
     }
   }
   // ragged end of the segment
-  for (; t < hi; t += (skl_u64)SKL_RTILE * SKL_RU) {
+  for (; t < hi; t += RT * SKL_RU) {
     SKL_T x[SKL_RU][RVEC];
     int cnt[SKL_RU];
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u) {
-      const skl_u64 e = t + (skl_u64)u * SKL_RTILE + (skl_u64)lane * RVEC;
+      const skl_u64 e = t + (skl_u64)u * RT + (skl_u64)lane * RVEC;
       cnt[u] = e >= hi ? 0 : (hi - e >= (skl_u64)RVEC ? RVEC : (int)(hi - e));
       ld.template load<RVEC>(e, cnt[u], x[u]);
     }
 #pragma unroll
     for (int u = 0; u < SKL_RU; ++u) {
-      const skl_u64 tl = t + (skl_u64)u * SKL_RTILE;
+      const skl_u64 tl = t + (skl_u64)u * RT;
       if (tl >= hi) break;
       SKL_T v = x[u][0];
 #pragma unroll
       for (int k = 1; k < RVEC; ++k)
         if (k < cnt[u]) v = op(v, x[u][k]);
       const skl_u64 rem = hi - tl;
-      const int nv = rem >= (skl_u64)SKL_RTILE ? 32 : (int)((rem + RVEC - 1) / RVEC);
+      const int nv = rem >= RT ? 32 : (int)((rem + RVEC - 1) / RVEC);
       v = skl_warp_fold(v, nv, op);
       v = skl_shfl(v, 0);
       acc = has ? op(acc, v) : v;

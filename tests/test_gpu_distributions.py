@@ -194,3 +194,22 @@ def test_lmosem_subset_small(ctx):
     assert rel_l2(fn.to_numpy(), fn_ref) <= 1e-4
     # invariant: sum f*c = #events with fp > 0
     assert abs(float(np.dot(f0.astype(np.float64), c.to_numpy().astype(np.float64))) - nhit) <= 1e-3 * nhit
+
+
+@pytest.mark.parametrize("n", [5, 4099, (1 << 20) + 7])
+def test_reduce_of_unaligned_parts(ctx, n):
+    """after overlap(1) -> block the parts keep their halo room, so device g's
+    first element sits 4 bytes into its buffer: Reduce takes the unaligned
+    (scalar) kernel, fused or not (found by tests/test_gpu_fuzz.py)"""
+    x = I.uniform_f32(63, n) - np.float32(0.25)
+    v = S.Vector.from_numpy(ctx, x).set_distribution(S.OVERLAP, 1)
+    v.set_distribution(S.BLOCK)
+    red = S.Reduce(ctx, A.SUM, S.F32)
+    ref = O.reduce_(O.OP_ADD_F32, x)
+    scale = float(np.abs(x).sum())
+    assert abs(float(red(v).scalar()) - ref) <= 1e-5 * scale
+    add = S.Zip(ctx, A.ADD, S.F32, S.F32, S.F32)
+    ref2 = O.reduce_(O.OP_ADD_F32, O.zip_(O.OZ_ADD_F32, x, x))
+    assert abs(float(red(add(v, v)).scalar()) - ref2) <= 1e-5 * 2 * scale
+    right = S.Reduce(ctx, A.RIGHT_F32, S.F32)
+    assert right(v).scalar() == x[-1]
