@@ -3,8 +3,9 @@
 every read.  It exercises the interplay of the state the library keeps per
 container: distributions and redistribution, lazy (deferred) Map/Zip results and
 their fusion into Reduce, chunked uploads consumed by Maps, pushed halos of
-MapOverlap outputs, host mirrors, in-place calls.  Bit-exact except the fp32
-Reduce (relative 1e-5)."""
+MapOverlap outputs, host mirrors, in-place calls, unaligned views (parts that
+keep halo room after overlap -> block), Scan and 1-D stencils.  Bit-exact except
+the fp32 Reduce and Scan (relative 1e-5)."""
 import numpy as np
 import pytest
 
@@ -35,6 +36,8 @@ def _program(G, seed, steps=60):
         add = S.Zip(ctx, A.ADD, S.F32, S.F32, S.F32)
         red = S.Reduce(ctx, A.SUM, S.F32)
         box = S.MapOverlap(ctx, A.BOX3, S.F32, S.F32, 1, S.NEAREST, 0.0)
+        box1 = S.MapOverlap(ctx, A.BOX1D, S.F32, S.F32, 1, S.NEAREST, 0.0)
+        scan = S.Scan(ctx, A.ADD, S.F32)
         n = SIZES[rng.integers(len(SIZES))]
         vecs = [S.Vector(ctx, S.F32, n) for _ in range(3)]
         shadow = [np.zeros(n, np.float32) for _ in range(3)]
@@ -47,7 +50,7 @@ def _program(G, seed, steps=60):
         dists = [(S.BLOCK, 0), (S.COPY, 0), (S.SINGLE, G - 1), (S.OVERLAP, 1), (S.BLOCK, 0)]
         log = []
         for step in range(steps):
-            op = int(rng.integers(11))
+            op = int(rng.integers(14))
             i, j, k = (int(x) for x in rng.integers(3, size=3))
             log.append((op, i, j, k))
             if op == 0:        # host write
@@ -100,6 +103,20 @@ def _program(G, seed, steps=60):
                 else:
                     d, a2 = dists[int(rng.integers(len(dists)))]
                     mat[i % 2].set_distribution(d, a2)
+            elif op == 11:     # Scan (fp32: relative L2 against the double oracle)
+                got = scan(vecs[i]).to_numpy().astype(np.float64)
+                ref = O.scan(O.OP_ADD_F32, shadow[i])
+                den = max(1e-30, float(np.linalg.norm(np.cumsum(np.abs(shadow[i].astype(np.float64))))))
+                assert float(np.linalg.norm(got - ref)) <= 1e-5 * den, log
+            elif op == 12:     # 1-D stencil into another vector
+                if i != j:
+                    box1(vecs[i], out=vecs[j])
+                    shadow[j] = O.mapoverlap1d(O.OS_BOX3, shadow[i], 1, O.OB_NEAREST, 0.0)
+            elif op == 13:     # a deferred chain materialised into an explicit output
+                if i == j:
+                    _no_overlap(vecs[i])
+                neg(sq(vecs[i]), out=vecs[j])
+                shadow[j] = O.map_(O.OM_NEG_F32, O.map_(O.OM_SQP1_F32, shadow[i]))
         for v, sh in zip(vecs, shadow):
             assert np.array_equal(v.to_numpy(), sh), log
         for m, sh in zip(mat, mshadow):
@@ -109,7 +126,7 @@ def _program(G, seed, steps=60):
 
 
 @pytest.mark.parametrize("G", [1, 2, 3])
-@pytest.mark.parametrize("seed", range(6))
+@pytest.mark.parametrize("seed", range(8))
 def test_random_programs(G, seed):
     require_gpu()
     _program(G, 1000 * G + seed)
