@@ -375,6 +375,20 @@ def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None):
             "algorithmic_bytes": bytes_per_step}
 
 
+def roof_l2(workload: str):
+    """L2-bound kernels (LM OSEM's gathers and vector atomics into an L2-resident
+    image): the fraction is ncu's lts__throughput of the committed capture.  A
+    random-access microbenchmark (tools/micro/l2_rates.cu, profiles/r01_l2_rates.txt)
+    is not a tight peak for a ray walk's partly local accesses, so no
+    bytes-per-second ratio is formed."""
+    pct = ncu_field(workload, "lts_pct_of_peak")
+    if pct is None:
+        return None
+    return {"bound": "l2", "achieved": round(pct, 1), "peak": 100.0, "unit": "% of L2 peak throughput",
+            "frac": round(pct / 100.0, 4), "source": "ncu lts__throughput.avg.pct_of_peak_sustained_elapsed, "
+            "committed capture (profiles/ncu_traffic.json)", "traffic": ncu_traffic(workload)}
+
+
 def bench_skeletons(args, D: Dist, P: dict, which):
     import torch
     from paper_conf_pact_steuwerg13_b200 import apps as A
@@ -731,6 +745,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                          "ms": round(ms, 4), "events_per_s": nev / (ms / 1e3), "map_ms": round(seg[0], 4),
                          "map_ms_generation_order": round(ms_raw, 4),
                          "visits_per_s_est": visits / (seg[0] / 1e3), "visits_est": visits,
+                         "roofline": roof_l2("lmosem"),
                          "rel_l2_c_sample": e, "check": "ok" if e <= 1e-4 else "FAIL"}
         for x in (ev, ev_raw, f, c, fn, evs):
             x.destroy()

@@ -2,6 +2,7 @@
 key counters) for bench.py's roofline.traffic field.
 
   python tools/ncu_traffic.py gpurun_out/prof_mandel_bench.ncu-rep:skl_map_vec:mandelbrot ...
+  python tools/ncu_traffic.py profiles/r01_ncu_raw_lmosem.csv:skl_map_vec:lmosem   (raw page CSV)
 
 Writes/updates profiles/ncu_traffic.json: {workload: {kernel, bytes_per_launch,
 dram_read, dram_write, duration_ns, ...}}.
@@ -27,6 +28,8 @@ KEYS = {
     "smsp__inst_executed.sum": "inst_executed",
     "smsp__issue_active.avg.pct_of_peak_sustained_active": "issue_active_pct",
     "smsp__thread_inst_executed_per_inst_executed.ratio": "threads_per_inst",
+    "lts__throughput.avg.pct_of_peak_sustained_elapsed": "lts_pct_of_peak",
+    "l1tex__throughput.avg.pct_of_peak_sustained_elapsed": "l1tex_pct_of_peak",
     "launch__grid_size": "grid",
     "launch__block_size": "block",
 }
@@ -35,7 +38,11 @@ SCALE = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "nsecond": 1, "use
 
 
 def summarise(rep: str, kernel: str):
-    out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    # a report, or the raw page already exported to CSV (profiles/r01_ncu_raw_*.csv)
+    if rep.endswith(".csv"):
+        out = open(rep).read()
+    else:
+        out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
     rows = list(csv.reader(io.StringIO(out)))
     head, units = rows[0], rows[1]
     res = None
@@ -65,7 +72,8 @@ if __name__ == "__main__":
         rep, kernel, work = arg.split(":")
         s = summarise(rep, kernel)
         if s:
-            s["report"] = os.path.basename(rep)
+            # a raw CSV keeps the name of the report it was exported from
+            s["report"] = data.get(work, {}).get("report") if rep.endswith(".csv") else os.path.basename(rep)
             data[work] = s
             print(work, json.dumps(s))
     with open(path, "w") as f:
