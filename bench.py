@@ -185,7 +185,8 @@ def make_context(D: Dist):
 
 
 class Timer:
-    """per-step CUDA-event timing with an L2 flush before each step"""
+    """per-step CUDA-event timing with an L2 flush before each step (outside the
+    events) and a host-ahead pre-roll before the first"""
 
     def __init__(self):
         import torch
@@ -208,6 +209,13 @@ class Timer:
         torch.cuda.synchronize()
         D.barrier()
         torch.cuda.synchronize()
+        # host-ahead pre-roll: a spin kernel (~0.2 ms per timed step, outside the
+        # events) keeps the GPU busy while the host enqueues the timed steps, so
+        # the events bracket device execution and not host submission gaps
+        # (latency-bound steps such as the 2^20 dot product are shorter than their
+        # host enqueue time).  Steps that synchronise with the host (e2e) are
+        # unaffected: their first event is recorded after the spin.
+        torch.cuda._sleep(int(min(K, 100) * 4e5))
         evs = []
         for _ in range(K):
             if flush:
