@@ -3,7 +3,7 @@
 task statement; DESIGN.md §"Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,sobel,gauss,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
+                    [--skeletons all|none|dot,sobel,gauss,redist,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
 block-distributed Matrix<float2> of pixel coordinates (MAX_ITER 1000, window
@@ -397,6 +397,139 @@ def roof_l2(workload: str):
             "committed capture (profiles/ncu_traffic.json)", "traffic": ncu_traffic(workload)}
 
 
+def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
+    """SURVEY 8(a) rows a9 (halo refresh) and a10 (redistribution) on ONE physical
+    GPU: a context of G = 4 logical devices (one process, separate memory per
+    device, all on the bench's stream), so every transfer is an on-GPU
+    device-to-device copy (HBM read + write) instead of an NVLink transfer.  The
+    roofline counts 2 x the bytes moved (read + write) plus the combine kernel's
+    traffic against the measured HBM copy bandwidth."""
+    import torch
+    from paper_conf_pact_steuwerg13_b200 import apps as A
+    from paper_conf_pact_steuwerg13_b200 import inputs as I
+    from paper_conf_pact_steuwerg13_b200 import skl as S
+    import oracle as O
+    G, N = 4, 150
+    nvox = N ** 3
+    c4 = S.Context(G, devices=[D.local] * G)
+    st = torch.cuda.current_stream()
+    for gg in range(G):
+        c4.set_stream(gg, st.cuda_stream)
+    out = {}
+    img = I.uniform_f32(I.SEED_DOT_A, nvox)
+
+    # a10: block -> copy (all-gather of the LM OSEM image).  Each step first
+    # rewrites the block parts (identity Map from w), which makes the replicas
+    # stale, so the gather moves data every step (copy -> block afterwards keeps
+    # each device's own slice and moves nothing, A26)
+    w = S.Vector.from_numpy(c4, img).set_distribution(S.BLOCK)
+    v = S.Vector(c4, S.F32, nvox).set_distribution(S.BLOCK)
+    ident = S.Map(c4, A.IDENT_F32, S.F32, S.F32)
+
+    def step_bc(marks):
+        ident(w, out=v)
+        if marks:
+            marks[0].record()
+        v.set_distribution(S.COPY)
+        if marks:
+            marks[1].record()
+        v.set_distribution(S.BLOCK)
+
+    p0 = c4.counter("p2p_bytes")
+    ms, seg = timer.run(step_bc, K, W, D, marks=2)
+    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    v.set_distribution(S.COPY)
+    ok = bool(np.array_equal(v.to_numpy(), img)) and moved >= (G - 1) * nvox * 4
+    out["redist_block_to_copy"] = {
+        "workload": f"block -> copy of a 150^3 fp32 Vector (13.5 MB), {G} logical devices on one GPU",
+        "ms": round(seg[1], 4), "bytes_moved": moved,
+        "roofline": roof_hbm(2 * moved, seg[1], P), "check": "ok" if ok else "FAIL"}
+
+    # a10: copy(+) -> block (LM OSEM's c): every device scatters into its own
+    # zeroed replica (a void Map with a WRITE extra argument, as the LM OSEM
+    # step does), then the combine exchanges slices and folds them in device order
+    addf = S.Reduce(c4, A.ADD, S.F32)
+    cv = S.Vector(c4, S.F32, nvox)
+    idx = S.Vector.from_numpy(c4, np.arange(nvox, dtype=np.int32)).set_distribution(S.BLOCK)
+    touch = S.Map(c4, "void touch(int i, float* c) { c[i] = 1.0f; }", S.I32, S.VOID, extra=[S.F32 | S.PTR])
+
+    def step_cb(marks):
+        cv.set_distribution(S.COPY, 0, addf)
+        cv.fill(0.0)
+        touch(idx, (cv, S.WRITE))
+        if marks:
+            marks[0].record()
+        cv.set_distribution(S.BLOCK)
+
+    p0 = c4.counter("p2p_bytes")
+    ms, seg = timer.run(step_cb, K, W, D, marks=1)
+    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    ok = bool(np.all(cv.to_numpy() == 1.0))
+    traffic = 2 * moved + (G + 1) * nvox * 4       # transfers + combine (G slices in, 1 out)
+    out["redist_copy_add_to_block"] = {
+        "workload": f"copy(+) -> block of a 150^3 fp32 Vector, {G} logical devices on one GPU "
+                    "(slices exchanged, then folded in device order)",
+        "ms": round(seg[1], 4), "bytes_moved": moved,
+        "roofline": roof_hbm(traffic, seg[1], P), "check": "ok" if ok else "FAIL"}
+    for x in (w, v, cv, idx):
+        x.destroy()
+
+    # a9: halo refresh of an overlap(2) 8192^2 fp32 image after a stencil, and the
+    # 10-iteration Gaussian with the refresh vs the fused halo push (DESIGN 6.5)
+    R = Cc = 8192
+    im = I.image_f32(I.SEED_GAUSS, R, Cc)
+    c4.set_option("block_threads", 128)
+    gau = S.MapOverlap(c4, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    c4.set_option("block_threads", 256)
+    a = S.Matrix.from_numpy(c4, im)
+    b = S.Matrix(c4, S.F32, R, Cc)
+    t = S.Matrix(c4, S.F32, R, Cc)
+    c4.set_option("halo_push", 0)
+
+    def step_halo(marks):
+        gau(a, out=b)
+        if marks:
+            marks[0].record()
+        b.set_distribution(S.OVERLAP, 2)
+
+    p0 = c4.counter("p2p_bytes")
+    ms, seg = timer.run(step_halo, K, W, D, marks=1)
+    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    out["halo_refresh"] = {
+        "workload": f"overlap(2) halo refresh of an 8192^2 fp32 Matrix after a stencil, {G} logical devices "
+                    f"on one GPU ({2 * (G - 1)} transfers of 2 rows)",
+        "ms": round(seg[1], 4), "bytes_moved": moved, "latency_bound": True}
+    ITER = 10
+    sub = im[3970:4094]
+    ref = sub
+    for _ in range(ITER):
+        ref = O.mapoverlap2d(O.OS_GAUSS5, ref, 2, O.OB_NEAREST, 0.0)
+    for push in (0, 1):
+        c4.set_option("halo_push", push)
+
+        def step_it(_):
+            gau(a, out=b)
+            for k in range(ITER - 1):
+                gau(b, out=t) if k % 2 == 0 else gau(t, out=b)
+
+        p0, h0 = c4.counter("p2p_bytes"), c4.counter("halo_push_bytes")
+        ms, _ = timer.run(step_it, max(3, K // 4), W, D)
+        reps = max(3, K // 4) + W
+        fin = t if (ITER - 1) % 2 == 1 else b
+        ok = bool(np.array_equal(fin.to_numpy()[4000:4064], ref[30:94]))
+        out[f"gauss_iter10_g{G}_{'push' if push else 'refresh'}"] = {
+            "workload": f"10 x Gaussian 5x5 on {G} logical devices of one GPU, halos "
+                        + ("pushed by the stencil kernel into the neighbours (fused)" if push
+                           else "refreshed by copies between iterations"),
+            "ms": round(ms, 4), "p2p_bytes_per_step": (c4.counter("p2p_bytes") - p0) / reps,
+            "halo_push_bytes_per_step": (c4.counter("halo_push_bytes") - h0) / reps,
+            "check": "ok" if ok else "FAIL"}
+    for x in (a, b, t):
+        x.destroy()
+    c4.finalize()
+    return out
+
+
 def bench_skeletons(args, D: Dist, P: dict, which):
     import torch
     from paper_conf_pact_steuwerg13_b200 import apps as A
@@ -488,6 +621,9 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         res["dot_sweep"] = {"workload": "fused sum(mult(A,B)) sweep 2^20..2^30 fp32 (no graph), cold L2, "
                                         "8 B/element", "points": sweep,
                             "check": "ok" if all(v["check"] == "ok" for v in sweep.values()) else "FAIL"}
+
+    if "redist" in which and D.world == 1:
+        res.update(bench_redist(ctx, timer, K, W, D, P))
 
     if "gauss_iter" in which:
         # K=10 iterated Gaussian (ping-pong); on several GPUs the halo
@@ -839,8 +975,8 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, D, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "scan_i32", "scan_f32", "lmosem", "lmosem_osem",
-         "allpairs"]
+        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "redist", "scan_i32", "scan_f32", "lmosem",
+         "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
     sk = bench_skeletons(args, D, P, which) if which else {}

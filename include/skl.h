@@ -125,6 +125,10 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * warp handles elements base + 32 j + l: for customising functions whose cost
  * varies per element, e.g. Mandelbrot; default 0), "ap_fast" (Allpairs
  * zip-reduce 128 x 128 tiles for 4-byte inputs with d % 4 == 0; default 1),
+ * "xfer_kernel" (1 = with several devices in this process, the moves of a
+ * redistribution or halo refresh into one GPU run as one batched copy kernel
+ * (peer loads over NVLink between GPUs); 0 = one cudaMemcpy(Peer)Async per
+ * move; default 1),
  * and the tuning keys "scan_variant", "scan_chunks", "scan_minb", "mo_rh",
  * "mo_cw", "mo_minb".  Environment defaults: SKL_BLOCK_THREADS,
  * SKL_DEBUG_BOUNDS; SKL_CACHE_DIR keeps compiled cubins on disk.              */

@@ -1,7 +1,9 @@
-// builtin.cu — the one kernel that needs no customising function: filling a
+// builtin.cu — the kernels that need no customising function: filling a
 // container's device parts with a value (skl_fill; used to zero the copy(+)
-// image replicas of LM OSEM before every subset, reading A25).  Compiled by
-// nvcc for sm_100a into libskl.so.
+// image replicas of LM OSEM before every subset, reading A25), and the batched
+// transfer kernel that executes all moves of a redistribution into one device
+// in a single launch (halo refresh P:L214-222).  Compiled by nvcc
+// for sm_100a into libskl.so.
 #include "skl_internal.h"
 
 namespace skl {
@@ -46,6 +48,121 @@ void launch_fill(Ctx* ctx, int g, void* dst, size_t bytes, const void* value, si
   }
   SKL_CUDA(cudaGetLastError());
   ctx->n_launch++;
+}
+
+// ---------------------------------------------------------------- batched transfers
+// One launch per destination GPU copies every segment of a redistribution plan
+// into it (one process, several devices: same-GPU copies, or loads from a peer
+// GPU's memory over NVLink when peer access is enabled).  Replaces one
+// cudaMemcpy(Peer)Async per segment: a block->copy of G parts is G-1 segments per
+// device, a halo refresh 2 small ones, and the per-copy launch latency
+// dominated both.  Each segment is copied in units of W bytes,
+// W = 16 when source and destination share their misalignment mod 16, else the
+// largest power of two both share (block parts of 4-byte elements: 8 or 4);
+// the unaligned head and tail (< 16 bytes) go bytewise.  The segments' bodies
+// are laid end to end in a byte space (each padded to 16 bytes) cut into
+// 32 KB chunks, one chunk per block iteration.
+constexpr unsigned long long SKL_XCHB = 32768;
+struct XferSegs {
+  const unsigned char* src[kXferMaxSegs];
+  unsigned char* dst[kXferMaxSegs];
+  unsigned long long len[kXferMaxSegs];        // body bytes (a multiple of the unit)
+  unsigned long long start[kXferMaxSegs + 1];  // byte-space offsets (16-byte multiples)
+  unsigned char unit[kXferMaxSegs];            // 16, 8, 4 or 1
+  // unaligned heads and tails (< 16 bytes each), copied bytewise
+  const unsigned char* bsrc[2 * kXferMaxSegs];
+  unsigned char* bdst[2 * kXferMaxSegs];
+  unsigned char blen[2 * kXferMaxSegs];
+  int nseg, nsmall;
+};
+
+template <class U>
+__device__ __forceinline__ void skl_xfer_range(const unsigned char* s0, unsigned char* d0, unsigned long long lo,
+                                               unsigned long long hi) {
+  const U* __restrict__ s = (const U*)s0;
+  U* __restrict__ d = (U*)d0;
+  unsigned long long i = lo / sizeof(U) + threadIdx.x;
+  const unsigned long long e = hi / sizeof(U);
+  // four loads in flight per thread, then four stores
+  for (; i + 3 * 256 < e; i += 4 * 256) {
+    const U a = __ldcs(s + i), b = __ldcs(s + i + 256), c = __ldcs(s + i + 512), f = __ldcs(s + i + 768);
+    __stcs(d + i, a);
+    __stcs(d + i + 256, b);
+    __stcs(d + i + 512, c);
+    __stcs(d + i + 768, f);
+  }
+  for (; i < e; i += 256) __stcs(d + i, __ldcs(s + i));
+}
+
+__global__ void __launch_bounds__(256) skl_xfer_batch(const XferSegs S) {
+  if (blockIdx.x == gridDim.x - 1)
+    for (int q = (int)threadIdx.x; q < S.nsmall * 16; q += 256) {
+      const int k = q >> 4, b = q & 15;
+      if (b < S.blen[k]) S.bdst[k][b] = S.bsrc[k][b];
+    }
+  const unsigned long long total = S.start[S.nseg];
+  for (unsigned long long c0 = (unsigned long long)blockIdx.x * SKL_XCHB; c0 < total;
+       c0 += (unsigned long long)gridDim.x * SKL_XCHB) {
+    const unsigned long long c1 = c0 + SKL_XCHB < total ? c0 + SKL_XCHB : total;
+    int k = 0;
+    while (S.start[k + 1] <= c0) ++k;  // first segment of the chunk (block-uniform)
+    for (; k < S.nseg && S.start[k] < c1; ++k) {
+      // chunk bounds relative to the segment (16-byte multiples), clipped to its body
+      unsigned long long lo = c0 > S.start[k] ? c0 - S.start[k] : 0;
+      unsigned long long hi = c1 - S.start[k];
+      if (hi > S.len[k]) hi = S.len[k];
+      if (lo >= hi) continue;
+      switch (S.unit[k]) {
+        case 16: skl_xfer_range<uint4>(S.src[k], S.dst[k], lo, hi); break;
+        case 8: skl_xfer_range<uint2>(S.src[k], S.dst[k], lo, hi); break;
+        case 4: skl_xfer_range<unsigned>(S.src[k], S.dst[k], lo, hi); break;
+        default: skl_xfer_range<unsigned char>(S.src[k], S.dst[k], lo, hi); break;
+      }
+    }
+  }
+}
+
+void launch_xfer_batch(Ctx* ctx, int g, const std::vector<XferSeg>& segs) {
+  Device& D = ctx->D(g);
+  ctx->set_device(g);
+  for (size_t b = 0; b < segs.size(); b += kXferMaxSegs) {
+    XferSegs S;
+    S.nseg = (int)std::min<size_t>(kXferMaxSegs, segs.size() - b);
+    S.nsmall = 0;
+    S.start[0] = 0;
+    auto small = [&](const unsigned char* src, unsigned char* dst, size_t n) {
+      if (n == 0) return;
+      S.bsrc[S.nsmall] = src;
+      S.bdst[S.nsmall] = dst;
+      S.blen[S.nsmall] = (unsigned char)n;
+      S.nsmall++;
+    };
+    for (int k = 0; k < S.nseg; ++k) {
+      const XferSeg& x = segs[b + (size_t)k];
+      const unsigned char* sp = (const unsigned char*)x.src;
+      unsigned char* dp = (unsigned char*)x.dst;
+      // unit: the largest power of two (<= 16) dividing src - dst
+      const uintptr_t diff = ((uintptr_t)sp - (uintptr_t)dp) & 15u;
+      const size_t W = diff == 0 ? 16 : (diff & (0u - diff));
+      const size_t head = std::min<size_t>(x.bytes, (W - (uintptr_t)dp % W) % W);
+      const size_t body = (x.bytes - head) / W * W;
+      small(sp, dp, head);
+      if (x.bytes - head - body >= 16) fail(SKL_ERR_CUDA, "internal: transfer tail");
+      small(sp + head + body, dp + head + body, x.bytes - head - body);
+      S.src[k] = sp + head;
+      S.dst[k] = dp + head;
+      S.len[k] = body;
+      S.unit[k] = (unsigned char)W;
+      S.start[k + 1] = S.start[k] + (body + 15) / 16 * 16;
+    }
+    const unsigned long long total = S.start[S.nseg];
+    if (total == 0 && S.nsmall == 0) continue;
+    const unsigned grid = (unsigned)std::max<unsigned long long>(
+        1, std::min<unsigned long long>((total + SKL_XCHB - 1) / SKL_XCHB, (unsigned long long)D.sm_count * 8));
+    skl_xfer_batch<<<grid, 256, 0, D.stream>>>(S);
+    SKL_CUDA(cudaGetLastError());
+    ctx->n_launch++;
+  }
 }
 
 }  // namespace skl

@@ -206,7 +206,23 @@ void nccl_destroy(Ctx* ctx) {
 void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes, PtrFn& p) {
   if (tr.empty()) return;
   if (!ctx->dist_mode) {
+    // one process: the moves into each device run as ONE batched copy kernel on
+    // that device's stream (same-GPU sources, or peer loads over NVLink);
+    // sources without peer access use the copy engines
     barrier_streams(ctx);
+    // one launch per PHYSICAL destination GPU (logical devices sharing a GPU
+    // are served by one kernel on the first one's stream; the barriers around
+    // order it with every device stream)
+    std::vector<int> launcher((size_t)ctx->G);
+    for (int g = 0; g < ctx->G; ++g) {
+      launcher[(size_t)g] = g;
+      for (int h = 0; h < g; ++h)
+        if (ctx->D(h).phys == ctx->D(g).phys) {
+          launcher[(size_t)g] = h;
+          break;
+        }
+    }
+    std::vector<std::vector<XferSeg>> batch((size_t)ctx->G);
     for (const Transfer& t : tr) {
       const size_t bytes = t.n * unit_bytes;
       if (bytes == 0) continue;
@@ -214,13 +230,20 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
       Device& D = ctx->D(t.dst);
       void* s = p.src(t);
       void* d = p.dst(t);
+      ctx->p2p += (long long)bytes;
+      const int lg = launcher[(size_t)t.dst];
+      if (ctx->xfer_kernel && ctx->peer_ok[(size_t)lg][(size_t)t.src]) {
+        batch[(size_t)lg].push_back(XferSeg{s, d, bytes});
+        continue;
+      }
       SKL_CUDA(cudaSetDevice(D.phys));
       if (S.phys == D.phys)
         SKL_CUDA(cudaMemcpyAsync(d, s, bytes, cudaMemcpyDeviceToDevice, D.stream));
       else
         SKL_CUDA(cudaMemcpyPeerAsync(d, D.phys, s, S.phys, bytes, D.stream));
-      ctx->p2p += (long long)bytes;
     }
+    for (int g = 0; g < ctx->G; ++g)
+      if (!batch[(size_t)g].empty()) launch_xfer_batch(ctx, g, batch[(size_t)g]);
     barrier_streams(ctx);
     return;
   }

@@ -83,6 +83,8 @@ void cont_destroy(Cont* c) {
   materialize_dependents(c);
   drop_lazy(c);
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) free_part(c, g);
+  for (size_t g = 0; g < c->stage.size(); ++g)
+    if (c->stage[g]) device_free(ctx, (int)g, c->stage[g]);
   if (c->host) cudaFreeHost(c->host);
   ctx->conts.erase(c);
   delete c;
@@ -409,9 +411,23 @@ static void combine_to_block(Cont* c) {
     if (r.empty()) continue;
     for (int h = 0; h < G; ++h) tr.push_back(Transfer{h, g, r.lo, r.lo, r.size(), h});
   }
+  // staging slots of device g: G replica slices, each padded to a multiple of
+  // 16 elements (so every slot starts 16-byte aligned for the vector combine)
+  auto slot_elems = [&](const Range& r) { return (r.size() * c->cols + 15) / 16 * 16; };
+  // staging is kept with the container between combines (LM OSEM combines
+  // every subset): no allocation on the steady-state path
+  c->stage.resize((size_t)G, nullptr);
+  c->stage_bytes.resize((size_t)G, 0);
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
     const Range r = block_range(U, G, g);
-    if (!r.empty()) staging[(size_t)g] = device_alloc(ctx, g, (size_t)G * r.size() * ub);
+    if (r.empty()) continue;
+    const size_t need = (size_t)G * slot_elems(r) * c->elt;
+    if (c->stage_bytes[(size_t)g] < need) {
+      device_free(ctx, g, c->stage[(size_t)g]);
+      c->stage[(size_t)g] = device_alloc(ctx, g, need);
+      c->stage_bytes[(size_t)g] = need;
+    }
+    staging[(size_t)g] = c->stage[(size_t)g];
   }
   struct StagePtrs : PtrFn {
     Cont* c;
@@ -421,7 +437,8 @@ static void combine_to_block(Cont* c) {
     void* src(const Transfer& t) override { return part_ptr(c, t.src, t.src_unit); }
     void* dst(const Transfer& t) override {
       const Range r = block_range(U, G, t.dst);
-      return (char*)(*st)[(size_t)t.dst] + ((size_t)t.slot * r.size() + (t.dst_unit - r.lo)) * c->unit_bytes();
+      const size_t slot = (r.size() * c->cols + 15) / 16 * 16 * c->elt;
+      return (char*)(*st)[(size_t)t.dst] + (size_t)t.slot * slot + (t.dst_unit - r.lo) * c->unit_bytes();
     }
   } sp;
   sp.c = c;
@@ -429,19 +446,24 @@ static void combine_to_block(Cont* c) {
   sp.U = U;
   sp.G = G;
   run_transfers(ctx, tr, ub, sp);
-  // replace the replicas by the folded blocks
+  // the folded block of device g goes into its replica's buffer (it covers
+  // the block range; every read of that slice went to staging, and the
+  // transfers finished at run_transfers' closing barrier)
   for (int g = ctx->first_local; g < ctx->first_local + ctx->nlocal; ++g) {
     const Range r = block_range(U, G, g);
-    free_part(c, g);
-    if (r.empty()) continue;
-    Part& p = c->parts[(size_t)g];
     const Range ar = alloc_range(c, blk, g);
-    p.ptr = device_alloc(ctx, g, ar.size() * ub);
-    p.buf = ar;
-    p.cap_bytes = ar.size() * ub;
-    run_combine(c->combine, g, staging[(size_t)g], r.size() * c->cols, G, part_ptr(c, g, r.lo),
-                r.size() * c->cols);
-    device_free(ctx, g, staging[(size_t)g]);
+    Part& p = c->parts[(size_t)g];
+    if (r.empty()) {
+      free_part(c, g);
+      continue;
+    }
+    if (!p.ptr || !p.buf.contains(ar)) {
+      free_part(c, g);
+      p.ptr = device_alloc(ctx, g, ar.size() * ub);
+      p.buf = ar;
+      p.cap_bytes = ar.size() * ub;
+    }
+    run_combine(c->combine, g, staging[(size_t)g], slot_elems(r), G, part_ptr(c, g, r.lo), r.size() * c->cols);
   }
   c->dist = blk;
   c->diverged = false;

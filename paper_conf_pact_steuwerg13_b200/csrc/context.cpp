@@ -250,6 +250,11 @@ void event_put(Ctx* ctx, int g, cudaEvent_t e) {
 // consumers (G <= 8, so at most 64 event waits).
 void barrier_streams(Ctx* ctx) {
   if (ctx->nlocal <= 1) return;
+  // devices that share a stream (e.g. logical devices handed one caller
+  // stream) are already ordered with each other
+  bool one_stream = true;
+  for (auto& d : ctx->dev) one_stream = one_stream && d.stream == ctx->dev[0].stream;
+  if (one_stream) return;
   for (auto& d : ctx->dev) {
     SKL_CUDA(cudaSetDevice(d.phys));
     SKL_CUDA(cudaEventRecord(d.ev, d.stream));
@@ -257,7 +262,7 @@ void barrier_streams(Ctx* ctx) {
   for (auto& a : ctx->dev) {
     SKL_CUDA(cudaSetDevice(a.phys));
     for (auto& b : ctx->dev)
-      if (&a != &b) SKL_CUDA(cudaStreamWaitEvent(a.stream, b.ev, 0));
+      if (&a != &b && a.stream != b.stream) SKL_CUDA(cudaStreamWaitEvent(a.stream, b.ev, 0));
   }
 }
 

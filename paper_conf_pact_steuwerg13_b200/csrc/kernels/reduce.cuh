@@ -221,14 +221,60 @@ skl_reduce_zip_sc(const SKL_ZL* __restrict__ l, const SKL_ZR* __restrict__ r, sk
 // Ordered fold of `nrep` staged values per element (copy(+) -> block combine,
 // reading A25; and the cross-GPU fold of Reduce partials): out[i] =
 // s[0][i] (+) s[1][i] (+) ... (+) s[nrep-1][i], GPU order.
+// All replicas' loads of an element (up to SKL_CMAXR) are issued before the
+// fold, so a thread has nrep loads in flight instead of one round trip per
+// replica; with `vec` (stride a multiple of SKL_RVEC, 16-byte aligned buffers)
+// every load and store is 16 bytes wide.
+#define SKL_CMAXR 8
+template <int V>
+__device__ __forceinline__ void skl_combine_run(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep,
+                                                SKL_T* __restrict__ out, skl_u64 n_chunks) {
+  SklOp op;
+  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i < n_chunks;
+       i += (skl_u64)gridDim.x * SKL_BLOCK) {
+    SklChunk<SKL_T, V> x[SKL_CMAXR];
+#pragma unroll
+    for (int r = 0; r < SKL_CMAXR; ++r)
+      if (r < nrep) {
+        if (V > 1) {
+          x[r].q[0] = skl_ld16(staging + (skl_u64)r * stride + i * V);
+        } else {
+          x[r].e[0] = staging[(skl_u64)r * stride + i];
+        }
+      }
+    SklChunk<SKL_T, V> a = x[0];
+#pragma unroll
+    for (int r = 1; r < SKL_CMAXR; ++r)
+      if (r < nrep) {
+#pragma unroll
+        for (int k = 0; k < V; ++k) a.e[k] = op(a.e[k], x[r].e[k]);
+      }
+    for (int r = SKL_CMAXR; r < nrep; ++r)  // more than SKL_CMAXR devices
+#pragma unroll
+      for (int k = 0; k < V; ++k) a.e[k] = op(a.e[k], staging[(skl_u64)r * stride + i * V + k]);
+    if (V > 1) skl_st16(out + i * V, a.q[0]);
+    else out[i] = a.e[0];
+  }
+}
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_combine(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep, SKL_T* __restrict__ out,
-            skl_u64 n) {
-  SklOp op;
-  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i < n;
-       i += (skl_u64)gridDim.x * SKL_BLOCK) {
-    SKL_T a = staging[i];
-    for (int r = 1; r < nrep; ++r) a = op(a, staging[(skl_u64)r * stride + i]);
-    out[i] = a;
+            skl_u64 n, int vec) {
+#if SKL_RVEC > 1
+  if (vec) {
+    const skl_u64 nc = n / SKL_RVEC;
+    skl_combine_run<SKL_RVEC>(staging, stride, nrep, out, nc);
+    // scalar tail (< SKL_RVEC elements), block 0
+    const skl_u64 t0 = nc * SKL_RVEC;
+    if (blockIdx.x == 0 && threadIdx.x < n - t0) {
+      SklOp op;
+      const skl_u64 i = t0 + threadIdx.x;
+      SKL_T a = staging[i];
+      for (int r = 1; r < nrep; ++r) a = op(a, staging[(skl_u64)r * stride + i]);
+      out[i] = a;
+    }
+    return;
   }
+#endif
+  (void)vec;
+  skl_combine_run<1>(staging, stride, nrep, out, n);
 }

@@ -570,9 +570,14 @@ void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int n
   if (!s || (s->kind != K_REDUCE && s->kind != K_SCAN)) fail(SKL_ERR_INVALID_ARG, "combine needs a Reduce skeleton");
   Ctx* ctx = s->ctx;
   unsigned long long stride = stride_elems, n = nelem;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(nelem, (size_t)s->block),
+  // 16-byte path: the element size divides 16, the replica stride is a whole
+  // number of 16-byte words and both buffers are 16-byte aligned
+  const size_t st = ctx->type(s->tin).size;
+  int vec = 16 % st == 0 && st < 16 && (stride_elems * st) % 16 == 0 && aligned16(staging) && aligned16(dst);
+  const size_t per = vec ? 16 / st : 1;
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)s->block),
                                                            (size_t)ctx->D(g).sm_count * 8));
-  void* args[] = {(void*)&staging, &stride, &nrep, &dst, &n};
+  void* args[] = {(void*)&staging, &stride, &nrep, &dst, &n, &vec};
   launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(s->block), 0, args);
 }
 

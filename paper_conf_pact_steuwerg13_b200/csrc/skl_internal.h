@@ -140,6 +140,7 @@ struct Ctx {
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
+  int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
   int ap_fast = 1;             // Allpairs zip-reduce: 128-row tiles (4-byte inputs, d % 4 == 0)
   int ap_tile = 0;             // Allpairs tile columns: 0 = by wave fill, 8 = 128, 4 = 64           // MapOverlap stores its border rows into the neighbours' halos
@@ -209,6 +210,8 @@ struct Cont {
   bool halo_valid = false;   // overlap halos valid too
   bool diverged = false;     // copy replicas written independently
   Skel* combine = nullptr;   // copy(+) combine function (A25)
+  std::vector<void*> stage;  // combine staging per device (kept for the next combine)
+  std::vector<size_t> stage_bytes;
   std::vector<Part> parts;   // indexed by global device; only local ones used
   void* host = nullptr;      // pinned host mirror (lazily allocated)
   bool host_valid = false;
@@ -253,6 +256,15 @@ struct PtrFn {
   virtual ~PtrFn() = default;
 };
 void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes, PtrFn& p);
+// one batched copy launch on device g's stream (builtin.cu); sources are on
+// g's GPU or a peer with access enabled
+constexpr int kXferMaxSegs = 32;
+struct XferSeg {
+  const void* src;
+  void* dst;
+  size_t bytes;
+};
+void launch_xfer_batch(Ctx* ctx, int g, const std::vector<XferSeg>& segs);
 void barrier_streams(Ctx* ctx);  // every local stream waits for every other
 cudaEvent_t event_get(Ctx* ctx, int g);
 void event_put(Ctx* ctx, int g, cudaEvent_t e);
