@@ -129,15 +129,20 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * redistribution or halo refresh into one GPU run as one batched copy kernel
  * (peer loads over NVLink between GPUs); 0 = one cudaMemcpy(Peer)Async per
  * move; default 1),
+ * "mo_ws" (1 = 2-D MapOverlap tiles are staged by a TMA producer warp into a
+ * ring of "mo_ws_stages" shared-memory buffers consumed by the other warps of
+ * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged
+ * row <= 256 units; otherwise the one-tile-per-block kernel runs),
  * and the tuning keys "scan_variant", "scan_chunks", "scan_minb", "mo_rh",
- * "mo_cw", "mo_minb".  Environment defaults: SKL_BLOCK_THREADS,
+ * "mo_cw", "mo_minb", "mo_ws_minb".  Environment defaults: SKL_BLOCK_THREADS,
  * SKL_DEBUG_BOUNDS; SKL_CACHE_DIR keeps compiled cubins on disk.              */
 skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
 /* Counters: "launches" (kernels this library launched), "compiles" (NVRTC runs),
  * "cache_hits", "h2d_bytes", "d2h_bytes", "p2p_bytes" (device-to-device copy
  * bytes), "halo_push_bytes" (halo bytes stored by MapOverlap kernels directly
  * into neighbour devices' memory), "disk_cache_hits" (cubins loaded from
- * SKL_CACHE_DIR instead of compiled).                                          */
+ * SKL_CACHE_DIR instead of compiled), "tma_launches" (MapOverlap launches of
+ * the TMA / warp-specialised kernel).                                          */
 skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value);
 const char* skl_last_error(void);
 

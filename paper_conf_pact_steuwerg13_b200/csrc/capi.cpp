@@ -199,6 +199,14 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->scan_minb = (int)value;
     } else if (k == "mo_persist") {
       c->mo_persist = value ? 1 : 0;
+    } else if (k == "mo_ws") {
+      c->mo_ws = value ? 1 : 0;
+    } else if (k == "mo_ws_stages") {
+      if (value < 2 || value > 8) fail(SKL_ERR_INVALID_ARG, "mo_ws_stages in [2,8]");
+      c->mo_ws_stages = (int)value;
+    } else if (k == "mo_ws_minb") {
+      if (value < 0 || value > 32) fail(SKL_ERR_INVALID_ARG, "mo_ws_minb in [0,32]");
+      c->mo_ws_minb = (int)value;
     } else if (k == "mo_minb") {
       if (value < 0 || value > 32) fail(SKL_ERR_INVALID_ARG, "mo_minb in [0,32]");
       c->mo_minb = (int)value;
@@ -246,6 +254,7 @@ skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value) {
     else if (k == "p2p_bytes") *value = c->p2p;
     else if (k == "halo_push_bytes") *value = c->pushed;
     else if (k == "disk_cache_hits") *value = c->n_disk_hit;
+    else if (k == "tma_launches") *value = c->n_tma;
     else fail(SKL_ERR_INVALID_ARG, "unknown counter " + k);
   });
 }

@@ -228,6 +228,127 @@ skl_mo2d_p(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT*
   }
   (void)in_rows;
 }
+
+// ------------------------------------------------------------------ 2-D, TMA + warp specialisation
+// Persistent resident blocks of SKL_BLOCK consumer threads plus one producer
+// warp.  The producer's elected lane stages tile after tile with one TMA box
+// copy each (cp.async.bulk.tensor.2d: the whole (TH + 2d) x PITCH window in one
+// instruction, out-of-matrix cells zero-filled by the copy engine) into a ring
+// of nstages shared-memory buffers, signalling a "full" mbarrier by transaction
+// bytes; the consumers wait on it, apply f exactly as skl_mo2d does
+// (skl_mo_apply) and release the buffer through an "empty" mbarrier (one arrival
+// per consumer warp).  Consumer threads issue no staging instructions and the
+// next tiles' loads are always in flight while f runs.  Border tiles whose
+// boundary mode is not "zero" (NEAREST, or NEUTRAL with a non-zero value) are
+// patched in shared memory by the consumers before f runs.
+struct alignas(64) SklTmap {
+  unsigned long long opaque[16];
+};
+#define SKL_WS_MAXS 8
+#ifndef SKL_WS_MINB
+#define SKL_WS_MINB 1
+#endif
+__device__ __forceinline__ void skl_mbar_wait(unsigned a, unsigned parity) {
+  unsigned done;
+  do {
+    asm volatile(
+        "{ .reg .pred p; mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2; selp.u32 %0, 1, 0, p; }"
+        : "=r"(done) : "r"(a), "r"(parity) : "memory");
+  } while (!done);
+}
+__device__ __forceinline__ void skl_bar_consumers() {
+  asm volatile("bar.sync 1, %0;" ::"n"(SKL_BLOCK) : "memory");
+}
+
+// Out-of-matrix cells of a TMA-staged tile (zero-filled) get the boundary mode's
+// value: NEAREST copies the nearest in-matrix row, then column (each coordinate
+// clamped independently, A20); NEUTRAL writes the neutral value.
+__device__ __forceinline__ void skl_mo_fix(SKL_TIN* tile, const SklMoGeo& G, int r0, int c0, SKL_TIN neutral) {
+  const int gr0 = r0 - SKL_D, gc0 = c0 - SKL_A;
+  const int top = gr0 < 0 ? -gr0 : 0, bot = G.Ri - gr0;  // rows [top, bot) are inside
+  const int left = gc0 < 0 ? -gc0 : 0, right = G.Ci - gc0;
+#if SKL_BOUNDARY == 1
+  if (top > 0 || bot < SKL_SROWS) {
+    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
+      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+      if (i < top) tile[q] = tile[top * SKL_PITCH + j];
+      else if (i >= bot) tile[q] = tile[(bot - 1) * SKL_PITCH + j];
+    }
+    skl_bar_consumers();
+  }
+  if (left > 0 || right < SKL_PITCH) {
+    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
+      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+      if (j < left) tile[q] = tile[i * SKL_PITCH + left];
+      else if (j >= right) tile[q] = tile[i * SKL_PITCH + right - 1];
+    }
+  }
+#else
+  for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
+    const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+    if (i < top || i >= bot || j < left || j >= right) tile[q] = neutral;
+  }
+#endif
+  skl_bar_consumers();
+}
+
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK + 32, SKL_WS_MINB)
+skl_mo2d_ws(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, long in_row0, long out_row0,
+            long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok, SKL_TOUT* __restrict__ push_up,
+            SKL_TOUT* __restrict__ push_down, long hd, int tiles_x, int ntiles, int nstages, int fix, int xscale) {
+  extern __shared__ __align__(128) unsigned char skl_mo_dyn[];
+  __shared__ __align__(8) unsigned long long bars[2 * SKL_WS_MAXS];
+  constexpr unsigned TB = SKL_SROWS * SKL_PITCH * (unsigned)sizeof(SKL_TIN);
+  constexpr unsigned TS = (TB + 127u) / 128u * 128u;  // TMA destinations are 128-byte aligned
+  const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
+  const unsigned raw = (unsigned)__cvta_generic_to_shared(skl_mo_dyn);
+  const unsigned base = (raw + 127u) & ~127u;
+  const unsigned full0 = (unsigned)__cvta_generic_to_shared(bars), empty0 = full0 + 8u * SKL_WS_MAXS;
+  if (threadIdx.x == 0) {
+    for (int s = 0; s < nstages; ++s) {
+      asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(full0 + 8u * s) : "memory");
+      asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(empty0 + 8u * s), "n"(SKL_BLOCK / 32)
+                   : "memory");
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  if (warp == SKL_BLOCK / 32) {  // producer
+    if (lane == 0) {
+      int k = 0;
+      for (int t = blockIdx.x; t < ntiles; t += gridDim.x, ++k) {
+        const int s = k % nstages;
+        if (k >= nstages) skl_mbar_wait(empty0 + 8u * s, ((k / nstages) & 1) ^ 1);
+        asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(full0 + 8u * s), "n"(TB)
+                     : "memory");
+        const int r0 = G.rb + (t / tiles_x) * SKL_TH, c0 = (t % tiles_x) * SKL_TW;
+        asm volatile(
+            "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], "
+            "[%4];" ::"r"(base + TS * s),
+            "l"((unsigned long long)&tmap), "r"((c0 - SKL_A) * xscale), "r"(r0 - SKL_D - G.irow0),
+            "r"(full0 + 8u * s)
+            : "memory");
+      }
+    }
+    return;
+  }
+  int k = 0;
+  for (int t = blockIdx.x; t < ntiles; t += gridDim.x, ++k) {
+    const int s = k % nstages;
+    skl_mbar_wait(full0 + 8u * s, (k / nstages) & 1);
+    SKL_TIN* tile = (SKL_TIN*)(skl_mo_dyn + (base - raw) + TS * s);
+    const int r0 = G.rb + (t / tiles_x) * SKL_TH, c0 = (t % tiles_x) * SKL_TW;
+    const bool border = fix && (r0 - SKL_D < 0 || r0 + SKL_TH + SKL_D > G.Ri || c0 - SKL_A < 0 ||
+                                c0 + SKL_TW + SKL_A > G.Ci);
+    if (border) skl_mo_fix(tile, G, r0, c0, neutral);
+    skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
+    // generic-proxy writes of the patch must be ordered before the next TMA write
+    if (border) asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    __syncwarp();
+    if (lane == 0) asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(empty0 + 8u * s) : "memory");
+  }
+}
 #else
 // ------------------------------------------------------------------ 1-D (vector)
 #define SKL_SLEN (SKL_TW + 2 * SKL_A)

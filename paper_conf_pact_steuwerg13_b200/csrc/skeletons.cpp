@@ -16,7 +16,17 @@
 #include <cstdio>
 #include <numeric>
 
+#include <cuda.h>
+#include <cudaTypedefs.h>
+
 #include "skl_internal.h"
+
+namespace skl {
+struct alignas(64) SklTensorMap {
+  unsigned char b[128];
+};
+static_assert(sizeof(SklTensorMap) == sizeof(CUtensorMap), "tensor map size");
+}  // namespace skl
 
 namespace skl {
 
@@ -201,6 +211,11 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       // occupancy and cost 30 % - and 128 for wider elements)
       const int minb = ctx->mo_minb > 0 ? ctx->mo_minb : std::max(1, 65536 / (nthr * (si >= 4 ? 128 : 64)));
       defs += "#define SKL_MO_MINB " + std::to_string(minb) + "\n";
+      // the TMA / warp-specialised kernel (one extra producer warp) keeps the same
+      // per-thread register budget
+      const int wsminb =
+          ctx->mo_ws_minb > 0 ? ctx->mo_ws_minb : std::max(1, 65536 / ((nthr + 32) * (si >= 4 ? 128 : 64)));
+      defs += "#define SKL_WS_MINB " + std::to_string(wsminb) + "\n";
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;
@@ -847,6 +862,46 @@ static bool plan_halo_push(Ctx* ctx, Cont* o, size_t d, std::vector<void*>& up, 
   return true;
 }
 
+// TMA descriptor of a device's input part for skl_mo2d_ws: a 2-D tiled map over
+// rows x columns (row pitch C * elt bytes, a multiple of 16), box = the staged
+// window (pitch x srows elements).  Elements are described as 8/4/2/1-byte
+// units (the largest dividing elt; xscale units per element).  Returns false
+// when TMA cannot describe it (box wider than 256 units, no driver entry
+// point): the caller uses skl_mo2d.
+static bool encode_tile_map(SklTensorMap* tm, const void* base, size_t elt, size_t C, size_t rows, size_t pitch,
+                            size_t srows, int* xscale) {
+  static PFN_cuTensorMapEncodeTiled_v12000 enc = nullptr;
+  static bool tried = false;
+  if (!tried) {
+    tried = true;
+    cudaDriverEntryPointQueryResult q;
+    void* fn = nullptr;
+    if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      enc = (PFN_cuTensorMapEncodeTiled_v12000)fn;
+    else
+      (void)cudaGetLastError();
+  }
+  if (!enc) return false;
+  const size_t unit = elt % 8 == 0 ? 8 : elt % 4 == 0 ? 4 : elt % 2 == 0 ? 2 : 1;
+  const size_t sc = elt / unit;
+  if (pitch * sc > 256 || srows > 256 || rows == 0 || rows >= (1ull << 31) || C * sc >= (1ull << 31)) return false;
+  const CUtensorMapDataType dt = unit == 8 ? CU_TENSOR_MAP_DATA_TYPE_UINT64
+                                 : unit == 4 ? CU_TENSOR_MAP_DATA_TYPE_UINT32
+                                 : unit == 2 ? CU_TENSOR_MAP_DATA_TYPE_UINT16
+                                             : CU_TENSOR_MAP_DATA_TYPE_UINT8;
+  const cuuint64_t dims[2] = {(cuuint64_t)(C * sc), (cuuint64_t)rows};
+  const cuuint64_t strides[1] = {(cuuint64_t)(C * elt)};
+  const cuuint32_t box[2] = {(cuuint32_t)(pitch * sc), (cuuint32_t)srows};
+  const cuuint32_t estr[2] = {1, 1};
+  const CUresult r = enc((CUtensorMap*)tm, dt, 2, const_cast<void*>(base), dims, strides, box, estr,
+                         CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE,
+                         CU_TENSOR_MAP_L2_PROMOTION_L2_128B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  if (r != CUDA_SUCCESS) return false;
+  *xscale = (int)sc;
+  return true;
+}
+
 void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   if (s->kind != K_MAPOVERLAP) fail(SKL_ERR_INVALID_ARG, "not a MapOverlap skeleton");
   Ctx* ctx = s->ctx;
@@ -895,7 +950,27 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                       s->neutral.data(), &vec_ok, &pu, &pd, &hd};
       const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
                       (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
-      if (ctx->mo_persist) {
+      SklTensorMap tm;
+      int xscale = 1;
+      if (ctx->mo_ws && vec_ok &&
+          encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
+                          (size_t)(s->mo_th + 2 * s->d), &xscale)) {
+        // TMA producer warp + consumer warps over a ring of staged tiles
+        const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;
+        const int nst = ctx->mo_ws_stages;
+        const size_t smem = (size_t)nst * ((tile_bytes + 127) / 128 * 128) + 128;
+        int tiles_x = (int)grid.x, ntiles = (int)(grid.x * grid.y);
+        const int nthr = s->block + 32;
+        const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_mo2d_ws", nthr, smem));
+        const size_t pgrid = std::min((size_t)ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
+        // fix: border tiles need patching unless the boundary value is zero
+        int fix = s->boundary == 1 ? 1 : 0;
+        for (unsigned char b : s->neutral) fix |= b != 0;
+        void* wargs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
+                         &pu, &pd, &hd, &tiles_x, &ntiles, (void*)&nst, &fix, &xscale};
+        launch(ctx, g, s->prog, "skl_mo2d_ws", dim3((unsigned)pgrid), dim3((unsigned)nthr), smem, wargs);
+        ctx->n_tma++;
+      } else if (ctx->mo_persist) {
         // resident blocks walk the tiles with two staging buffers (load of tile
         // k+1 overlaps f on tile k)
         const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;

@@ -137,6 +137,9 @@ struct Ctx {
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
   int mo_persist = 0;          // MapOverlap 2-D: persistent blocks, double-buffered tiles
+  int mo_ws = 0;               // MapOverlap 2-D: TMA producer warp + consumer warps (skl_mo2d_ws)
+  int mo_ws_stages = 4;        //   shared-memory ring depth
+  int mo_ws_minb = 0;          //   resident blocks per SM the registers must allow (0 = auto)
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
@@ -153,7 +156,7 @@ struct Ctx {
   // only: 3 / 4 / 6 without look-back (wrong results, the pipeline's ceiling)
   int scan_variant = 6;
   // counters
-  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0}, n_disk_hit{0};
+  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0}, n_disk_hit{0}, n_tma{0};
   int composed_id = 0;  // names of composed Map chains (lazy fusion)
   // optional caller-provided device allocator (skl_set_allocator)
   void* (*user_alloc)(size_t, int, void*, void*) = nullptr;

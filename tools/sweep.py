@@ -2,7 +2,7 @@
 variants).  Prints one line per configuration: device ms per call (CUDA events,
 L2 flushed), plus a parity flag against the oracle where cheap.
 
-  python tools/sweep.py mandel|lmosem|scan|mo
+  python tools/sweep.py mandel|lmosem|scan|mo|mows
 """
 import os
 import sys
@@ -243,6 +243,54 @@ def mo():
                 ok = f" bitexact={np.array_equal(o.to_numpy()[4000:4064], ref)}"
             print(f"mo {name:9s} block={bt} rh={rh} cw={cw8 if t == S.U8 else cw32} minb={cfg[4] if len(cfg) > 4 else 0} persist={cfg[5] if len(cfg) > 5 else 0}: {ms:.4f} ms  "
                   f"{bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s{ok}", flush=True)
+            x.destroy()
+            o.destroy()
+        c.finalize()
+
+
+def mows():
+    """TMA / warp-specialised MapOverlap (mo_ws) against the one-tile-per-block
+    kernel.  MOWS_CFGS="block,rh,cw,ws,stages,wsminb;..." (0 = automatic).  The
+    full output image is compared with the plain kernel's (bit-exact)."""
+    img8 = I.image_u8(5, 8192, 8192)
+    imgf = I.image_f32(6, 8192, 8192)
+    cfgs = [tuple(int(x) for x in t.split(",")) for t in
+            os.environ.get("MOWS_CFGS", "256,0,0,0,4,0").split(";")]
+    work = [w for w in (("ident_u8", A.IDENT2D_U8, S.U8, 1, S.NEUTRAL, img8),
+                        ("sobel", A.SOBEL, S.U8, 1, S.NEUTRAL, img8),
+                        ("ident_f32", A.IDENT2D, S.F32, 2, S.NEAREST, imgf),
+                        ("gauss", A.gaussian5(), S.F32, 2, S.NEAREST, imgf))
+            if w[0] in os.environ.get("MOWS_WORK", "ident_u8,sobel,ident_f32,gauss").split(",")]
+    refs = {}
+    c0 = ctx_with({"block_threads": 256 if True else 0})
+    for name, src, t, d, bnd, img in work:
+        if name == "gauss":
+            c0.set_option("block_threads", 128)
+        m = S.MapOverlap(c0, src, t, t, d, bnd, 0)
+        c0.set_option("block_threads", 256)
+        x = S.Matrix.from_numpy(c0, img)
+        o = m(x)
+        ms = timeit(lambda: m(x, out=o))
+        refs[name] = o.to_numpy()
+        print(f"mows {name:9s} plain (bench config): {ms:.4f} ms", flush=True)
+        x.destroy()
+        o.destroy()
+    c0.finalize()
+    for cfg in cfgs:
+        bt, rh, cw, ws, st, wm = cfg
+        c = ctx_with({"block_threads": bt, "mo_ws": ws, "mo_ws_stages": st, "mo_ws_minb": wm,
+                      "mo_rh": rh, "mo_cw": cw})
+        for name, src, t, d, bnd, img in work:
+            m = S.MapOverlap(c, src, t, t, d, bnd, 0)
+            x = S.Matrix.from_numpy(c, img)
+            o = m(x)
+            n0 = c.counter("tma_launches")
+            ms = timeit(lambda: m(x, out=o))
+            tma = c.counter("tma_launches") > n0
+            ok = np.array_equal(o.to_numpy(), refs[name])
+            bpp = 2 * img.itemsize
+            print(f"mows {name:9s} block={bt} rh={rh} cw={cw} ws={ws} stages={st} wsminb={wm} tma={tma}: "
+                  f"{ms:.4f} ms  {bpp * img.size / (ms / 1e3) / 1e9:.0f} GB/s same={ok}", flush=True)
             x.destroy()
             o.destroy()
         c.finalize()
