@@ -125,6 +125,9 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * warp handles elements base + 32 j + l: for customising functions whose cost
  * varies per element, e.g. Mandelbrot; default 0), "ap_fast" (Allpairs
  * zip-reduce 128 x 128 tiles for 4-byte inputs with d % 4 == 0; default 1),
+ * "ap_hybrid" (1 = when the 128 x 128 tiles leave the last wave less than half
+ * full, that wave runs as 128 x 64 halves; default 1), "ap_tile" (0 = automatic,
+ * 8 / 4 = force 128 / 64 tile columns, 2 = force the hybrid),
  * "xfer_kernel" (1 = with several devices in this process, the moves of a
  * redistribution or halo refresh into one GPU run as one batched copy kernel
  * (peer loads over NVLink between GPUs); 0 = one cudaMemcpy(Peer)Async per

@@ -96,7 +96,16 @@ void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out) {
         bool narrow = eff(t4, 3 * sms) * 0.82 > eff(t8, 2 * sms);
         if (ctx->ap_tile == 8) narrow = false;
         if (ctx->ap_tile == 4) narrow = true;
-        if (narrow)
+        // hybrid: whole waves of 128 x 128 tiles, the partial last wave as
+        // 128 x 64 halves (when they fit one wave of 2 blocks per SM)
+        const size_t slots = 2 * sms, rem = t8 % slots;
+        const bool hybrid = (ctx->ap_tile == 0 || ctx->ap_tile == 2) && ctx->ap_hybrid && t8 > slots &&
+                            rem != 0 && 2 * rem <= slots;
+        if (hybrid || ctx->ap_tile == 2) {
+          long nwide = (long)(t8 - rem), tiles_x = (long)cdiv(m, 128);
+          void* hargs[] = {(void*)&pa, (void*)&pb, &pc, &nn, &mm, &dd, &nwide, &tiles_x};
+          launch(ctx, g, s->prog, "skl_ap_zrh", dim3((unsigned)(t8 + rem)), dim3(256), 0, hargs);
+        } else if (narrow)
           launch(ctx, g, s->prog, "skl_ap_zr4", dim3((unsigned)cdiv(m, 64), (unsigned)rows), dim3(256), 0, args);
         else
           launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)rows), dim3(256), 0, args);

@@ -222,8 +222,10 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->xfer_chunks = (int)value;
     } else if (k == "map_interleave") {
       c->map_interleave = value ? 1 : 0;
+    } else if (k == "ap_hybrid") {
+      c->ap_hybrid = value ? 1 : 0;
     } else if (k == "ap_tile") {
-      if (value != 0 && value != 4 && value != 8) fail(SKL_ERR_INVALID_ARG, "ap_tile in {0,4,8}");
+      if (value != 0 && value != 2 && value != 4 && value != 8) fail(SKL_ERR_INVALID_ARG, "ap_tile in {0,2,4,8}");
       c->ap_tile = (int)value;
     } else if (k == "ap_fast") {
       c->ap_fast = value ? 1 : 0;

@@ -119,15 +119,16 @@ __device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][TC], const SKL_T
     }
   }
 }
-// One 128 x (16 TC) tile of C per block of 256 threads, 8 x TC per thread.
+// One 128 x (16 TC) tile of C at (i0, j0) per block of 256 threads, 8 x TC per
+// thread; sm holds 2 * (128 + 16 TC) * AQ_P elements.
+#define AQ_STAGE(TC) ((AQ_BM + 16 * (TC)) * AQ_P)
 template <int TC>
 __device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B,
-                                            SKL_TOUT* __restrict__ Cm, long n, long m, long d) {
+                                            SKL_TOUT* __restrict__ Cm, long n, long m, long d, long i0, long j0,
+                                            SKL_TIN* sm) {
   constexpr int BN = 16 * TC;                      // tile columns (rows of B)
-  constexpr int STAGE = (AQ_BM + BN) * AQ_P;
-  __shared__ __align__(16) SKL_TIN sm[2 * STAGE];
+  constexpr int STAGE = AQ_STAGE(TC);
   const int tx = threadIdx.x & 15, ty = threadIdx.x >> 4;
-  const long i0 = (long)blockIdx.y * AQ_BM, j0 = (long)blockIdx.x * BN;
   const long nfull = d / AQ_BK;
   // chunk q of a (rows x 16) slab: row q / 4, k-quad q % 4 (rows beyond n / m
   // are clamped to the last one: loaded, never stored)
@@ -214,12 +215,32 @@ __device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const
 extern "C" __global__ void __launch_bounds__(256, 2)
 skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
            long n, long m, long d) {
-  skl_ap_tile<8>(A, B, Cm, n, m, d);
+  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(8)];
+  skl_ap_tile<8>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 128, sm);
 }
 extern "C" __global__ void __launch_bounds__(256, 3)
 skl_ap_zr4(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
            long n, long m, long d) {
-  skl_ap_tile<4>(A, B, Cm, n, m, d);
+  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(4)];
+  skl_ap_tile<4>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 64, sm);
+}
+// Wave-quantisation fix: the 128 x 128 tiles (row-major, tiles_x per row) that
+// fill whole waves run as such (blocks 0 .. nwide-1); each tile of the last,
+// partial wave is split into two 128 x 64 halves (blocks nwide ..), so the
+// last wave has twice the blocks, each half the work.  Every C element is still
+// folded in k order by one thread (bit-exact).
+extern "C" __global__ void __launch_bounds__(256, 2)
+skl_ap_zrh(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
+           long n, long m, long d, long nwide, long tiles_x) {
+  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(8)];
+  const long b = blockIdx.x;
+  if (b < nwide) {
+    skl_ap_tile<8>(A, B, Cm, n, m, d, (b / tiles_x) * AQ_BM, (b % tiles_x) * 128, sm);
+  } else {
+    const long t = nwide + (b - nwide) / 2;
+    const long j0 = (t % tiles_x) * 128 + ((b - nwide) & 1) * 64;
+    if (j0 < m) skl_ap_tile<4>(A, B, Cm, n, m, d, (t / tiles_x) * AQ_BM, j0, sm);
+  }
 }
 #endif
 #else

@@ -75,9 +75,10 @@ def test_size_mismatch(ctx, sk):
     assert e.value.name == "SIZE_MISMATCH"
 
 
-@pytest.mark.parametrize("tile", [4, 8])
+@pytest.mark.parametrize("tile", [2, 4, 8])
 def test_forced_tile_widths_bitexact(ctx, sk, tile):
-    """both 128-row kernels (128 x 64 and 128 x 128 tiles of C) agree with the oracle"""
+    """the 128-row kernels (128 x 64 and 128 x 128 tiles of C, and the hybrid of
+    both, here with every tile split) agree with the oracle"""
     ctx.set_option("ap_tile", tile)
     try:
         for n, m, d in ((130, 200, 64), (257, 129, 100), (5, 300, 4)):
@@ -88,3 +89,17 @@ def test_forced_tile_widths_bitexact(ctx, sk, tile):
             assert np.array_equal(sk["man_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_MANHATTAN, a, b))
     finally:
         ctx.set_option("ap_tile", 0)
+
+
+def test_hybrid_last_wave_bitexact(ctx, sk):
+    """automatic hybrid: 18 x 18 = 324 tiles of 128 x 128 on one device leave the
+    last wave (296 slots) 28 tiles deep, which run as 56 halves of 128 x 64;
+    ragged n and m put some halves partly or wholly beyond the matrix"""
+    G = ctx.ndev
+    for n, m, d in ((2304 * G, 2304, 8), (2300 * G - 3, 2290, 12)):
+        a = I.uniform_f32(87, n * d).reshape(n, d) - np.float32(0.5)
+        b = I.uniform_f32(88, m * d).reshape(m, d) - np.float32(0.5)
+        ma = S.Matrix.from_numpy(ctx, a).set_distribution(S.BLOCK)
+        mb = S.Matrix.from_numpy(ctx, b)
+        assert np.array_equal(sk["dot_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_DOT, a, b))
+        assert np.array_equal(sk["man_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_MANHATTAN, a, b))
