@@ -30,6 +30,7 @@ Skel* allpairs_create(Ctx* ctx, const char* src, const char* entry, const char* 
   s->ap_zr = rsrc != nullptr;
   std::string defs = "#define SKL_BLOCK 256\n#define SKL_DEBUG_BOUNDS 0\n";
   defs += std::string("#define SKL_AP_FAST ") + (si == 4 ? "1" : "0") + "\n";
+  if (ctx->ap_bk) defs += "#define SKL_AP_BK " + std::to_string(ctx->ap_bk) + "\n";
   defs += "#define SKL_TIN " + ctx->type(tin).name + "\n#define SKL_TOUT " + ctx->type(tout).name + "\n";
   std::string body;
   if (s->ap_zr) {
@@ -98,17 +99,20 @@ void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out) {
         if (ctx->ap_tile == 4) narrow = true;
         // hybrid: whole waves of 128 x 128 tiles, the partial last wave as
         // 128 x 64 halves (when they fit one wave of 2 blocks per SM)
+        // shared memory: two stages of (128 + tile columns) rows x (bk + 4) elements
+        const size_t bk = ctx->ap_bk ? (size_t)ctx->ap_bk : 16;
+        const size_t sm8 = 2 * (128 + 128) * (bk + 4) * si, sm4 = 2 * (128 + 64) * (bk + 4) * si;
         const size_t slots = 2 * sms, rem = t8 % slots;
         const bool hybrid = (ctx->ap_tile == 0 || ctx->ap_tile == 2) && ctx->ap_hybrid && t8 > slots &&
                             rem != 0 && 2 * rem <= slots;
         if (hybrid || ctx->ap_tile == 2) {
           long nwide = (long)(t8 - rem), tiles_x = (long)cdiv(m, 128);
           void* hargs[] = {(void*)&pa, (void*)&pb, &pc, &nn, &mm, &dd, &nwide, &tiles_x};
-          launch(ctx, g, s->prog, "skl_ap_zrh", dim3((unsigned)(t8 + rem)), dim3(256), 0, hargs);
+          launch(ctx, g, s->prog, "skl_ap_zrh", dim3((unsigned)(t8 + rem)), dim3(256), sm8, hargs);
         } else if (narrow)
-          launch(ctx, g, s->prog, "skl_ap_zr4", dim3((unsigned)cdiv(m, 64), (unsigned)rows), dim3(256), 0, args);
+          launch(ctx, g, s->prog, "skl_ap_zr4", dim3((unsigned)cdiv(m, 64), (unsigned)rows), dim3(256), sm4, args);
         else
-          launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)rows), dim3(256), 0, args);
+          launch(ctx, g, s->prog, "skl_ap_zr8", dim3((unsigned)cdiv(m, 128), (unsigned)rows), dim3(256), sm8, args);
       } else {
         launch(ctx, g, s->prog, "skl_ap_zr", dim3((unsigned)cdiv(m, 64), (unsigned)cdiv(r.size(), 64)),
                dim3(256), 0, args);

@@ -222,6 +222,9 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->xfer_chunks = (int)value;
     } else if (k == "map_interleave") {
       c->map_interleave = value ? 1 : 0;
+    } else if (k == "ap_bk") {
+      if (value != 0 && value != 16 && value != 32) fail(SKL_ERR_INVALID_ARG, "ap_bk in {0,16,32}");
+      c->ap_bk = (int)value;
     } else if (k == "ap_hybrid") {
       c->ap_hybrid = value ? 1 : 0;
     } else if (k == "ap_tile") {

@@ -87,8 +87,13 @@ skl_ap_zr(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT
 // a double buffer; per k-quad a thread issues 16 LDS.128 for 512 FP32 ops.
 // Every accumulator is still folded in k order (bit-exact with the oracle).
 #define AQ_BM 128
+#ifdef SKL_AP_BK
+#define AQ_BK SKL_AP_BK
+#else
 #define AQ_BK 16
+#endif
 #define AQ_P (AQ_BK + 4)
+#define AQ_CPR (AQ_BK / 4)   // 16-byte chunks per staged row
 union SklAp4 {
   uint4 q;
   SKL_TIN e[4];
@@ -97,18 +102,19 @@ __device__ __forceinline__ void skl_ap_cp16(void* smem, const void* g) {
   const unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
   asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(sa), "l"(g) : "memory");
 }
+// 16 k of a staged slice, from column koff (unrolled body; deeper slices loop over it)
 template <bool FIRST, int TC>
-__device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][TC], const SKL_TIN* As, const SKL_TIN* Bs,
-                                             int tx, int ty) {
+__device__ __forceinline__ void skl_ap_slice16(SKL_TOUT (&acc)[8][TC], const SKL_TIN* As, const SKL_TIN* Bs,
+                                               int tx, int ty, int koff) {
 #pragma unroll
-  for (int kq = 0; kq < AQ_BK; kq += 4) {
+  for (int kq = 0; kq < 16; kq += 4) {
     SklAp4 a[8];
 #pragma unroll
-    for (int r = 0; r < 8; ++r) a[r].q = *(const uint4*)&As[(ty + 16 * r) * AQ_P + kq];
+    for (int r = 0; r < 8; ++r) a[r].q = *(const uint4*)&As[(ty + 16 * r) * AQ_P + koff + kq];
 #pragma unroll
     for (int c = 0; c < TC; ++c) {
       SklAp4 b;
-      b.q = *(const uint4*)&Bs[(tx + 16 * c) * AQ_P + kq];
+      b.q = *(const uint4*)&Bs[(tx + 16 * c) * AQ_P + koff + kq];
 #pragma unroll
       for (int j = 0; j < 4; ++j)
 #pragma unroll
@@ -118,6 +124,13 @@ __device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][TC], const SKL_T
         }
     }
   }
+}
+template <bool FIRST, int TC>
+__device__ __forceinline__ void skl_ap_slice(SKL_TOUT (&acc)[8][TC], const SKL_TIN* As, const SKL_TIN* Bs,
+                                             int tx, int ty) {
+  skl_ap_slice16<FIRST, TC>(acc, As, Bs, tx, ty, 0);
+#pragma unroll 1
+  for (int k16 = 16; k16 < AQ_BK; k16 += 16) skl_ap_slice16<false, TC>(acc, As, Bs, tx, ty, k16);
 }
 // One 128 x (16 TC) tile of C at (i0, j0) per block of 256 threads, 8 x TC per
 // thread; sm holds 2 * (128 + 16 TC) * AQ_P elements.
@@ -132,16 +145,16 @@ __device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const
   const long nfull = d / AQ_BK;
   // chunk q of a (rows x 16) slab: row q / 4, k-quad q % 4 (rows beyond n / m
   // are clamped to the last one: loaded, never stored)
-  constexpr int HA = AQ_BM * 4 / 256, HB = BN * 4 / 256;   // chunks per thread
+  constexpr int HA = AQ_BM * AQ_CPR / 256, HB = BN * AQ_CPR / 256;   // chunks per thread
   long ra[HA], rb[HB];
 #pragma unroll
   for (int h = 0; h < HA; ++h) {
-    const int r = (threadIdx.x + h * 256) >> 2;
+    const int r = (threadIdx.x + h * 256) / AQ_CPR;
     ra[h] = (i0 + r < n ? i0 + r : n - 1) * d;
   }
 #pragma unroll
   for (int h = 0; h < HB; ++h) {
-    const int r = (threadIdx.x + h * 256) >> 2;
+    const int r = (threadIdx.x + h * 256) / AQ_CPR;
     rb[h] = (j0 + r < m ? j0 + r : m - 1) * d;
   }
   auto stage = [&](int st, long k0) {
@@ -149,12 +162,12 @@ __device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const
     SKL_TIN* Bs = As + AQ_BM * AQ_P;
 #pragma unroll
     for (int h = 0; h < HA; ++h) {
-      const int q = threadIdx.x + h * 256, r = q >> 2, kq = (q & 3) * 4;
+      const int q = threadIdx.x + h * 256, r = q / AQ_CPR, kq = (q % AQ_CPR) * 4;
       skl_ap_cp16(&As[r * AQ_P + kq], A + ra[h] + k0 + kq);
     }
 #pragma unroll
     for (int h = 0; h < HB; ++h) {
-      const int q = threadIdx.x + h * 256, r = q >> 2, kq = (q & 3) * 4;
+      const int q = threadIdx.x + h * 256, r = q / AQ_CPR, kq = (q % AQ_CPR) * 4;
       skl_ap_cp16(&Bs[r * AQ_P + kq], B + rb[h] + k0 + kq);
     }
   };
@@ -215,14 +228,14 @@ __device__ __forceinline__ void skl_ap_tile(const SKL_TIN* __restrict__ A, const
 extern "C" __global__ void __launch_bounds__(256, 2)
 skl_ap_zr8(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
            long n, long m, long d) {
-  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(8)];
-  skl_ap_tile<8>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 128, sm);
+  extern __shared__ __align__(16) unsigned char skl_ap_dyn[];   // 2 * AQ_STAGE(8) elements
+  skl_ap_tile<8>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 128, (SKL_TIN*)skl_ap_dyn);
 }
 extern "C" __global__ void __launch_bounds__(256, 3)
 skl_ap_zr4(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
            long n, long m, long d) {
-  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(4)];
-  skl_ap_tile<4>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 64, sm);
+  extern __shared__ __align__(16) unsigned char skl_ap_dyn[];   // 2 * AQ_STAGE(4) elements
+  skl_ap_tile<4>(A, B, Cm, n, m, d, (long)blockIdx.y * AQ_BM, (long)blockIdx.x * 64, (SKL_TIN*)skl_ap_dyn);
 }
 // Wave-quantisation fix: the 128 x 128 tiles (row-major, tiles_x per row) that
 // fill whole waves run as such (blocks 0 .. nwide-1); each tile of the last,
@@ -232,7 +245,8 @@ skl_ap_zr4(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOU
 extern "C" __global__ void __launch_bounds__(256, 2)
 skl_ap_zrh(const SKL_TIN* __restrict__ A, const SKL_TIN* __restrict__ B, SKL_TOUT* __restrict__ Cm,
            long n, long m, long d, long nwide, long tiles_x) {
-  __shared__ __align__(16) SKL_TIN sm[2 * AQ_STAGE(8)];
+  extern __shared__ __align__(16) unsigned char skl_ap_dyn[];   // 2 * AQ_STAGE(8) elements
+  SKL_TIN* sm = (SKL_TIN*)skl_ap_dyn;
   const long b = blockIdx.x;
   if (b < nwide) {
     skl_ap_tile<8>(A, B, Cm, n, m, d, (b / tiles_x) * AQ_BM, (b % tiles_x) * 128, sm);

@@ -147,6 +147,7 @@ struct Ctx {
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
   int ap_fast = 1;             // Allpairs zip-reduce: 128-row tiles (4-byte inputs, d % 4 == 0)
   int ap_tile = 0;             // Allpairs tile columns: 0 = by wave fill, 8 = 128, 4 = 64, 2 = hybrid
+  int ap_bk = 0;               // Allpairs 128-row kernels: k-slice depth (0 = 16)
   int ap_hybrid = 1;           // Allpairs: last partial wave of 128 x 128 tiles as 128 x 64 halves           // MapOverlap stores its border rows into the neighbours' halos
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 6 = one block per tile, tile kept in shared memory, low

@@ -103,3 +103,21 @@ def test_hybrid_last_wave_bitexact(ctx, sk):
         mb = S.Matrix.from_numpy(ctx, b)
         assert np.array_equal(sk["dot_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_DOT, a, b))
         assert np.array_equal(sk["man_zr"](ma, mb).to_numpy(), O.allpairs(O.AP_MANHATTAN, a, b))
+
+
+@pytest.mark.parametrize("tile", [0, 4, 8])
+def test_k_slice_32_bitexact(ctx, sk, tile):
+    """32-deep k-slices (ap_bk=32, dynamic shared memory): d below one slice,
+    one slice plus a tail, several slices plus a tail"""
+    ctx.set_option("ap_bk", 32)
+    ctx.set_option("ap_tile", tile)
+    try:
+        sk2 = S.Allpairs(ctx, A.MULT, S.F32, S.F32, reduce=A.ADD)
+        for n, m, d in ((130, 200, 20), (257, 129, 36), (129, 300, 100), (64, 64, 64)):
+            a = I.uniform_f32(89, n * d).reshape(n, d) - np.float32(0.5)
+            b = I.uniform_f32(90, m * d).reshape(m, d) - np.float32(0.5)
+            ma, mb = S.Matrix.from_numpy(ctx, a), S.Matrix.from_numpy(ctx, b)
+            assert np.array_equal(sk2(ma, mb).to_numpy(), O.allpairs(O.AP_DOT, a, b))
+    finally:
+        ctx.set_option("ap_bk", 0)
+        ctx.set_option("ap_tile", 0)

@@ -111,9 +111,10 @@ def dot20():
 
 
 def allpairs():
-    """AP_CFGS="tile,...": 4096^3 dot and 4096x4096x128 Manhattan, zip-reduce form"""
-    for tile in (int(x) for x in os.environ.get("AP_CFGS", "0").split(",")):
-        c = ctx_with({"ap_tile": tile})
+    """AP_CFGS="tile[:bk],...": 4096^3 dot and 4096x4096x128 Manhattan, zip-reduce form"""
+    for cfg in os.environ.get("AP_CFGS", "0").split(","):
+        tile, bk = (int(v) for v in (cfg.split(":") + ["0"])[:2])
+        c = ctx_with({"ap_tile": tile, "ap_bk": bk})
         for name, z, dd in (("dot", A.MULT, 4096), ("manhattan", A.ABSDIFF, 128)):
             a = I.uniform_f32(81, 4096 * dd).reshape(4096, dd)
             b = I.uniform_f32(82, 4096 * dd).reshape(4096, dd)
@@ -125,7 +126,7 @@ def allpairs():
             fn = O.AP_DOT if z == A.MULT else O.AP_MANHATTAN
             ok = np.array_equal(cg[:16, :40], O.allpairs(fn, a[:16], b[:40]))
             tf = 2.0 * 4096 * 4096 * dd / (ms / 1e3) / 1e12
-            print(f"allpairs {name:9s} tile={tile}: {ms:.4f} ms  {tf:.2f} TFLOP/s  bitexact={ok}", flush=True)
+            print(f"allpairs {name:9s} tile={tile} bk={bk}: {ms:.4f} ms  {tf:.2f} TFLOP/s  bitexact={ok}", flush=True)
         c.finalize()
 
 
