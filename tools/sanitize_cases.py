@@ -107,8 +107,38 @@ def logical_devices(G):
     ctx.finalize()
 
 
+def tma_and_hybrid(G):
+    """TMA / warp-specialised MapOverlap (mbarrier ring, border patching, parts
+    with halo rows on G logical devices, fused halo push) and the hybrid Allpairs
+    launch (every tile split)"""
+    ctx = S.Context(G, devices=[0] * G)
+    ctx.set_option("mo_ws", 1)
+    ctx.set_option("mo_ws_stages", 2)
+    ctx.set_option("mo_cw", 4)
+    ctx.set_option("ap_tile", 2)
+    n0 = ctx.counter("tma_launches")
+    img8 = I.image_u8(5, 70, 144)
+    sob = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+    assert np.array_equal(sob(S.Matrix.from_numpy(ctx, img8)).to_numpy(),
+                          O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0))
+    imgf = I.image_f32(6, 150, 272)
+    gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    g2 = gau(gau(S.Matrix.from_numpy(ctx, imgf)))
+    r1 = O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0)
+    assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
+    assert ctx.counter("tma_launches") - n0 == 3 * G
+    a = I.uniform_f32(8, 130 * 36).reshape(130, 36)
+    b = I.uniform_f32(9, 200 * 36).reshape(200, 36)
+    ap = S.Allpairs(ctx, A.MULT, S.F32, S.F32, reduce=A.ADD)
+    assert np.array_equal(ap(S.Matrix.from_numpy(ctx, a).set_distribution(S.BLOCK),
+                             S.Matrix.from_numpy(ctx, b)).to_numpy(), O.allpairs(O.AP_DOT, a, b))
+    ctx.finalize()
+
+
 if __name__ == "__main__":
     one_device({})
     one_device({"scan_variant": 3, "map_interleave": 1, "block_threads": 128})
     logical_devices(3)
+    tma_and_hybrid(1)
+    tma_and_hybrid(2)
     print("sanitize cases ok", flush=True)
