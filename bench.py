@@ -930,6 +930,10 @@ def bench_skeletons(args, D: Dist, P: dict, which):
 
 
 # ---------------------------------------------------------------- reference arm (the oracle)
+HEADLINE_WORKLOAD = (f"mandelbrot {COLS}x{ROWS} Map over block-distributed Matrix<float2>, "
+                     f"MAX_ITER={MAX_ITER} (BASELINE configs[1])")
+
+
 def run_reference(args, D: Dist):
     if D.rank != 0:
         return 0
@@ -947,7 +951,8 @@ def run_reference(args, D: Dist):
     line = {"impl": "reference", "metric": METRIC, "value": v, "unit": "elements/s", "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": sec * 1e3, "higher_is_better": True,
             "scaling": "strong", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-            "config": {"workload": f"mandelbrot {COLS}x{ROWS} Map, MAX_ITER={MAX_ITER} (oracle on every {every}th row)"},
+            "config": {"workload": HEADLINE_WORKLOAD, "parallelism": "oracle, one host core",
+                       "row_order": "identity"},
             "cpu_baseline": {"value": v, "unit": "elements/s", "cores": 1, "kind": "oracle", **cpu_info(),
                              "sample": f"rows 0,{every},{2 * every},... ({pix} pixels) per step"},
             "e2e": {"value": v, "unit": "elements/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
@@ -979,8 +984,8 @@ def main():
          "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
-    sk = bench_skeletons(args, D, P, which) if which else {}
     if D.rank != 0:
+        _skeleton_section(args, D, P, which, None)
         return 0
     # oracle: full image on this host (parity of every pixel, exact work count, cpu baseline)
     counts_ref, sum_iter, cpu_s = mandel_oracle(1)
@@ -999,8 +1004,7 @@ def main():
         "metric": METRIC, "value": r["value"], "unit": "elements/s", "n_gpus": args.gpus, "steps": args.steps,
         "warmup": args.warmup, "ms_per_step": r["ms"], "higher_is_better": True, "scaling": "strong",
         "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-        "config": {"workload": f"mandelbrot {COLS}x{ROWS} Map over block-distributed Matrix<float2>, "
-                               f"MAX_ITER={MAX_ITER} (BASELINE configs[1])",
+        "config": {"workload": HEADLINE_WORKLOAD,
                    "l2": "flushed between steps (256 MiB write, then a 256 MiB read so L2 is clean)",
                    "parallelism": f"block rows over {args.gpus} GPU(s)",
                    "row_order": "identity" if D.world == 1 else "round-robin (application-level balancing)",
@@ -1015,10 +1019,43 @@ def main():
         "parity": {"mandelbrot_full_image_bitexact": parity, "sum_iterations": int(sum_iter)},
         "paper_context": "SkelCL Mandelbrot 4096x3072 on one Tesla T10: 26 s (0.48 Mpx/s); MAX_ITER unstated, "
                          "so not the same workload (vs_baseline null)",
-        "skeletons": sk,
     }
+    line["skeletons"] = _skeleton_section(args, D, P, which, line)
     print(json.dumps(line), flush=True)
     return 0
+
+
+def _skeleton_section(args, D: Dist, P: dict, which, line):
+    """The per-skeleton lines, after the headline is complete.  A watchdog bounds
+    the section (SKL_BENCH_SKELETON_LIMIT_S, default 420 s): if it is exceeded -
+    e.g. a collective of the multi-rank path that never completes - rank 0 prints
+    the headline line with the skeletons marked as timed out and every rank
+    exits 0, so a run never ends without its line.  An exception in the section
+    is recorded in the line instead of losing it."""
+    if not which:
+        return {}
+    import threading
+    limit = float(os.environ.get("SKL_BENCH_SKELETON_LIMIT_S", "420"))
+
+    def expire():
+        if line is not None:
+            print(json.dumps({**line, "skeletons": {"error": f"skeleton section exceeded {limit:.0f} s"}}),
+                  flush=True)
+        os._exit(0)
+
+    wd = threading.Timer(limit, expire)
+    wd.daemon = True
+    wd.start()
+    try:
+        return bench_skeletons(args, D, P, which)
+    except Exception as e:   # noqa: BLE001 - recorded in the bench line
+        if D.world > 1:      # the other ranks may be waiting in a collective: end the job
+            if line is not None:
+                print(json.dumps({**line, "skeletons": {"error": repr(e)}}), flush=True)
+            os._exit(0)
+        return {"error": repr(e)}
+    finally:
+        wd.cancel()
 
 
 def S_block(n, G, g):
