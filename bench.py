@@ -3,7 +3,7 @@
 task statement; DESIGN.md §"Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,sobel,gauss,redist,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
+                    [--skeletons all|none|dot,sobel,gauss,gauss_iter,sobel_iter,redist,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
 block-distributed Matrix<float2> of pixel coordinates (MAX_ITER 1000, window
@@ -625,38 +625,48 @@ def bench_skeletons(args, D: Dist, P: dict, which):
     if "redist" in which and D.world == 1:
         res.update(bench_redist(ctx, timer, K, W, D, P))
 
-    if "gauss_iter" in which:
-        # K=10 iterated Gaussian (ping-pong); on several GPUs the halo
-        # rows move between iterations (NCCL, one process per GPU)
+    for it_name in ("gauss_iter", "sobel_iter"):
+        if it_name not in which:
+            continue
+        # K=10 iterated stencil (ping-pong); on several GPUs the
+        # halo rows move between iterations (NCCL, one process per GPU)
         R = C = 8192
-        img = I.image_f32(I.SEED_GAUSS, R, C)
-        ctx.set_option("block_threads", 128)
-        gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
-        ctx.set_option("block_threads", 256)
+        if it_name == "gauss_iter":
+            img = I.image_f32(I.SEED_GAUSS, R, C)
+            ctx.set_option("block_threads", 128)
+            st = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+            ctx.set_option("block_threads", 256)
+            dt, okind, dd, ob, nv = S.F32, O.OS_GAUSS5, 2, O.OB_NEAREST, 0.0
+            desc = "Gaussian 5x5 f32"
+        else:
+            img = I.image_u8(I.SEED_SOBEL, R, C)
+            st = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            dt, okind, dd, ob, nv = S.U8, O.OS_SOBEL, 1, O.OB_NEUTRAL, 0
+            desc = "Sobel u8"
         a = S.Matrix.from_numpy(ctx, img)
-        b = S.Matrix(ctx, S.F32, R, C)
-        t = S.Matrix(ctx, S.F32, R, C)
+        b = S.Matrix(ctx, dt, R, C)
+        t = S.Matrix(ctx, dt, R, C)
         ITER = 10
 
         def step(_):
-            gau(a, out=b)
+            st(a, out=b)
             for k in range(ITER - 1):
-                gau(b, out=t) if k % 2 == 0 else gau(t, out=b)
+                st(b, out=t) if k % 2 == 0 else st(t, out=b)
 
         ms, _ = timer.run(step, max(3, K // 4), W, D)
         ms = D.max(ms)
         # parity: rows 4000..4063 after 10 iterations (the oracle iterates a band wide
-        # enough that its edges do not reach the checked rows: 10 x d = 20 rows)
+        # enough that its edges do not reach the checked rows: 10 x d <= 20 rows)
         sub = img[3970:4094]
         r = sub
         for _ in range(ITER):
-            r = O.mapoverlap2d(O.OS_GAUSS5, r, 2, O.OB_NEAREST, 0.0)
+            r = O.mapoverlap2d(okind, r, dd, ob, nv)
         fin = (t if (ITER - 1) % 2 == 1 else b)
         ok = bool(np.array_equal(fin.to_numpy()[4000:4064], r[30:94]))
-        res["gauss_iter10"] = {"workload": f"10 x Gaussian 5x5 f32 MapOverlap {R}x{C}, ping-pong (halo refresh "
-                                           "between iterations on >1 GPU)",
-                               "ms": round(ms, 4), "ms_per_iteration": round(ms / ITER, 4),
-                               "elements_per_s": ITER * R * C / (ms / 1e3), "check": "ok" if ok else "FAIL"}
+        res[it_name.replace("_iter", "_iter10")] = {
+            "workload": f"10 x {desc} MapOverlap {R}x{C}, ping-pong (halo refresh between iterations on >1 GPU)",
+            "ms": round(ms, 4), "ms_per_iteration": round(ms / ITER, 4),
+            "elements_per_s": ITER * R * C / (ms / 1e3), "check": "ok" if ok else "FAIL"}
         for x in (a, b, t):
             x.destroy()
 
@@ -980,7 +990,7 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, D, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "redist", "scan_i32", "scan_f32", "lmosem",
+        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32", "scan_f32", "lmosem",
          "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
