@@ -131,7 +131,11 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * "xfer_kernel" (1 = with several devices in this process, the moves of a
  * redistribution or halo refresh into one GPU run as one batched copy kernel
  * (peer loads over NVLink between GPUs); 0 = one cudaMemcpy(Peer)Async per
- * move; default 1),
+ * move; default 1), "combine_peer" (copy(+) -> block with every device in
+ * this process: 1 = each device folds its slice straight out of the peers'
+ * replicas in one kernel, no staging copy; logical devices of one GPU share one
+ * launch; 2 = one kernel per device even then; 0 = slices exchanged into
+ * staging, then folded; default 1),
  * "mo_ws" (1 = 2-D MapOverlap tiles are staged by a TMA producer warp into a
  * ring of "mo_ws_stages" shared-memory buffers consumed by the other warps of
  * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged

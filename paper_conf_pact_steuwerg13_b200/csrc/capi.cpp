@@ -215,6 +215,12 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       (k == "mo_rh" ? c->mo_rh : c->mo_cw) = (int)value;
     } else if (k == "lazy_fusion") {
       c->lazy_fusion = value ? 1 : 0;
+    } else if (k == "combine_unroll") {
+      if (value < 0 || value > 8) fail(SKL_ERR_INVALID_ARG, "combine_unroll in [0,8]");
+      c->combine_unroll = (int)value;
+    } else if (k == "combine_peer") {
+      if (value < 0 || value > 2) fail(SKL_ERR_INVALID_ARG, "combine_peer in {0,1,2}");
+      c->combine_peer = (int)value;
     } else if (k == "xfer_kernel") {
       c->xfer_kernel = value ? 1 : 0;
     } else if (k == "xfer_chunks") {

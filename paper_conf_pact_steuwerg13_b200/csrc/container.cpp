@@ -404,6 +404,44 @@ static void combine_to_block(Cont* c) {
     set_valid(c, blk, false);
     return;
   }
+  // one process driving every device, each able to load from every replica,
+  // <= 8 replicas: one fused exchange + fold kernel per device (peer loads), the
+  // fold written in place into the device's own replica
+  bool fused = ctx->combine_peer && ctx->xfer_kernel && !ctx->dist_mode && ctx->nlocal == G && G <= 8;
+  for (int g = 0; fused && g < G; ++g)
+    for (int h = 0; h < G; ++h)
+      fused = fused && ctx->peer_ok[(size_t)g][(size_t)h] && c->parts[(size_t)h].ptr &&
+              c->parts[(size_t)h].buf.contains(Range{0, U});
+  if (fused) {
+    NvtxRange nr("skl_combine_peer");
+    barrier_streams(ctx);  // every replica is final before any device reads it
+    std::vector<const void*> srcs((size_t)G);
+    bool one_gpu = ctx->combine_peer != 2;  // 2: one kernel per device even on one GPU (tests)
+    for (int g = 0; g < G; ++g) one_gpu = one_gpu && ctx->D(g).phys == ctx->D(0).phys;
+    if (one_gpu) {
+      // logical devices of one GPU: every slice folded by one launch
+      for (int h = 0; h < G; ++h) srcs[(size_t)h] = part_ptr(c, h, 0);
+      ctx->p2p += (long long)((size_t)(G - 1) * U * ub);
+      run_combine_all(c->combine, 0, srcs.data(), G, U * c->cols, (U + (size_t)G - 1) / (size_t)G * c->cols);
+    }
+    for (int g = 0; g < G && !one_gpu; ++g) {
+      const Range r = block_range(U, G, g);
+      if (r.empty()) continue;
+      for (int h = 0; h < G; ++h) srcs[(size_t)h] = part_ptr(c, h, r.lo);
+      ctx->p2p += (long long)((size_t)(G - 1) * r.size() * ub);
+      run_combine_peer(c->combine, g, srcs.data(), G, part_ptr(c, g, r.lo), r.size() * c->cols);
+    }
+    barrier_streams(ctx);  // no device overwrites its replica while a peer still reads it
+    for (int g = 0; g < G; ++g)
+      if (block_range(U, G, g).empty()) free_part(c, g);
+    c->dist = blk;
+    c->diverged = false;
+    c->dev_valid = true;
+    c->halo_valid = false;
+    c->halo_ready = 0;
+    set_valid(c, blk, false);
+    return;
+  }
   std::vector<void*> staging((size_t)G, nullptr);
   std::vector<Transfer> tr;
   for (int g = 0; g < G; ++g) {

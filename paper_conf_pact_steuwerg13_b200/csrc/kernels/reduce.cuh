@@ -278,3 +278,158 @@ skl_combine(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep, SKL_T* 
   (void)vec;
   skl_combine_run<1>(staging, stride, nrep, out, n);
 }
+
+// copy(+) -> block fused with its exchange (reading A25; one process driving
+// every device): device g folds its block slice straight out of every replica
+// (peer loads over NVLink, or the same GPU for logical devices) in device order,
+// out[i] = src[0][i] (+) src[1][i] (+) ... (+) src[nrep-1][i], and writes the
+// result in place into its own replica - a reduce-scatter with the user's
+// operator in one kernel, no staging copy.  In place is safe: device g writes
+// only its own slice of its own replica, which no other device reads.
+struct SklSrcs {
+  const SKL_T* p[SKL_CMAXR];
+};
+template <int V>
+__device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep, SKL_T* out, skl_u64 n_chunks) {
+  SklOp op;
+  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i < n_chunks;
+       i += (skl_u64)gridDim.x * SKL_BLOCK) {
+    SklChunk<SKL_T, V> x[SKL_CMAXR];
+#pragma unroll
+    for (int r = 0; r < SKL_CMAXR; ++r)
+      if (r < nrep) {
+        if (V > 1) x[r].q[0] = skl_ld16(s.p[r] + i * V);
+        else x[r].e[0] = s.p[r][i];
+      }
+    SklChunk<SKL_T, V> a = x[0];
+#pragma unroll
+    for (int r = 1; r < SKL_CMAXR; ++r)
+      if (r < nrep) {
+#pragma unroll
+        for (int k = 0; k < V; ++k) a.e[k] = op(a.e[k], x[r].e[k]);
+      }
+    if (V > 1) skl_st16(out + i * V, a.q[0]);
+    else out[i] = a.e[0];
+  }
+}
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
+#if SKL_RVEC > 1
+  if (vec) {
+    const skl_u64 nc = n / SKL_RVEC;
+    skl_combine_peer_run<SKL_RVEC>(s, nrep, out, nc);
+    const skl_u64 t0 = nc * SKL_RVEC;
+    if (blockIdx.x == 0 && threadIdx.x < n - t0) {
+      SklOp op;
+      const skl_u64 i = t0 + threadIdx.x;
+      SKL_T a = s.p[0][i];
+#pragma unroll
+      for (int r = 1; r < SKL_CMAXR; ++r)   // constant indices: the pointers stay in registers
+        if (r < nrep) a = op(a, s.p[r][i]);
+      out[i] = a;
+    }
+    return;
+  }
+#endif
+  (void)vec;
+  skl_combine_peer_run<1>(s, nrep, out, n);
+}
+
+// The same fold for logical devices sharing one GPU, in ONE launch: bases[h] is
+// replica h at unit 0 (every replica covers all n elements); element e belongs
+// to device e / chunk, whose replica receives the fold (chunk = the block
+// distribution's ceil(units / G) units in elements; a multiple of SKL_RVEC for
+// the 16-byte path).
+#ifndef SKL_CUNR
+#define SKL_CUNR 2
+#endif
+// SKL_CUNR chunks per thread and step: all their replica loads are issued
+// before the first store (the output aliases a replica, so the compiler cannot
+// hoist the next step's loads above this step's stores on its own)
+// Replica of the device owning element e: e / chunk through a float reciprocal
+// (within one of the true quotient for any e < 2^40 and <= 8 devices), fixed by
+// two exact compares - a 64-bit integer division is a ~100-instruction software
+// routine and made this kernel issue-bound - then selected with constant
+// indices (the pointer table stays in registers).
+__device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, skl_u64 e, skl_u64 chunk,
+                                                    float inv_chunk) {
+  int o = (int)((float)e * inv_chunk);
+  if ((skl_u64)o * chunk > e) --o;
+  if ((skl_u64)(o + 1) * chunk <= e) ++o;
+  o = o < 0 ? 0 : (o > nrep - 1 ? nrep - 1 : o);
+  SKL_T* out = const_cast<SKL_T*>(s.p[0]);
+#pragma unroll
+  for (int r = 1; r < SKL_CMAXR; ++r)
+    if (r == o) out = const_cast<SKL_T*>(s.p[r]);
+  return out;
+}
+template <int V>
+__device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, skl_u64 n_chunks, skl_u64 chunk) {
+  SklOp op;
+  const float inv_chunk = 1.0f / (float)chunk;
+  const skl_u64 stride = (skl_u64)gridDim.x * SKL_BLOCK;
+  for (skl_u64 i0 = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i0 < n_chunks; i0 += stride * SKL_CUNR) {
+    SklChunk<SKL_T, V> a[SKL_CUNR];
+    // replicas in groups of 4 (registers for 4, not SKL_CMAXR, replica chunks
+    // per step), folded left to right as each group arrives
+#pragma unroll
+    for (int g0 = 0; g0 < SKL_CMAXR; g0 += 4) {
+      if (g0 >= nrep) break;
+      SklChunk<SKL_T, V> x[SKL_CUNR][4];
+#pragma unroll
+      for (int u = 0; u < SKL_CUNR; ++u) {
+        const skl_u64 i = i0 + (skl_u64)u * stride;
+        if (i < n_chunks) {
+#pragma unroll
+          for (int j = 0; j < 4; ++j)
+            if (g0 + j < nrep) {
+              if (V > 1) x[u][j].q[0] = skl_ld16(s.p[g0 + j] + i * V);
+              else x[u][j].e[0] = s.p[g0 + j][i];
+            }
+        }
+      }
+#pragma unroll
+      for (int u = 0; u < SKL_CUNR; ++u)
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+          if (g0 + j < nrep) {
+            if (g0 + j == 0) {
+              a[u] = x[u][0];
+            } else {
+#pragma unroll
+              for (int k = 0; k < V; ++k) a[u].e[k] = op(a[u].e[k], x[u][j].e[k]);
+            }
+          }
+    }
+#pragma unroll
+    for (int u = 0; u < SKL_CUNR; ++u) {
+      const skl_u64 i = i0 + (skl_u64)u * stride;
+      if (i >= n_chunks) break;
+      SKL_T* out = skl_combine_owner(s, nrep, i * V, chunk, inv_chunk);
+      if (V > 1) skl_st16(out + i * V, a[u].q[0]);
+      else out[i] = a[u].e[0];
+    }
+  }
+}
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+skl_combine_all(const SklSrcs s, int nrep, skl_u64 n, skl_u64 chunk, int vec) {
+#if SKL_RVEC > 1
+  if (vec) {
+    const skl_u64 nc = n / SKL_RVEC;
+    skl_combine_all_run<SKL_RVEC>(s, nrep, nc, chunk);
+    const skl_u64 t0 = nc * SKL_RVEC;
+    if (blockIdx.x == 0 && threadIdx.x < n - t0) {
+      SklOp op;
+      const skl_u64 i = t0 + threadIdx.x;
+      SKL_T a = s.p[0][i];
+#pragma unroll
+      for (int r = 1; r < SKL_CMAXR; ++r)
+        if (r < nrep) a = op(a, s.p[r][i]);
+      skl_combine_owner(s, nrep, i, chunk, 1.0f / (float)chunk)[i] = a;
+    }
+    return;
+  }
+#endif
+  (void)vec;
+  skl_combine_all_run<1>(s, nrep, n, chunk);
+}

@@ -149,6 +149,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
         defs += "#define SKL_LBW " + std::to_string(ctx->scan_lbw) + "\n";
         defs += "#define SKL_SUB " + std::to_string(s->scan_sub) + "\n";
       }
+      if (ctx->combine_unroll) defs += "#define SKL_CUNR " + std::to_string(ctx->combine_unroll) + "\n";
       body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +
              kernel_template("reduce.cuh") + (kind == K_SCAN ? kernel_template("scan.cuh") : "");
       break;
@@ -594,6 +595,54 @@ void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int n
                                                            (size_t)ctx->D(g).sm_count * 8));
   void* args[] = {(void*)&staging, &stride, &nrep, &dst, &n, &vec};
   launch(ctx, g, s->prog, "skl_combine", dim3((unsigned)grid), dim3(s->block), 0, args);
+}
+
+// copy(+) -> block fused with its exchange (reduce.cuh skl_combine_peer): srcs
+// are nrep <= 8 device pointers (this device's and its peers' replicas at the
+// slice), dst this device's replica at the slice (may equal srcs[g]).
+void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* dst, size_t nelem) {
+  if (!s || (s->kind != K_REDUCE && s->kind != K_SCAN)) fail(SKL_ERR_INVALID_ARG, "combine needs a Reduce skeleton");
+  if (nrep < 1 || nrep > 8) fail(SKL_ERR_INVALID_ARG, "run_combine_peer: 1..8 replicas");
+  Ctx* ctx = s->ctx;
+  struct {
+    const void* p[8];
+  } sp{};
+  const size_t st = ctx->type(s->tin).size;
+  int vec = 16 % st == 0 && st < 16 && aligned16(dst);
+  for (int r = 0; r < nrep; ++r) {
+    sp.p[r] = srcs[r];
+    vec = vec && aligned16(srcs[r]);
+  }
+  unsigned long long n = nelem;
+  const size_t per = vec ? 16 / st : 1;
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)s->block),
+                                                           (size_t)ctx->D(g).sm_count * 8));
+  void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec};
+  launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(s->block), 0, args);
+}
+
+// The same for logical devices sharing one GPU: one launch on device g over all
+// n elements; bases[h] = replica h at unit 0, element e goes to replica
+// e / chunk_elems.
+void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t nelem, size_t chunk_elems) {
+  if (!s || (s->kind != K_REDUCE && s->kind != K_SCAN)) fail(SKL_ERR_INVALID_ARG, "combine needs a Reduce skeleton");
+  if (nrep < 1 || nrep > 8) fail(SKL_ERR_INVALID_ARG, "run_combine_all: 1..8 replicas");
+  Ctx* ctx = s->ctx;
+  struct {
+    const void* p[8];
+  } sp{};
+  const size_t st = ctx->type(s->tin).size;
+  int vec = 16 % st == 0 && st < 16 && chunk_elems % (16 / st) == 0;
+  for (int r = 0; r < nrep; ++r) {
+    sp.p[r] = bases[r];
+    vec = vec && aligned16(bases[r]);
+  }
+  unsigned long long n = nelem, ch = chunk_elems;
+  const size_t per = vec ? 16 / st : 1;
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)s->block),
+                                                           (size_t)ctx->D(g).sm_count * 8));
+  void* args[] = {(void*)&sp, &nrep, &n, &ch, &vec};
+  launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(s->block), 0, args);
 }
 
 // Fused program: the Zip/Map's and the Reduce's customising functions in one

@@ -141,14 +141,17 @@ struct Ctx {
   int mo_ws_stages = 4;        //   shared-memory ring depth
   int mo_ws_minb = 0;          //   resident blocks per SM the registers must allow (0 = auto)
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
-  int halo_push = 1;
+  int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
   int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
+  int combine_unroll = 0;      // copy(+) -> block fold: chunks per thread and step (0 = 2)
+  int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
+                               // (0 = staged exchange then fold, 2 = one kernel per device even on one GPU)
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
   int ap_fast = 1;             // Allpairs zip-reduce: 128-row tiles (4-byte inputs, d % 4 == 0)
   int ap_tile = 0;             // Allpairs tile columns: 0 = by wave fill, 8 = 128, 4 = 64, 2 = hybrid
   int ap_bk = 0;               // Allpairs 128-row kernels: k-slice depth (0 = 16)
-  int ap_hybrid = 1;           // Allpairs: last partial wave of 128 x 128 tiles as 128 x 64 halves           // MapOverlap stores its border rows into the neighbours' halos
+  int ap_hybrid = 1;           // Allpairs: last partial wave of 128 x 128 tiles as 128 x 64 halves
   std::vector<std::vector<char>> peer_ok;  // [g][h]: device g can store to device h's memory
   // Scan schedule: 6 = one block per tile, tile kept in shared memory, low
   // register count so 5 tiles fit per SM (default, fastest measured: 5.8 TB/s
@@ -337,6 +340,8 @@ void run_allpairs(Skel* s, Cont* a, Cont* b, Cont** out);
 // ordered combine of G staged replica slices into dst (A25), on device g
 void run_combine(Skel* s, int g, const void* staging, size_t stride_elems, int nrep, void* dst,
                  size_t nelem);
+void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* dst, size_t nelem);
+void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t nelem, size_t chunk_elems);
 void* device_alloc(Ctx* ctx, int g, size_t bytes);
 void device_free(Ctx* ctx, int g, void* p);
 void check_debug_flag(Ctx* ctx);

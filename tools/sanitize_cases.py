@@ -104,6 +104,20 @@ def logical_devices(G):
         f = O.lmosem(ev[lo:hi], N, f)[1].astype(np.float32)
     assert rel(osem.image(), f) <= 1e-4
     osem.destroy()
+    # copy(+) -> block: one-launch fused fold (1), per-device fused kernels (2), staged (0)
+    addf = S.Reduce(ctx, A.ADD, S.F32)
+    idx = S.Vector.from_numpy(ctx, np.arange(5003, dtype=np.int32) % 4099).set_distribution(S.BLOCK)
+    touch = S.Map(ctx, "void touch(int i, float* c) { atomicAdd(&c[i], 1.0f); }", S.I32, S.VOID,
+                  extra=[S.F32 | S.PTR])
+    want = np.bincount(np.arange(5003) % 4099, minlength=4099).astype(np.float32)
+    for peer in (1, 2, 0):
+        ctx.set_option("combine_peer", peer)
+        cv = S.Vector(ctx, S.F32, 4099).set_distribution(S.COPY, 0, addf)
+        cv.fill(0.0)
+        touch(idx, (cv, S.WRITE))
+        cv.set_distribution(S.BLOCK)
+        assert np.array_equal(cv.to_numpy(), want)
+    ctx.set_option("combine_peer", 1)
     ctx.finalize()
 
 
