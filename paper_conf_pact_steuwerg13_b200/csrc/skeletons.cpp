@@ -752,6 +752,19 @@ void run_reduce(Skel* s, Cont* in, Cont** out) {
     // partial lands in its own slot i on its own device
     reduce_on_device(s, g, source(g, r), r.size() * in->cols, (char*)stage[g] + (size_t)i * st);
   }
+  // one process driving every device: the destination folds the partials
+  // straight out of the participants' memory (peer loads), one kernel, no copy
+  bool fused = ctx->combine_peer && !ctx->dist_mode && ctx->nlocal == ctx->G && P <= 8 && dsts.size() == 1;
+  for (int i = 0; fused && i < P; ++i) fused = ctx->peer_ok[(size_t)dsts[0]][(size_t)parts[(size_t)i]];
+  if (fused) {
+    std::vector<const void*> srcs((size_t)P);
+    for (int i = 0; i < P; ++i) srcs[(size_t)i] = (char*)stage[parts[(size_t)i]] + (size_t)i * st;
+    barrier_streams(ctx);  // every partial is written
+    run_combine_peer(s, dsts[0], srcs.data(), P, part_ptr(o, dsts[0], 0), 1);
+    barrier_streams(ctx);  // no device rewrites its partial slot while it is read
+    mark_written(o);
+    return;
+  }
   std::vector<Transfer> tr;
   for (int dg : dsts)
     for (int i = 0; i < P; ++i)
