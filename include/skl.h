@@ -141,7 +141,7 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged
  * row <= 256 units; otherwise the one-tile-per-block kernel runs),
  * and the tuning keys "scan_variant", "scan_chunks", "scan_minb", "mo_rh",
- * "mo_cw", "mo_minb", "mo_ws_minb".  Environment defaults: SKL_BLOCK_THREADS,
+ * "mo_cw", "mo_minb", "mo_ws_minb", "ap_bk", "combine_unroll".  Environment defaults: SKL_BLOCK_THREADS,
  * SKL_DEBUG_BOUNDS; SKL_CACHE_DIR keeps compiled cubins on disk.              */
 skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
 /* Counters: "launches" (kernels this library launched), "compiles" (NVRTC runs),
