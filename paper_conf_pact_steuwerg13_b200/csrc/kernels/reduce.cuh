@@ -286,14 +286,20 @@ skl_combine(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep, SKL_T* 
 // result in place into its own replica - a reduce-scatter with the user's
 // operator in one kernel, no staging copy.  In place is safe: device g writes
 // only its own slice of its own replica, which no other device reads.
+// 512-thread blocks for the peer folds, one chunk per thread and step (40
+// registers; 2 chunks measured slower: 4 replicas 22.6 vs 34.8 us,
+// tools/combine_sweep.py)
+#ifndef SKL_CBLOCK
+#define SKL_CBLOCK 512
+#endif
 struct SklSrcs {
   const SKL_T* p[SKL_CMAXR];
 };
 template <int V>
 __device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep, SKL_T* out, skl_u64 n_chunks) {
   SklOp op;
-  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i < n_chunks;
-       i += (skl_u64)gridDim.x * SKL_BLOCK) {
+  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_CBLOCK + threadIdx.x; i < n_chunks;
+       i += (skl_u64)gridDim.x * SKL_CBLOCK) {
     SklChunk<SKL_T, V> x[SKL_CMAXR];
 #pragma unroll
     for (int r = 0; r < SKL_CMAXR; ++r)
@@ -312,7 +318,7 @@ __device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep,
     else out[i] = a.e[0];
   }
 }
-extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
 skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
 #if SKL_RVEC > 1
   if (vec) {
@@ -341,7 +347,7 @@ skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
 // distribution's ceil(units / G) units in elements; a multiple of SKL_RVEC for
 // the 16-byte path).
 #ifndef SKL_CUNR
-#define SKL_CUNR 2
+#define SKL_CUNR 1
 #endif
 // SKL_CUNR chunks per thread and step: all their replica loads are issued
 // before the first store (the output aliases a replica, so the compiler cannot
@@ -367,8 +373,8 @@ template <int V>
 __device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, skl_u64 n_chunks, skl_u64 chunk) {
   SklOp op;
   const float inv_chunk = 1.0f / (float)chunk;
-  const skl_u64 stride = (skl_u64)gridDim.x * SKL_BLOCK;
-  for (skl_u64 i0 = (skl_u64)blockIdx.x * SKL_BLOCK + threadIdx.x; i0 < n_chunks; i0 += stride * SKL_CUNR) {
+  const skl_u64 stride = (skl_u64)gridDim.x * SKL_CBLOCK;
+  for (skl_u64 i0 = (skl_u64)blockIdx.x * SKL_CBLOCK + threadIdx.x; i0 < n_chunks; i0 += stride * SKL_CUNR) {
     SklChunk<SKL_T, V> a[SKL_CUNR];
     // replicas in groups of 4 (registers for 4, not SKL_CMAXR, replica chunks
     // per step), folded left to right as each group arrives
@@ -411,7 +417,7 @@ __device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, 
     }
   }
 }
-extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
+extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
 skl_combine_all(const SklSrcs s, int nrep, skl_u64 n, skl_u64 chunk, int vec) {
 #if SKL_RVEC > 1
   if (vec) {

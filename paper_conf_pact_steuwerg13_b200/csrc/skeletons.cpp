@@ -615,10 +615,10 @@ void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* d
   }
   unsigned long long n = nelem;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)s->block),
-                                                           (size_t)ctx->D(g).sm_count * 8));
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)512),
+                                                           (size_t)ctx->D(g).sm_count * 4));
   void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec};
-  launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(s->block), 0, args);
+  launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(512), 0, args);  // SKL_CBLOCK
 }
 
 // The same for logical devices sharing one GPU: one launch on device g over all
@@ -639,10 +639,10 @@ void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t 
   }
   unsigned long long n = nelem, ch = chunk_elems;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)s->block),
-                                                           (size_t)ctx->D(g).sm_count * 8));
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)512),
+                                                           (size_t)ctx->D(g).sm_count * 4));
   void* args[] = {(void*)&sp, &nrep, &n, &ch, &vec};
-  launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(s->block), 0, args);
+  launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(512), 0, args);  // SKL_CBLOCK
 }
 
 // Fused program: the Zip/Map's and the Reduce's customising functions in one

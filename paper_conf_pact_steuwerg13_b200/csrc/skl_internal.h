@@ -144,7 +144,7 @@ struct Ctx {
   int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
   int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
-  int combine_unroll = 0;      // copy(+) -> block fold: chunks per thread and step (0 = 2)
+  int combine_unroll = 0;      // copy(+) -> block fold: chunks per thread and step (0 = 1)
   int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
                                // (0 = staged exchange then fold, 2 = one kernel per device even on one GPU)
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
