@@ -20,10 +20,9 @@ _SO = os.path.join(_HERE, "liboracle.so")
 _SRC = os.path.join(_HERE, "oracle.cpp")
 
 # enums mirrored from oracle.h
-OM_NEG_F32, OM_SQP1_F32, OM_INV_U8, OM_AFFINE_I32, OM_IDENT_F32 = range(5)
-OZ_ADD_F32, OZ_MULT_F32, OZ_SUB_I32, OZ_MULT_F64 = range(4)
-(OP_ADD_F32, OP_ADD_I32, OP_MAX_F32, OP_LEFT_F32, OP_RIGHT_F32, OP_AFFINE_U32,
- OP_ADD_F64, OP_MIN_I32) = range(8)
+OM_NEG_F32, OM_SQP1_F32, OM_INV_U8, OM_AFFINE_I32 = range(4)
+OZ_ADD_F32, OZ_MULT_F32, OZ_SUB_I32 = range(3)
+OP_ADD_F32, OP_ADD_I32, OP_MAX_F32, OP_LEFT_F32, OP_RIGHT_F32, OP_AFFINE_U32 = range(6)
 OS_IDENT, OS_SHIFT_X, OS_SHIFT_Y, OS_BOX3, OS_SOBEL, OS_GAUSS5 = range(6)
 OB_NEUTRAL, OB_NEAREST = 0, 1
 
@@ -77,8 +76,7 @@ def _p(a: np.ndarray):
 
 
 _MAP_T = {OM_NEG_F32: (np.float32, np.float32), OM_SQP1_F32: (np.float32, np.float32),
-          OM_INV_U8: (np.uint8, np.uint8), OM_AFFINE_I32: (np.int32, np.int32),
-          OM_IDENT_F32: (np.float32, np.float32)}
+          OM_INV_U8: (np.uint8, np.uint8), OM_AFFINE_I32: (np.int32, np.int32)}
 
 
 def map_(fn: int, x: np.ndarray) -> np.ndarray:
@@ -104,8 +102,7 @@ def row_sums(counts: np.ndarray) -> np.ndarray:
     return s
 
 
-_ZIP_T = {OZ_ADD_F32: np.float32, OZ_MULT_F32: np.float32, OZ_SUB_I32: np.int32,
-          OZ_MULT_F64: np.float64}
+_ZIP_T = {OZ_ADD_F32: np.float32, OZ_MULT_F32: np.float32, OZ_SUB_I32: np.int32}
 
 
 def zip_(fn: int, l: np.ndarray, r: np.ndarray) -> np.ndarray:
@@ -122,8 +119,7 @@ def zip_(fn: int, l: np.ndarray, r: np.ndarray) -> np.ndarray:
 # element dtype in, result dtype out; affine pairs are uint32 [..., 2]
 _OP_T = {OP_ADD_F32: (np.float32, np.float64), OP_ADD_I32: (np.int32, np.int32),
          OP_MAX_F32: (np.float32, np.float32), OP_LEFT_F32: (np.float32, np.float32),
-         OP_RIGHT_F32: (np.float32, np.float32), OP_AFFINE_U32: (np.uint32, np.uint32),
-         OP_ADD_F64: (np.float64, np.float64), OP_MIN_I32: (np.int32, np.int32)}
+         OP_RIGHT_F32: (np.float32, np.float32), OP_AFFINE_U32: (np.uint32, np.uint32)}
 
 
 def _nelem(op, x):

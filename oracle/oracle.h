@@ -35,7 +35,6 @@ enum oracle_map_fn {
   OM_SQP1_F32 = 1,    /* x*x + 1.0f  (two roundings: pins -fmad=false)           */
   OM_INV_U8 = 2,      /* 255 - x                                               */
   OM_AFFINE_I32 = 3,  /* 3*x + 7 mod 2^32 (A28)                                */
-  OM_IDENT_F32 = 4,   /* x                                                     */
 };
 int oracle_map(int fn, const void* in, void* out, size_t n);
 
@@ -51,7 +50,6 @@ enum oracle_zip_fn {
   OZ_ADD_F32 = 0,   /* "float func(float x,float y){return x+y;}" P:L261       */
   OZ_MULT_F32 = 1,  /* "float mult(float x,float y){return x*y;}" P:L290-291   */
   OZ_SUB_I32 = 2,   /* x - y mod 2^32                                          */
-  OZ_MULT_F64 = 3,
 };
 int oracle_zip(int fn, const void* l, const void* r, void* out, size_t n);
 
@@ -64,8 +62,6 @@ enum oracle_op {
   OP_RIGHT_F32 = 4,  /* y (right projection)                                    */
   OP_AFFINE_U32 = 5, /* (a1,b1)+(a2,b2) = (a1*a2, b1*a2+b2) mod 2^32; elements are
                         uint32 pairs: composition "first map 1, then map 2"     */
-  OP_ADD_F64 = 6,    /* x+y on double                                           */
-  OP_MIN_I32 = 7,
 };
 /* Left fold acc = v[0]; acc = acc (+) v[i].  n == 0 -> returns -1 (A11).
  * out holds one element of the result type (double for OP_ADD_F32).           */

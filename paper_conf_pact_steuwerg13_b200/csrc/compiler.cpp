@@ -183,7 +183,9 @@ Program* compile(Ctx* ctx, const std::string& source, std::string* log_out) {
   return raw;
 }
 
-static cudaKernel_t get_kernel(Program* prog, const char* kernel, size_t smem) {
+// The dynamic shared-memory limit is a per-device attribute of the kernel: it is
+// raised once per (physical device, kernel), so a second GPU gets it as well.
+static cudaKernel_t get_kernel(Program* prog, int phys, const char* kernel, size_t smem) {
   auto it = prog->kernels.find(kernel);
   cudaKernel_t k;
   if (it == prog->kernels.end()) {
@@ -193,10 +195,11 @@ static cudaKernel_t get_kernel(Program* prog, const char* kernel, size_t smem) {
     k = it->second;
   }
   if (smem > 16 * 1024) {  // static + dynamic may exceed the 48 KB default: raise the limit
-    auto s = prog->smem_set.find(kernel);
+    const std::string key = std::to_string(phys) + "/" + kernel;
+    auto s = prog->smem_set.find(key);
     if (s == prog->smem_set.end() || s->second < smem) {
-      SKL_CUDA(cudaFuncSetAttribute((const void*)k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
-      prog->smem_set[kernel] = smem;
+      SKL_CUDA(cudaKernelSetAttributeForDevice(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem, phys));
+      prog->smem_set[key] = smem;
     }
   }
   return k;
@@ -204,11 +207,13 @@ static cudaKernel_t get_kernel(Program* prog, const char* kernel, size_t smem) {
 
 // Resident blocks per SM for a kernel at a block size / dynamic smem (persistent grids).
 int occupancy(Ctx* ctx, int g, Program* prog, const char* kernel, int block, size_t smem) {
-  const std::string key = std::string(kernel) + "/" + std::to_string(block) + "/" + std::to_string(smem);
+  const int phys = ctx->D(g).phys;
+  const std::string key = std::to_string(phys) + "/" + kernel + "/" + std::to_string(block) + "/" +
+                          std::to_string(smem);
   auto it = prog->occ.find(key);
   if (it != prog->occ.end()) return it->second;
   ctx->set_device(g);
-  cudaKernel_t k = get_kernel(prog, kernel, smem);
+  cudaKernel_t k = get_kernel(prog, phys, kernel, smem);
   int nb = 0;
   SKL_CUDA(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, (const void*)k, block, smem));
   prog->occ[key] = nb;
@@ -220,7 +225,7 @@ void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 
   if (grid.x == 0 || grid.y == 0 || grid.z == 0) return;
   Device& D = ctx->D(g);
   ctx->set_device(g);
-  cudaKernel_t k = get_kernel(prog, kernel, smem);
+  cudaKernel_t k = get_kernel(prog, D.phys, kernel, smem);
   SKL_CUDA(cudaLaunchKernel((const void*)k, grid, block, args, smem, D.stream));
   ctx->n_launch++;
 }

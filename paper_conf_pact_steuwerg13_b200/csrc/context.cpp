@@ -110,13 +110,27 @@ Ctx* ctx_create_local(int ndev, const int* devices) {
         fail(SKL_ERR_INVALID_ARG, "device ordinal out of range");
       init_device(c, c->dev[(size_t)g]);
     }
-    // peer access between distinct physical GPUs (NVLink / NVSwitch)
+    // peer access between distinct physical GPUs (NVLink / NVSwitch).  Two
+    // grants are needed for a kernel on GPU a to load/store GPU b's buffers:
+    // cudaDeviceEnablePeerAccess covers cudaMalloc memory (and the caller's
+    // allocator, e.g. torch's), and cudaMemPoolSetAccess gives a access to b's
+    // default stream-ordered pool, where device_alloc places every part and
+    // scratch buffer.  peer_ok[a][b] is set only when both succeed; otherwise
+    // the moves from b into a use the copy engines (cudaMemcpyPeerAsync) and the
+    // fused peer kernels (halo push, copy(+)->block fold, Reduce fold) stay off.
     c->peer_ok.assign((size_t)c->G, std::vector<char>((size_t)c->G, 0));
+    std::map<std::pair<int, int>, char> phys_ok;  // (a.phys, b.phys) -> granted
     for (auto& a : c->dev)
       for (auto& b : c->dev) {
         char& ok = c->peer_ok[(size_t)a.global][(size_t)b.global];
         if (a.phys == b.phys) {
           ok = 1;
+          continue;
+        }
+        auto key = std::make_pair(a.phys, b.phys);
+        auto it = phys_ok.find(key);
+        if (it != phys_ok.end()) {
+          ok = it->second;
           continue;
         }
         int can = 0;
@@ -125,9 +139,21 @@ Ctx* ctx_create_local(int ndev, const int* devices) {
           cudaSetDevice(a.phys);
           cudaError_t pe = cudaDeviceEnablePeerAccess(b.phys, 0);
           if (pe == cudaErrorPeerAccessAlreadyEnabled) pe = cudaSuccess;
+          if (pe == cudaSuccess) {
+            cudaMemPool_t bpool;
+            pe = cudaDeviceGetDefaultMemPool(&bpool, b.phys);
+            if (pe == cudaSuccess) {
+              cudaMemAccessDesc desc{};
+              desc.location.type = cudaMemLocationTypeDevice;
+              desc.location.id = a.phys;
+              desc.flags = cudaMemAccessFlagsProtReadWrite;
+              pe = cudaMemPoolSetAccess(bpool, &desc, 1);
+            }
+          }
           if (pe != cudaSuccess) cudaGetLastError();
           ok = pe == cudaSuccess;
         }
+        phys_ok[key] = ok;
       }
   } catch (...) {
     delete c;

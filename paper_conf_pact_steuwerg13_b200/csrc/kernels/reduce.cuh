@@ -290,7 +290,7 @@ skl_combine(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep, SKL_T* 
 // registers; 2 chunks measured slower: 4 replicas 22.6 vs 34.8 us,
 // tools/combine_sweep.py)
 #ifndef SKL_CBLOCK
-#define SKL_CBLOCK 512
+#error "SKL_CBLOCK (kCombineBlock, skl_internal.h) must be defined by the program source"
 #endif
 struct SklSrcs {
   const SKL_T* p[SKL_CMAXR];

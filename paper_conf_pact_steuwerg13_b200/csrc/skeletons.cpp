@@ -49,6 +49,7 @@ size_t ceil_div(size_t a, size_t b) { return (a + b - 1) / b; }
 std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
   std::string s;
   s += "#define SKL_BLOCK " + std::to_string(block) + "\n";
+  s += "#define SKL_CBLOCK " + std::to_string(kCombineBlock) + "\n";
   s += "#define SKL_DEBUG_BOUNDS " + std::to_string(ctx->debug_bounds ? 1 : 0) + "\n";
   s += "#define SKL_FUNC " + entry + "\n";
   return s;
@@ -615,10 +616,10 @@ void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* d
   }
   unsigned long long n = nelem;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)512),
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock),
                                                            (size_t)ctx->D(g).sm_count * 4));
   void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec};
-  launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(512), 0, args);  // SKL_CBLOCK
+  launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(kCombineBlock), 0, args);
 }
 
 // The same for logical devices sharing one GPU: one launch on device g over all
@@ -639,10 +640,10 @@ void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t 
   }
   unsigned long long n = nelem, ch = chunk_elems;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)512),
+  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock),
                                                            (size_t)ctx->D(g).sm_count * 4));
   void* args[] = {(void*)&sp, &nrep, &n, &ch, &vec};
-  launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(512), 0, args);  // SKL_CBLOCK
+  launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(kCombineBlock), 0, args);
 }
 
 // Fused program: the Zip/Map's and the Reduce's customising functions in one
@@ -754,7 +755,9 @@ void run_reduce(Skel* s, Cont* in, Cont** out) {
   }
   // one process driving every device: the destination folds the partials
   // straight out of the participants' memory (peer loads), one kernel, no copy
-  bool fused = ctx->combine_peer && !ctx->dist_mode && ctx->nlocal == ctx->G && P <= 8 && dsts.size() == 1;
+  // (the same gate as the copy(+)->block fold: xfer_kernel=0 turns every peer kernel off)
+  bool fused = ctx->combine_peer && ctx->xfer_kernel && !ctx->dist_mode && ctx->nlocal == ctx->G && P <= 8 &&
+               dsts.size() == 1;
   for (int i = 0; fused && i < P; ++i) fused = ctx->peer_ok[(size_t)dsts[0]][(size_t)parts[(size_t)i]];
   if (fused) {
     std::vector<const void*> srcs((size_t)P);

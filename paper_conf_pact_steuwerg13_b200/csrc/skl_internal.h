@@ -267,6 +267,9 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
 // one batched copy launch on device g's stream (builtin.cu); sources are on
 // g's GPU or a peer with access enabled
 constexpr int kXferMaxSegs = 32;
+// threads per block of the peer folds (skl_combine_peer / skl_combine_all); the
+// Reduce/Scan programs are compiled with SKL_CBLOCK set to this value
+constexpr int kCombineBlock = 512;
 struct XferSeg {
   const void* src;
   void* dst;

@@ -431,3 +431,52 @@ def test_lmosem_geometry_hit_rate():
     ev = I.lmosem_events(I.SEED_LMOSEM, 20000, N)
     _, _, nhit, _ = O.lmosem(ev, N, np.ones(N ** 3, np.float32))
     assert 0.60 < nhit / 20000 < 0.72
+
+
+# ------------------------------------------------------------------ pins added in round 2
+def test_row_sums_closed_forms_and_bruteforce():
+    # constant-count matrix: every row sums to cols * k (closed form); counts near
+    # 2^32 make the total overflow 32 bits, so a 32-bit accumulator fails
+    for rows, cols, k in ((1, 1, 7), (3, 5, 1000), (4, 3, 2**32 - 1)):
+        s = O.row_sums(np.full((rows, cols), k, np.uint32))
+        assert s.dtype == np.uint64 and np.array_equal(s, np.full(rows, cols * k, np.uint64))
+    # brute force (pure Python) on a random matrix, and a one-hot matrix that
+    # catches a transposed index (row r holds its only non-zero in column r)
+    c = I.uniform_int(41, 7 * 13, 0, 100000, np.uint64).astype(np.uint32).reshape(7, 13)
+    s = O.row_sums(c)
+    for r in range(7):
+        assert int(s[r]) == sum(int(v) for v in c[r])
+    eye = np.zeros((5, 9), np.uint32)
+    for r in range(5):
+        eye[r, r] = r + 1
+    assert np.array_equal(O.row_sums(eye), np.arange(1, 6, dtype=np.uint64))
+    # the Mandelbrot total equals the sum of its row sums
+    counts, tot = O.mandelbrot(I.mandel_grid(24, 32), 300)
+    assert int(O.row_sums(counts).sum()) == tot
+
+
+def test_gaussian_weights_agree_with_the_user_program():
+    # the user program (apps.gaussian5) and the oracle derive the W1
+    # weights independently; they must agree bit for bit, and the %.9g literals
+    # printed into the customising-function source must round-trip to them.
+    import re
+    from paper_conf_pact_steuwerg13_b200 import apps as A
+    w = O.gauss5_weights()
+    assert np.array_equal(A.gauss5_weights().view(np.uint32), w.view(np.uint32))
+    lits = [np.float32(float(m)) for m in re.findall(r"acc \+ ([0-9.e+-]+)f \* get", A.gaussian5())]
+    assert len(lits) == 25
+    assert np.array_equal(np.array(lits, np.float32).view(np.uint32), w.reshape(-1).view(np.uint32))
+
+
+@pytest.mark.parametrize("G", [1, 2, 3, 8])
+def test_combine_affine_is_gpu_order_fold(G):
+    # A25: replicas folded in GPU order 0..G-1 with a non-commutative operator
+    n = 50
+    p = I.uniform_int(42 + G, G * n * 2, 0, 2**32 - 1, np.uint64).astype(np.uint32).reshape(G, n, 2)
+    out = O.combine(O.OP_AFFINE_U32, p)
+    for i in (0, 17, n - 1):
+        a, b = out[i]
+        for x in (0, 3, 2**31 + 5):
+            assert (int(a) * x + int(b)) % 2**32 == _affine_apply(p[:, i], x)
+    # fp32 + accumulated in double: G ones -> G exactly
+    assert np.all(O.combine(O.OP_ADD_F32, np.ones((G, n), np.float32)) == float(G))
