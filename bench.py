@@ -1,25 +1,40 @@
 #!/usr/bin/env python
 """bench.py — the SkelCL hot path on B200 (BASELINE.json metric, contract in the
-task statement; DESIGN.md §"Measurement").
+task statement; DESIGN.md §7 "Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,sobel,gauss,gauss_iter,sobel_iter,redist,scan_i32,scan_f32,lmosem,lmosem_osem,allpairs]
+                    [--skeletons all|none|dot,dot_sweep,sobel,gauss,gauss_iter,sobel_iter,redist,
+                                 scan_i32,scan_f32,lmosem,lmosem_osem,allpairs,mandel_plain]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
 block-distributed Matrix<float2> of pixel coordinates (MAX_ITER 1000, window
 A22).  One step = one Map over the whole matrix.  value = pixels/s over all
-ranks.  The per-skeleton lines of the metric ("GB/s & elements/s per skeleton",
+GPUs.  The per-skeleton lines of the metric ("GB/s & elements/s per skeleton",
 configs[0], [2], [3], [4]) go in "skeletons".
 
+Who drives the GPUs:
+  * under torchrun (WORLD_SIZE > 1): one process per GPU (the library's SPMD
+    mode, skl_init_dist; rank r drives LOCAL_RANK's GPU); the bench's own
+    plumbing (barriers, max over ranks) is a gloo process group on the host, so
+    the only NCCL communicator in the process is the library's;
+  * without torchrun, --gpus N: one process drives N physical GPUs (skl_init with
+    N devices: the fused peer kernels over NVLink).  N larger than the visible
+    GPU count is an error, never a silent fallback to logical devices.
+n_gpus in the line is the library's device count (skl_num_devices).
+
 Timing: W untimed warm-up steps; K timed steps, each bracketed by CUDA events on
-the stream the library launches on (torch's current stream, handed to the
-library with skl_set_stream), with a 256 MiB L2 flush (write) before every step
-outside the events; barrier + synchronize around the timed region; max over
-ranks.  nvidia-smi clocks are sampled during the timed region.
+the stream the library launches on (a torch stream per device handed to the
+library with skl_set_stream; with several devices in one process every other
+device's stream joins the first one's start and end events, so a step spans all
+GPUs), with an L2 flush (256 MiB write + 256 MiB read on every GPU) before every
+step outside the events; barrier + synchronize around the timed region; the
+median over steps (mean and min reported too); max over ranks.  nvidia-smi
+clocks are sampled during the timed region.  Exit status is non-zero when a
+parity check fails or a section raises or times out (the line is printed first).
 
 --impl reference: the CPU oracle (oracle/, plain single-threaded C++) timed on
 this host on a bounded sample of the same workload (the paper's method has no
-reference code to install: DESIGN.md §"Reference arm").
+reference code to install: DESIGN.md §7 "Reference arm").
 """
 from __future__ import annotations
 
@@ -62,8 +77,8 @@ REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_c
 
 
 class ClockSampler:
-    def __init__(self, index: int):
-        self.index = index
+    def __init__(self, indices):
+        self.indices = list(indices)
         self.samples = []
         self._p = None
         self._t = None
@@ -71,7 +86,7 @@ class ClockSampler:
     def start(self):
         try:
             self._p = subprocess.Popen(
-                ["nvidia-smi", "-i", str(self.index),
+                ["nvidia-smi", "-i", ",".join(str(i) for i in self.indices),
                  "--query-gpu=clocks.sm,clocks.max.sm,clocks_event_reasons.active", "--format=csv,noheader,nounits",
                  "-lms", "100"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
         except Exception:
@@ -108,32 +123,49 @@ class ClockSampler:
                 "reasons": [v for k, v in REASONS.items() if mask & k and k != 0x1], "samples": len(self.samples)}
 
 
-# ---------------------------------------------------------------- distributed plumbing
-class Dist:
+# ---------------------------------------------------------------- who drives which GPU
+class Env:
+    """Process layout.  spmd: one process per GPU (torchrun); else one process
+    driving `G` physical GPUs.  `local` = [(global device g, CUDA ordinal)]."""
+
     def __init__(self, gpus: int):
+        import torch
         self.world = int(os.environ.get("WORLD_SIZE", "1"))
         self.rank = int(os.environ.get("RANK", "0"))
-        self.local = int(os.environ.get("LOCAL_RANK", "0"))
+        local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+        # SKL_BENCH_FORCE_DIST=1: the one-process-per-GPU path (collective host
+        # reads, max over ranks) even at world size 1, to exercise it on one GPU
+        force = os.environ.get("SKL_BENCH_FORCE_DIST", "0") == "1"
+        self.spmd = self.world > 1 or force
         self.pg = None
-        # SKL_BENCH_FORCE_DIST=1: the one-process-per-GPU path (NCCL communicator,
-        # collective host reads, max over ranks) even at world size 1, so that it
-        # can be exercised on a single GPU
-        self.force = os.environ.get("SKL_BENCH_FORCE_DIST", "0") == "1"
-        # SKL_COMM=shm (several ranks on one GPU, testing only): the library's
-        # shared-memory transport and a gloo process group for the bench plumbing
-        self.gloo = os.environ.get("SKL_COMM", "") == "shm"
-        if self.gloo:
-            import torch
-            self.local %= max(1, torch.cuda.device_count())   # ranks may share a GPU
-        if self.world > 1 or self.force:
-            import torch
+        nvis = torch.cuda.device_count()
+        if self.spmd:
+            if gpus not in (1, self.world):
+                raise SystemExit(f"--gpus {gpus} does not match WORLD_SIZE {self.world}")
+            # SKL_COMM=shm (tests): several ranks may share one GPU
+            phys = local_rank % max(1, nvis) if os.environ.get("SKL_COMM", "") == "shm" else local_rank
+            if phys >= nvis:
+                raise SystemExit(f"LOCAL_RANK {local_rank} but only {nvis} visible GPU(s)")
+            self.G = self.world
+            self.local = [(self.rank, phys)]
             import torch.distributed as dist
-            torch.cuda.set_device(self.local)
-            if self.gloo:
-                dist.init_process_group("gloo")
-            else:
-                dist.init_process_group("nccl", device_id=torch.device("cuda", self.local))
+            torch.cuda.set_device(phys)
+            # bench plumbing (barriers, max/sum of host floats) on gloo: the data
+            # path's NCCL communicator is the library's own (one per process)
+            dist.init_process_group("gloo")
             self.pg = dist
+        else:
+            if gpus > nvis:
+                raise SystemExit(f"--gpus {gpus} but only {nvis} visible GPU(s)")
+            self.G = gpus
+            self.local = [(g, g) for g in range(gpus)]
+            torch.cuda.set_device(0)
+        self.phys = [p for _, p in self.local]
+
+    @property
+    def mode(self):
+        return "one process per GPU (torchrun, skl_init_dist)" if self.spmd else \
+            f"one process driving {self.G} GPU(s) (skl_init)"
 
     def barrier(self):
         if self.pg:
@@ -143,17 +175,23 @@ class Dist:
         if not self.pg:
             return v
         import torch
-        t = torch.tensor([v], dtype=torch.float64, device="cpu" if self.gloo else "cuda")
+        t = torch.tensor([v], dtype=torch.float64)
         self.pg.all_reduce(t, op=self.pg.ReduceOp.MAX)
         return float(t.item())
+
+    def min(self, v: float) -> float:
+        return -self.max(-v)
 
     def sum(self, v: float) -> float:
         if not self.pg:
             return v
         import torch
-        t = torch.tensor([v], dtype=torch.float64, device="cpu" if self.gloo else "cuda")
+        t = torch.tensor([v], dtype=torch.float64)
         self.pg.all_reduce(t)
         return float(t.item())
+
+    def all_ok(self, ok: bool) -> bool:
+        return self.min(1.0 if ok else 0.0) > 0.5
 
     def bcast_bytes(self, b: bytes) -> bytes:
         if not self.pg:
@@ -163,74 +201,129 @@ class Dist:
         return obj[0]
 
 
-def make_context(D: Dist):
+def make_context(E: Env, logical: int = 0):
+    """The library context for this process, launching on one torch stream per
+    local device (made current on that device).  logical > 0: that many logical
+    devices on the first local GPU (one process, one GPU: the redistribution
+    lines when only one GPU is available)."""
     import torch
     from paper_conf_pact_steuwerg13_b200 import skl as S
-    torch.cuda.set_device(D.local)
-    if D.world > 1 or D.force:
-        nid = S.Context.nccl_unique_id() if D.rank == 0 else b"\0" * 128
-        nid = D.bcast_bytes(nid)
-        ctx = S.Context.dist(D.rank, D.world, D.local, nid)
-        g = D.rank
+    if logical:
+        ctx = S.Context(logical, devices=[E.phys[0]] * logical)
+        local = [(g, E.phys[0]) for g in range(logical)]
+    elif E.spmd:
+        nid = S.Context.nccl_unique_id() if E.rank == 0 else b"\0" * 128
+        nid = E.bcast_bytes(nid)
+        ctx = S.Context.dist(E.rank, E.world, E.phys[0], nid)
+        local = E.local
     else:
-        ctx = S.Context(1, devices=[D.local])
-        g = 0
-    # the library launches on torch's current stream (a dedicated non-default
-    # stream, made current here): torch.cuda.Event timing then sees its kernels
-    s = torch.cuda.Stream(device=D.local)
-    torch.cuda.set_stream(s)
-    ctx.set_stream(g, s.cuda_stream)
-    assert ctx.stream(g) == s.cuda_stream != 0
-    return ctx, g
+        ctx = S.Context(E.G, devices=E.phys)
+        local = E.local
+    streams = {}
+    for g, phys in local:
+        if phys not in streams:
+            streams[phys] = torch.cuda.Stream(device=phys)
+            torch.cuda.set_stream(streams[phys])
+        ctx.set_stream(g, streams[phys].cuda_stream)
+        assert ctx.stream(g) == streams[phys].cuda_stream != 0
+    torch.cuda.set_device(local[0][1])
+    ctx._bench_local = local
+    ctx._bench_streams = [streams[p] for p in sorted(streams)]
+    return ctx
+
+
+class Mark:
+    """a segment boundary inside a step: every stream joins the first, then an
+    event is recorded there"""
+
+    def __init__(self, streams):
+        import torch
+        self.streams = streams
+        self.ev = torch.cuda.Event(enable_timing=True)
+
+    def record(self):
+        import torch
+        first = self.streams[0]
+        for s in self.streams[1:]:
+            e = torch.cuda.Event()
+            e.record(s)
+            first.wait_event(e)
+        self.ev.record(first)
+
+
+def stats(xs):
+    xs = [float(x) for x in xs]
+    return {"median": float(np.median(xs)), "mean": float(np.mean(xs)), "min": float(np.min(xs)), "n": len(xs)}
 
 
 class Timer:
-    """per-step CUDA-event timing with an L2 flush before each step (outside the
-    events) and a host-ahead pre-roll before the first"""
+    """per-step CUDA-event timing over every stream of a context, with an L2
+    flush on every GPU before each step (outside the events) and a host-ahead
+    pre-roll before the first"""
 
-    def __init__(self):
+    def __init__(self, ctx, E: Env):
         import torch
         self.torch = torch
-        self.flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")  # 256 MiB > 126 MB L2
-        self.sweep = torch.zeros(64 << 20, dtype=torch.float32, device="cuda")
-        self.sink = torch.zeros((), dtype=torch.float32, device="cuda")
+        self.E = E
+        self.streams = ctx._bench_streams
+        self.bufs = []
+        for s in self.streams:
+            d = s.device
+            self.bufs.append((s, torch.empty(64 << 20, dtype=torch.float32, device=d),
+                              torch.zeros(64 << 20, dtype=torch.float32, device=d),
+                              torch.zeros((), dtype=torch.float32, device=d)))
 
     def flush_l2(self):
         """write 256 MiB (evicts the working set), then read another 256 MiB so
         that L2 holds clean lines: the timed step starts cold, without paying
         for the write-back of the flush's dirty lines"""
-        self.flush.zero_()
-        self.sink.copy_(self.sweep.sum())
-
-    def run(self, step, K: int, W: int, D: Dist, marks: int = 0, flush: bool = True):
         torch = self.torch
+        for s, flush, sweep, sink in self.bufs:
+            with torch.cuda.stream(s):
+                flush.zero_()
+                sink.copy_(sweep.sum())
+
+    def run(self, step, K: int, W: int, marks: int = 0, flush: bool = True):
+        """returns (stats of the step times in ms, [median of each segment])"""
+        torch = self.torch
+        E = self.E
+        first, others = self.streams[0], self.streams[1:]
         for _ in range(W):
             step(None)
         torch.cuda.synchronize()
-        D.barrier()
-        torch.cuda.synchronize()
-        # host-ahead pre-roll: a spin kernel (~0.2 ms per timed step, outside the
+        for s in others:
+            torch.cuda.synchronize(s.device)
+        E.barrier()
+        # host-ahead pre-roll: a spin kernel (~0.4 ms per timed step, outside the
         # events) keeps the GPU busy while the host enqueues the timed steps, so
         # the events bracket device execution and not host submission gaps
         # (latency-bound steps such as the 2^20 dot product are shorter than their
         # host enqueue time).  Steps that synchronise with the host (e2e) are
         # unaffected: their first event is recorded after the spin.
-        torch.cuda._sleep(int(min(K, 100) * 4e5))
+        with torch.cuda.stream(first):
+            torch.cuda._sleep(int(min(K, 100) * 4e5))
         evs = []
         for _ in range(K):
             if flush:
                 self.flush_l2()
-            e = [torch.cuda.Event(enable_timing=True) for _ in range(2 + marks)]
-            e[0].record()
-            step(e[1:-1] if marks else None)
-            e[-1].record()
-            evs.append(e)
-        torch.cuda.synchronize()
-        D.barrier()
-        torch.cuda.synchronize()
+            e0 = torch.cuda.Event(enable_timing=True)
+            e0.record(first)
+            for s in others:
+                s.wait_event(e0)
+            ms = [Mark(self.streams) for _ in range(marks)]
+            step(ms if marks else None)
+            end = Mark(self.streams)
+            end.record()
+            evs.append([e0] + [m.ev for m in ms] + [end.ev])
+        for s in self.streams:
+            torch.cuda.synchronize(s.device)
+        E.barrier()
         step_ms = [e[0].elapsed_time(e[-1]) for e in evs]
-        seg_ms = [[e[i].elapsed_time(e[i + 1]) for i in range(len(e) - 1)] for e in evs]
-        return float(np.mean(step_ms)), [float(np.mean([s[i] for s in seg_ms])) for i in range(len(seg_ms[0]))]
+        seg = [[e[i].elapsed_time(e[i + 1]) for i in range(len(e) - 1)] for e in evs]
+        st = stats(step_ms)
+        # max over ranks (the slowest GPU sets the step)
+        st = {k: (E.max(v) if k != "n" else v) for k, v in st.items()}
+        return st, [E.max(float(np.median([s[i] for s in seg]))) for i in range(len(seg[0]))]
 
 
 # ---------------------------------------------------------------- headline: Mandelbrot
@@ -244,12 +337,12 @@ def row_order(rows: int, G: int) -> np.ndarray:
     return np.concatenate([np.arange(g, rows, G) for g in range(G)])
 
 
-def bench_mandelbrot(args, D: Dist, P: dict):
-    import torch
+def mandel_map(ctx, plain: bool = False):
     from paper_conf_pact_steuwerg13_b200 import apps as A
-    from paper_conf_pact_steuwerg13_b200 import inputs as I
     from paper_conf_pact_steuwerg13_b200 import skl as S
-    ctx, g = make_context(D)
+    if plain:
+        # the A22 loop as written (apps.mandelbrot), default Map configuration
+        return S.Map(ctx, A.mandelbrot(MAX_ITER), S.F32X2, S.U32)
     # user-side tuning (the paper's optional work-group size):
     # 1024-thread blocks, one 4-pixel chunk per thread, warp-interleaved pixels
     # (lanes of a warp iterate neighbouring pixels: less idle-lane time); the
@@ -264,49 +357,63 @@ def bench_mandelbrot(args, D: Dist, P: dict):
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
     ctx.set_option("map_interleave", 0)
-    order = row_order(ROWS, D.world)
+    return m
+
+
+def bench_mandelbrot(args, E: Env, P: dict):
+    import torch
+    from paper_conf_pact_steuwerg13_b200 import inputs as I
+    from paper_conf_pact_steuwerg13_b200 import skl as S
+    ctx = make_context(E)
+    m = mandel_map(ctx)
+    order = row_order(ROWS, E.G)
     grid = np.ascontiguousarray(I.mandel_grid(ROWS, COLS)[order])
     cin = S.Matrix(ctx, S.F32X2, ROWS, COLS).set_distribution(S.BLOCK)
     cin.copy_in(grid)
     out = S.Matrix(ctx, S.U32, ROWS, COLS)
-    timer = Timer()
+    timer = Timer(ctx, E)
     l0 = ctx.counter("launches")
 
     def step(_):
         m(cin, out=out)
 
-    clk = ClockSampler(D.local)
+    clk = ClockSampler(E.phys)
     clk.start()
-    ms, _ = timer.run(step, args.steps, args.warmup, D)
+    st, _ = timer.run(step, args.steps, args.warmup)
     clocks = clk.stop()
     launches = (ctx.counter("launches") - l0) // (args.steps + args.warmup)
-    ms = D.max(ms)
     counts = np.empty((ROWS, COLS), np.uint32)
     counts[order] = out.to_numpy().reshape(ROWS, COLS)   # whole result (collective), image row order
+    ms = st["median"]
     value = ROWS * COLS / (ms / 1e3)
 
-    # e2e through the public API: pinned host input -> copy_in -> Map -> copy_out (per rank: own block)
+    # e2e through the public API: pinned host input -> copy_in -> Map -> copy_out of
+    # every local device's block, every step
     pin_in = torch.empty(grid.nbytes, dtype=torch.uint8, pin_memory=True)
     pin_in.numpy()[:] = grid.view(np.uint8).ravel()
-    lo, hi = S.plan_range(ROWS, D.world, S.BLOCK, 0, g, False)
-    pin_out = torch.empty(max(1, (hi - lo) * COLS * 4), dtype=torch.uint8, pin_memory=True)
+    outs = []
+    for g, _ in E.local:
+        lo, hi = S.plan_range(ROWS, E.G, S.BLOCK, 0, g, False)
+        outs.append((g, lo, hi, torch.empty(max(1, (hi - lo) * COLS * 4), dtype=torch.uint8, pin_memory=True)))
     e_in = S.Matrix(ctx, S.F32X2, ROWS, COLS).set_distribution(S.BLOCK)
     e_out = S.Matrix(ctx, S.U32, ROWS, COLS)
 
     def e2e_step(_):
         e_in.copy_in_ptr(pin_in.data_ptr(), grid.nbytes)
         m(e_in, out=e_out)
-        from ctypes import c_void_p  # noqa
-        e_out.copy_out_part(g, pin_out.numpy())
+        for g, _, _, po in outs:
+            e_out.copy_out_part(g, po.numpy())
 
-    e2e_ms, _ = timer.run(e2e_step, max(3, args.steps // 3), 2, D)
-    e2e_ms = D.max(e2e_ms)
-    h2d = D.sum((hi - lo) * COLS * 8)
-    d2h = D.sum((hi - lo) * COLS * 4)
+    e2e, _ = timer.run(e2e_step, max(3, args.steps // 3), 2)
+    # SPMD: every rank uploads the whole input (host mirror semantics) but only its
+    # block is moved to its GPU; count the bytes that crossed PCIe
+    h2d = E.sum(sum((hi - lo) * COLS * 8 for _, lo, hi, _ in outs))
+    d2h = E.sum(sum((hi - lo) * COLS * 4 for _, lo, hi, _ in outs))
+    ndev = ctx.ndev
     ctx.finalize()
-    return dict(ms=ms, value=value, counts=counts, clocks=clocks, launches=launches,
-                e2e={"value": ROWS * COLS / (e2e_ms / 1e3), "unit": "elements/s", "ms_per_step": e2e_ms,
-                     "h2d_bytes_per_step": int(h2d), "d2h_bytes_per_step": int(d2h)})
+    return dict(st=st, value=value, counts=counts, clocks=clocks, launches=launches, ndev=ndev,
+                e2e={"value": ROWS * COLS / (e2e["median"] / 1e3), "unit": "elements/s", "ms_per_step": e2e["median"],
+                     "ms_min": e2e["min"], "h2d_bytes_per_step": int(h2d), "d2h_bytes_per_step": int(d2h)})
 
 
 def cpu_info() -> dict:
@@ -322,43 +429,46 @@ def cpu_info() -> dict:
     return {"cpu_model": model, "nproc": os.cpu_count()}
 
 
+class OneCore:
+    """pin this thread to one core (SURVEY 8(d) oracle timing), restored after"""
+
+    def __enter__(self):
+        self.allowed = os.sched_getaffinity(0) if hasattr(os, "sched_getaffinity") else None
+        if self.allowed:
+            os.sched_setaffinity(0, {min(self.allowed)})
+        return self
+
+    def __exit__(self, *a):
+        if self.allowed:
+            os.sched_setaffinity(0, self.allowed)
+
+
 def mandel_oracle(sample_every: int = 1):
     """CPU oracle on rows 0, s, 2s, ... (bounded sample); returns counts, sum iters, seconds"""
     import oracle as O
     from paper_conf_pact_steuwerg13_b200 import inputs as I
     grid = I.mandel_grid(ROWS, COLS)[::sample_every].copy()
-    # one thread pinned to one core (SURVEY 8(d)), the affinity restored afterwards
-    allowed = os.sched_getaffinity(0) if hasattr(os, "sched_getaffinity") else None
-    if allowed:
-        os.sched_setaffinity(0, {min(allowed)})
-    try:
+    with OneCore():
         t0 = time.perf_counter()
         counts, tot = O.mandelbrot(grid, MAX_ITER)
         sec = time.perf_counter() - t0
-    finally:
-        if allowed:
-            os.sched_setaffinity(0, allowed)
     return counts, tot, sec
 
 
 # ---------------------------------------------------------------- per-skeleton lines
-def ncu_traffic(workload: str):
-    """DRAM bytes per launch (dram__bytes_read.sum + dram__bytes_write.sum) of the
-    workload's dominant kernel from the committed ncu --set full summary
-    (profiles/ncu_traffic.json, written by tools/ncu_traffic.py), else None."""
-    f = os.path.join(ROOT, "profiles", "ncu_traffic.json")
-    try:
-        return float(json.load(open(f))[workload]["bytes_per_launch"])
-    except Exception:
-        return None
-
-
 def ncu_field(workload: str, key: str):
     f = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     try:
         return float(json.load(open(f))[workload][key])
     except Exception:
         return None
+
+
+def ncu_traffic(workload: str):
+    """DRAM bytes per launch (dram__bytes_read.sum + dram__bytes_write.sum) of the
+    workload's dominant kernel from the committed ncu --set full summary
+    (profiles/ncu_traffic.json, written by tools/ncu_traffic.py), else None."""
+    return ncu_field(workload, "bytes_per_launch")
 
 
 def roof_issue(workload: str, ms: float, P: dict, sms: int):
@@ -375,12 +485,22 @@ def roof_issue(workload: str, ms: float, P: dict, sms: int):
             "threads_per_inst": ncu_field(workload, "threads_per_inst")}
 
 
-def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None):
+def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None, ngpu: int = 1):
+    """algorithmic bytes / device time against the measured copy bandwidth of
+    `ngpu` GPUs"""
     gbs = bytes_per_step / (ms / 1e3) / 1e9
-    return {"bound": "hbm", "achieved": round(gbs, 1), "peak": P["hbm_gbs"], "unit": "GB/s",
-            "frac": round(gbs / P["hbm_gbs"], 4), "frac_of_nominal_8TBs": round(gbs / 8000.0, 4),
+    peak = P["hbm_gbs"] * ngpu
+    return {"bound": "hbm", "achieved": round(gbs, 1), "peak": peak, "unit": "GB/s",
+            "frac": round(gbs / peak, 4), "frac_of_nominal_8TBs": round(gbs / (8000.0 * ngpu), 4),
             "peak_source": P["source"], "traffic": ncu_traffic(workload) if workload else None,
             "algorithmic_bytes": bytes_per_step}
+
+
+def roof_alu(ops: float, ms: float, P: dict, sms: int, ngpu: int = 1, note: str = ""):
+    peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6 * ngpu
+    fl = ops / (ms / 1e3)
+    return {"bound": "alu", "achieved": fl / 1e12, "peak": peak / 1e12, "unit": "TFLOP/s", "frac": fl / peak,
+            "note": note}
 
 
 def roof_l2(workload: str):
@@ -397,24 +517,30 @@ def roof_l2(workload: str):
             "committed capture (profiles/ncu_traffic.json)", "traffic": ncu_traffic(workload)}
 
 
-def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
-    """SURVEY 8(a) rows a9 (halo refresh) and a10 (redistribution) on ONE physical
-    GPU: a context of G = 4 logical devices (one process, separate memory per
-    device, all on the bench's stream), so every transfer is an on-GPU
+def ms_fields(st: dict) -> dict:
+    return {"ms": round(st["median"], 4), "ms_min": round(st["min"], 4), "ms_mean": round(st["mean"], 4),
+            "timed_steps": st["n"], "statistic": "median"}
+
+
+def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
+    """SURVEY 8(a) rows a9 (halo refresh) and a10 (redistribution).  With N > 1
+    GPUs in this process: the N physical devices (peer loads/stores over NVLink).
+    With one GPU: a context of 4 logical devices on it (one process, separate
+    memory per device, all on the bench's stream), so every transfer is an on-GPU
     device-to-device copy (HBM read + write) instead of an NVLink transfer.  The
     roofline counts 2 x the bytes moved (read + write) plus the combine kernel's
     traffic against the measured HBM copy bandwidth."""
-    import torch
     from paper_conf_pact_steuwerg13_b200 import apps as A
     from paper_conf_pact_steuwerg13_b200 import inputs as I
     from paper_conf_pact_steuwerg13_b200 import skl as S
     import oracle as O
-    G, N = 4, 150
+    physical = E.G > 1
+    c4 = make_context(E) if physical else make_context(E, logical=4)
+    G = c4.ndev
+    where = f"{G} physical GPUs (NVLink)" if physical else f"{G} logical devices on one GPU"
+    timer = Timer(c4, E)
+    N = 150
     nvox = N ** 3
-    c4 = S.Context(G, devices=[D.local] * G)
-    st = torch.cuda.current_stream()
-    for gg in range(G):
-        c4.set_stream(gg, st.cuda_stream)
     out = {}
     img = I.uniform_f32(I.SEED_DOT_A, nvox)
 
@@ -436,14 +562,14 @@ def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
         v.set_distribution(S.BLOCK)
 
     p0 = c4.counter("p2p_bytes")
-    ms, seg = timer.run(step_bc, K, W, D, marks=2)
+    st, seg = timer.run(step_bc, K, W, marks=2)
     moved = (c4.counter("p2p_bytes") - p0) / (K + W)
     v.set_distribution(S.COPY)
     ok = bool(np.array_equal(v.to_numpy(), img)) and moved >= (G - 1) * nvox * 4
     out["redist_block_to_copy"] = {
-        "workload": f"block -> copy of a 150^3 fp32 Vector (13.5 MB), {G} logical devices on one GPU",
+        "workload": f"block -> copy of a 150^3 fp32 Vector (13.5 MB), {where}",
         "ms": round(seg[1], 4), "bytes_moved": moved,
-        "roofline": roof_hbm(2 * moved, seg[1], P), "check": "ok" if ok else "FAIL"}
+        "roofline": roof_hbm(2 * moved, seg[1], P, ngpu=G if physical else 1), "check": "ok" if ok else "FAIL"}
 
     # a10: copy(+) -> block (LM OSEM's c): every device scatters into its own
     # zeroed replica (a void Map with a WRITE extra argument, as the LM OSEM
@@ -464,23 +590,23 @@ def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
     # default: the exchange fused into the fold (combine_peer: each device folds
     # its slice straight out of every replica, in place); then the staged path
     # (slices copied into staging, then folded) for comparison
-    ms, seg = timer.run(step_cb, K, W, D, marks=1)
+    st, seg = timer.run(step_cb, K, W, marks=1)
     ok = bool(np.all(cv.to_numpy() == 1.0))
     c4.set_option("combine_peer", 0)
     p0 = c4.counter("p2p_bytes")
-    _, seg0 = timer.run(step_cb, K, W, D, marks=1)
+    _, seg0 = timer.run(step_cb, K, W, marks=1)
     moved = (c4.counter("p2p_bytes") - p0) / (K + W)
     ok = ok and bool(np.all(cv.to_numpy() == 1.0))
     c4.set_option("combine_peer", 1)
     traffic = (G + 1) * nvox * 4                   # fused: G replica slices in, 1 folded slice out
     out["redist_copy_add_to_block"] = {
-        "workload": f"copy(+) -> block of a 150^3 fp32 Vector, {G} logical devices on one GPU "
+        "workload": f"copy(+) -> block of a 150^3 fp32 Vector, {where} "
                     "(exchange fused into the device-order fold: every slice read straight from the replicas)",
         "ms": round(seg[1], 4), "algorithmic_bytes": traffic,
-        "roofline": roof_hbm(traffic, seg[1], P),
+        "roofline": roof_hbm(traffic, seg[1], P, ngpu=G if physical else 1),
         "staged": {"ms": round(seg0[1], 4), "bytes_moved": moved,
                    "note": "slices exchanged into staging, then folded (combine_peer=0)",
-                   "roofline": roof_hbm(2 * moved + traffic, seg0[1], P)},
+                   "roofline": roof_hbm(2 * moved + traffic, seg0[1], P, ngpu=G if physical else 1)},
         "check": "ok" if ok else "FAIL"}
     for x in (w, v, cv, idx):
         x.destroy()
@@ -504,17 +630,21 @@ def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
         b.set_distribution(S.OVERLAP, 2)
 
     p0 = c4.counter("p2p_bytes")
-    ms, seg = timer.run(step_halo, K, W, D, marks=1)
+    st, seg = timer.run(step_halo, K, W, marks=1)
     moved = (c4.counter("p2p_bytes") - p0) / (K + W)
     out["halo_refresh"] = {
-        "workload": f"overlap(2) halo refresh of an 8192^2 fp32 Matrix after a stencil, {G} logical devices "
-                    f"on one GPU ({2 * (G - 1)} transfers of 2 rows)",
+        "workload": f"overlap(2) halo refresh of an 8192^2 fp32 Matrix after a stencil, {where} "
+                    f"({2 * (G - 1)} transfers of 2 rows)",
         "ms": round(seg[1], 4), "bytes_moved": moved, "latency_bound": True}
     ITER = 10
-    sub = im[3970:4094]
+    # parity band across the device boundary nearest the middle
+    b0 = (R + G - 1) // G * (G // 2)
+    lo = max(0, b0 - 64)
+    sub = im[lo:b0 + 64 + 30]
     ref = sub
     for _ in range(ITER):
         ref = O.mapoverlap2d(O.OS_GAUSS5, ref, 2, O.OB_NEAREST, 0.0)
+    chk = slice(30, b0 - lo + 64) if lo > 0 else slice(0, b0 + 64)
     for push in (0, 1):
         c4.set_option("halo_push", push)
 
@@ -524,15 +654,16 @@ def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
                 gau(b, out=t) if k % 2 == 0 else gau(t, out=b)
 
         p0, h0 = c4.counter("p2p_bytes"), c4.counter("halo_push_bytes")
-        ms, _ = timer.run(step_it, max(3, K // 4), W, D)
-        reps = max(3, K // 4) + W
+        Ki = max(3, K // 4)
+        st, _ = timer.run(step_it, Ki, W)
+        reps = Ki + W
         fin = t if (ITER - 1) % 2 == 1 else b
-        ok = bool(np.array_equal(fin.to_numpy()[4000:4064], ref[30:94]))
+        ok = bool(np.array_equal(fin.to_numpy()[lo:lo + len(sub)][chk], ref[chk]))
         out[f"gauss_iter10_g{G}_{'push' if push else 'refresh'}"] = {
-            "workload": f"10 x Gaussian 5x5 on {G} logical devices of one GPU, halos "
+            "workload": f"10 x Gaussian 5x5 on {where}, halos "
                         + ("pushed by the stencil kernel into the neighbours (fused)" if push
                            else "refreshed by copies between iterations"),
-            "ms": round(ms, 4), "p2p_bytes_per_step": (c4.counter("p2p_bytes") - p0) / reps,
+            **ms_fields(st), "p2p_bytes_per_step": (c4.counter("p2p_bytes") - p0) / reps,
             "halo_push_bytes_per_step": (c4.counter("halo_push_bytes") - h0) / reps,
             "check": "ok" if ok else "FAIL"}
     for x in (a, b, t):
@@ -541,16 +672,51 @@ def bench_redist(ctx1, timer, K: int, W: int, D: Dist, P: dict) -> dict:
     return out
 
 
-def bench_skeletons(args, D: Dist, P: dict, which):
+def _part_tensor(cont, g, phys, typestr):
+    """torch view of device g's part of a container on CUDA device `phys`
+    (plumbing for the 4 GiB Scan vectors, which are generated on the device)"""
+    import torch
+    ptr, first, cnt = cont.local_part(g)
+
+    class View:
+        __cuda_array_interface__ = {"shape": (cnt,), "typestr": typestr, "data": (ptr, False), "version": 3,
+                                    "strides": None}
+    with torch.cuda.device(phys):
+        return torch.as_tensor(View(), device=f"cuda:{phys}"), first, cnt
+
+
+def bench_skeletons(args, E: Env, P: dict, which):
     import torch
     from paper_conf_pact_steuwerg13_b200 import apps as A
     from paper_conf_pact_steuwerg13_b200 import inputs as I
     from paper_conf_pact_steuwerg13_b200 import skl as S
     import oracle as O
-    ctx, g = make_context(D)
-    timer = Timer()
+    ctx = make_context(E)
+    timer = Timer(ctx, E)
     res = {}
-    K, W = max(3, args.steps // 2), max(3, args.warmup)
+    K, W = max(20, args.steps), max(3, args.warmup)
+    G = ctx.ndev
+    one_dev = len(ctx._bench_local) == 1
+    sms = torch.cuda.get_device_properties(E.phys[0]).multi_processor_count
+
+    if "mandel_plain" in which:
+        # the paper-form A22 loop (apps.mandelbrot) with the library's default Map
+        # configuration, next to the tuned headline (VERDICT r1: both measured)
+        m = mandel_map(ctx, plain=True)
+        order = row_order(ROWS, G)
+        grid = np.ascontiguousarray(I.mandel_grid(ROWS, COLS)[order])
+        cin = S.Matrix(ctx, S.F32X2, ROWS, COLS).set_distribution(S.BLOCK)
+        cin.copy_in(grid)
+        o = S.Matrix(ctx, S.U32, ROWS, COLS)
+        st, _ = timer.run(lambda _: m(cin, out=o), K, W)
+        counts = np.empty((ROWS, COLS), np.uint32)
+        counts[order] = o.to_numpy().reshape(ROWS, COLS)
+        res["mandel_plain"] = {"workload": "Mandelbrot 4096x3072 MAX 1000, the plain A22 loop (apps.mandelbrot: "
+                                           "escape test every iteration), default Map (256 threads, 4 chunks)",
+                               **ms_fields(st), "elements_per_s": ROWS * COLS / (st["median"] / 1e3),
+                               "_counts": counts}
+        for x in (cin, o):
+            x.destroy()
 
     if "dot" in which:
         for n in (1 << 20, 1 << 28):
@@ -565,18 +731,28 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                 # fused into the Reduce (one kernel, 8 B per element)
                 sm(mult(va, vb), out=s)
 
-            ms_eager, _ = timer.run(step, K, W, D)
-            ms_eager = D.max(ms_eager)
-            ms_warm = None
+            st_eager, _ = timer.run(step, K, W)
+            st_warm = None
+            floor = None
             # the same step recorded once as a CUDA graph and replayed (removes the
             # host enqueue time that dominates at 2^20 elements)
-            graph = ctx.capture(lambda: step(None)) if D.world == 1 else None
+            graph = ctx.capture(lambda: step(None)) if one_dev else None
             if graph is not None:
-                ms, _ = timer.run(lambda _: graph.launch(), K, W, D)
+                st, _ = timer.run(lambda _: graph.launch(), K, W)
                 if n == 1 << 20:   # 8 MiB fits L2: also the warm number (no flush)
-                    ms_warm, _ = timer.run(lambda _: graph.launch(), K, W, D, flush=False)
+                    st_warm, _ = timer.run(lambda _: graph.launch(), K, W, flush=False)
+                    # the floor of this step in the same run: a graph of ONE
+                    # one-element fill kernel between the same events
+                    tiny = S.Vector(ctx, S.F32, 1).set_distribution(S.BLOCK)
+                    gf = ctx.capture(lambda: tiny.fill(0.0))
+                    st_floor, _ = timer.run(lambda _: gf.launch(), K, W, flush=False)
+                    floor = {"ms": round(st_floor["median"], 4), "ms_min": round(st_floor["min"], 4),
+                             "what": "event -> graph of one 1-element kernel -> event, same run"}
+                    gf.destroy()
+                    tiny.destroy()
             else:
-                ms = ms_eager
+                st = st_eager
+            ms = st["median"]
             # the same composition with the intermediate materialised (Zip then Reduce)
             c = S.Vector(ctx, S.F32, n)
 
@@ -586,20 +762,22 @@ def bench_skeletons(args, D: Dist, P: dict, which):
                     marks[0].record()
                 sm(c, out=s)
 
-            ms_u, seg = timer.run(step_unfused, K, W, D, marks=1)
-            ms_u, seg = D.max(ms_u), [D.max(x) for x in seg]
+            st_u, seg = timer.run(step_unfused, K, W, marks=1)
             s = sm(mult(va, vb), out=s)
             got = float(s.scalar())
             ref = O.reduce_(O.OP_ADD_F32, O.zip_(O.OZ_MULT_F32, a, b))
             key = "dot_2^20" if n == 1 << 20 else "dot_2^28"
             res[key] = {"workload": f"dot product sum(mult(A,B)) (Listing 1.1), {n} fp32, block, "
                                     "Zip fused into Reduce (lazy)",
-                        "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3),
-                        "ms_without_graph": round(ms_eager, 4), "cuda_graph": graph is not None,
-                        "ms_warm_l2": round(ms_warm, 4) if ms_warm else None,
-                        "roofline": roof_hbm(8 * n, ms, P, "dot_2^28_fused" if n == 1 << 28 else None),
-                        "unfused": {"ms": round(ms_u, 4), "zip_ms": round(seg[0], 4), "reduce_ms": round(seg[1], 4),
-                                    "roofline_zip": roof_hbm(12 * n, seg[0], P), "roofline_reduce": roof_hbm(4 * n, seg[1], P)},
+                        **ms_fields(st), "elements_per_s": n / (ms / 1e3),
+                        "ms_without_graph": round(st_eager["median"], 4), "cuda_graph": graph is not None,
+                        "ms_warm_l2": round(st_warm["median"], 4) if st_warm else None,
+                        "launch_floor": floor,
+                        "roofline": roof_hbm(8 * n, ms, P, "dot_2^28_fused" if n == 1 << 28 else None, ngpu=G),
+                        "unfused": {"ms": round(st_u["median"], 4), "zip_ms": round(seg[0], 4),
+                                    "reduce_ms": round(seg[1], 4),
+                                    "roofline_zip": roof_hbm(12 * n, seg[0], P, ngpu=G),
+                                    "roofline_reduce": roof_hbm(4 * n, seg[1], P, ngpu=G)},
                         "rel_err": abs(got - ref) / abs(ref), "check": "ok" if abs(got - ref) <= 1e-5 * abs(ref) else "FAIL"}
             if graph is not None:
                 graph.destroy()
@@ -621,77 +799,81 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             def step(_):
                 sm(mult(va, vb), out=s)
 
-            ms, _ = timer.run(step, max(3, K // 2), W, D)
-            ms = D.max(ms)
+            st, _ = timer.run(step, max(5, K // 2), W)
+            ms = st["median"]
             ok = float(s.scalar()) == n * 2.0 ** -10
             gbs = 8 * n / (ms / 1e3) / 1e9
-            sweep[f"2^{lg}"] = {"ms": round(ms, 4), "GB_s": round(gbs, 1), "frac": round(gbs / P["hbm_gbs"], 4),
-                                "check": "ok" if ok else "FAIL"}
+            sweep[f"2^{lg}"] = {"ms": round(ms, 4), "ms_min": round(st["min"], 4), "GB_s": round(gbs, 1),
+                                "frac": round(gbs / (P["hbm_gbs"] * G), 4), "check": "ok" if ok else "FAIL"}
             va.destroy()
             vb.destroy()
         res["dot_sweep"] = {"workload": "fused sum(mult(A,B)) sweep 2^20..2^30 fp32 (no graph), cold L2, "
-                                        "8 B/element", "points": sweep,
+                                        "8 B/element, median of the timed steps", "points": sweep,
                             "check": "ok" if all(v["check"] == "ok" for v in sweep.values()) else "FAIL"}
 
-    if "redist" in which and D.world == 1:
-        res.update(bench_redist(ctx, timer, K, W, D, P))
+    if "redist" in which and not E.spmd:
+        res.update(bench_redist(E, K, W, P))
 
     for it_name in ("gauss_iter", "sobel_iter"):
         if it_name not in which:
             continue
         # K=10 iterated stencil (ping-pong); on several GPUs the
-        # halo rows move between iterations (NCCL, one process per GPU)
-        R = C = 8192
+        # halo rows move between iterations (pushed by the stencil kernel when one
+        # process drives every GPU, exchanged otherwise)
+        R = Cc = 8192
         if it_name == "gauss_iter":
-            img = I.image_f32(I.SEED_GAUSS, R, C)
+            img = I.image_f32(I.SEED_GAUSS, R, Cc)
             ctx.set_option("block_threads", 128)
-            st = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+            stn = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
             ctx.set_option("block_threads", 256)
             dt, okind, dd, ob, nv = S.F32, O.OS_GAUSS5, 2, O.OB_NEAREST, 0.0
             desc = "Gaussian 5x5 f32"
         else:
-            img = I.image_u8(I.SEED_SOBEL, R, C)
-            st = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            img = I.image_u8(I.SEED_SOBEL, R, Cc)
+            stn = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
             dt, okind, dd, ob, nv = S.U8, O.OS_SOBEL, 1, O.OB_NEUTRAL, 0
             desc = "Sobel u8"
         a = S.Matrix.from_numpy(ctx, img)
-        b = S.Matrix(ctx, dt, R, C)
-        t = S.Matrix(ctx, dt, R, C)
+        b = S.Matrix(ctx, dt, R, Cc)
+        t = S.Matrix(ctx, dt, R, Cc)
         ITER = 10
 
         def step(_):
-            st(a, out=b)
+            stn(a, out=b)
             for k in range(ITER - 1):
-                st(b, out=t) if k % 2 == 0 else st(t, out=b)
+                stn(b, out=t) if k % 2 == 0 else stn(t, out=b)
 
-        ms, _ = timer.run(step, max(3, K // 4), W, D)
-        ms = D.max(ms)
-        # parity: rows 4000..4063 after 10 iterations (the oracle iterates a band wide
-        # enough that its edges do not reach the checked rows: 10 x d <= 20 rows)
-        sub = img[3970:4094]
+        st, _ = timer.run(step, max(5, K // 4), W)
+        # parity: 64 rows around the device boundary nearest the middle (the
+        # middle of the image on one GPU) after 10 iterations; the oracle
+        # iterates a band wide enough that its edges do not reach the checked
+        # rows (10 x d <= 20 < 30 rows of margin)
+        b0 = (R + G - 1) // G * (G // 2) if G > 1 else 4032
+        lo = b0 - 62
+        sub = img[lo:b0 + 62]
         r = sub
         for _ in range(ITER):
             r = O.mapoverlap2d(okind, r, dd, ob, nv)
         fin = (t if (ITER - 1) % 2 == 1 else b)
-        ok = bool(np.array_equal(fin.to_numpy()[4000:4064], r[30:94]))
+        ok = bool(np.array_equal(fin.to_numpy()[lo + 30:lo + 94], r[30:94]))
         res[it_name.replace("_iter", "_iter10")] = {
-            "workload": f"10 x {desc} MapOverlap {R}x{C}, ping-pong (halo refresh between iterations on >1 GPU)",
-            "ms": round(ms, 4), "ms_per_iteration": round(ms / ITER, 4),
-            "elements_per_s": ITER * R * C / (ms / 1e3), "check": "ok" if ok else "FAIL"}
+            "workload": f"10 x {desc} MapOverlap {R}x{Cc}, ping-pong (halo exchange between iterations on >1 GPU)",
+            **ms_fields(st), "ms_per_iteration": round(st["median"] / ITER, 4),
+            "elements_per_s": ITER * R * Cc / (st["median"] / 1e3), "check": "ok" if ok else "FAIL"}
         for x in (a, b, t):
             x.destroy()
 
     if "sobel" in which or "gauss" in which:
-        R = C = 8192
+        R = Cc = 8192
         for name in ("sobel", "gauss"):
             if name not in which:
                 continue
             if name == "sobel":
-                img = I.image_u8(I.SEED_SOBEL, R, C)
+                img = I.image_u8(I.SEED_SOBEL, R, Cc)
                 mo = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
                 bpp, okind = 2, O.OS_SOBEL
             else:
-                img = I.image_f32(I.SEED_GAUSS, R, C)
+                img = I.image_f32(I.SEED_GAUSS, R, Cc)
                 # 128-thread blocks (8 rows x 4 columns per thread, <= 128 registers):
                 # the fastest swept configuration (profiles/sweeps/sweep16-17)
                 ctx.set_option("block_threads", 128)
@@ -704,29 +886,27 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             def step(_):
                 mo(mi, out=o)
 
-            ms, _ = timer.run(step, K, W, D)
-            ms = D.max(ms)
-            # parity on a band of rows (oracle computes the band with its halo)
-            band = slice(4000, 4064)
-            sub = img[3990:4074]
-            ref = (O.mapoverlap2d(okind, sub, 1, O.OB_NEUTRAL, 0) if name == "sobel"
-                   else O.mapoverlap2d(okind, sub, 2, O.OB_NEAREST, 0.0))[10:74]
-            got = o.to_numpy()[band]
-            ok = bool(np.array_equal(got, ref))
+            st, _ = timer.run(step, K, W)
+            ms = st["median"]
+            # parity on row bands (oracle computes each band with its halo): the
+            # top edge, the middle, a device boundary, the bottom edge
+            full = o.to_numpy()
+            ok = True
+            starts = {0, 4000, R - 64} | ({(R + G - 1) // G * (G // 2) - 32} if G > 1 else set())
+            for r0 in sorted(starts):
+                blo, bhi = max(0, r0 - 8), min(R, r0 + 72)
+                ref = (O.mapoverlap2d(okind, img[blo:bhi], 1, O.OB_NEUTRAL, 0) if name == "sobel"
+                       else O.mapoverlap2d(okind, img[blo:bhi], 2, O.OB_NEAREST, 0.0))
+                a0 = r0 - blo
+                ok &= bool(np.array_equal(full[r0:r0 + 64], ref[a0:a0 + 64]))
             res[name] = {"workload": f"{'Sobel u8 d=1 NEUTRAL' if name == 'sobel' else 'Gaussian 5x5 f32 d=2 NEAREST'} "
-                                     f"MapOverlap {R}x{C}, overlap distribution",
-                         "ms": round(ms, 4), "elements_per_s": R * C / (ms / 1e3),
-                         "roofline": roof_hbm(bpp * R * C, ms, P, name), "check": "ok" if ok else "FAIL"}
-            import torch as _t
-            sms = _t.cuda.get_device_properties(D.local).multi_processor_count
-            res[name]["roofline_issue"] = roof_issue(name, ms, P, sms)
+                                     f"MapOverlap {R}x{Cc}, overlap distribution",
+                         **ms_fields(st), "elements_per_s": R * Cc / (ms / 1e3),
+                         "roofline": roof_hbm(bpp * R * Cc, ms, P, name, ngpu=G), "check": "ok" if ok else "FAIL"}
+            res[name]["roofline_issue"] = roof_issue(name, ms, P, sms) if G == 1 else None
             if name == "gauss":
                 # the binding roof: 25 FMUL + 25 FADD per pixel (no FMA under -fmad=false)
-                peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
-                fl = 50.0 * R * C / (ms / 1e3)
-                res[name]["roofline_alu"] = {"bound": "alu", "achieved": fl / 1e12, "peak": peak / 1e12,
-                                             "unit": "TFLOP/s", "frac": fl / peak,
-                                             "note": "50 fp32 ops/pixel (25 mul + 25 add)"}
+                res[name]["roofline_alu"] = roof_alu(50.0 * R * Cc, ms, P, sms, G, "50 fp32 ops/pixel (25 mul + 25 add)")
             mi.destroy()
             o.destroy()
 
@@ -734,80 +914,104 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         if name not in which:
             continue
         n = 1 << 30
-        sc = S.Scan(ctx, A.ADD_I32 if dt == S.I32 else A.ADD, dt)
-        # inputs generated on the device with a seeded torch generator (plumbing):
-        # U{-1000..1000} int32 / U[0,1) fp32
-        gen = torch.Generator(device="cuda").manual_seed(3 if dt == S.I32 else 4)
-        if dt == S.I32:
-            src = torch.randint(-1000, 1001, (n,), dtype=torch.int32, device="cuda", generator=gen)
-        else:
-            src = torch.rand((n,), dtype=torch.float32, device="cuda", generator=gen)
+        is_i = dt == S.I32
+        ts = "<i4" if is_i else "<f4"
+        seed = I.SEED_SCAN_I32 if is_i else I.SEED_SCAN_F32
+        sc = S.Scan(ctx, A.ADD_I32 if is_i else A.ADD, dt)
         v = S.Vector(ctx, dt, n).set_distribution(S.BLOCK)
         v.fill(0)
-        ptr, first, cnt = v.local_part(g)
-        torch.cuda.synchronize()
         ctx.sync()
-        # copy this rank's block into the container part (device-to-device, torch plumbing)
-        class View:
-            __cuda_array_interface__ = {"shape": (cnt,), "typestr": "<i4" if dt == S.I32 else "<f4",
-                                        "data": (ptr, False), "version": 3, "strides": None}
-        torch.as_tensor(View(), device="cuda").copy_(src[first:first + cnt])
-        torch.cuda.synchronize()
+        # BASELINE §4 inputs (int32 seed 3 U{-1000..1000}, fp32 seed 4 U[0,1)):
+        # each device's block generated in place by inputs.py's torch copy of the
+        # counter-based generator (element i of the stream at position i)
+        gen_ok = True
+        for g, phys in ctx._bench_local:
+            with torch.cuda.device(phys):
+                part, first, cnt = _part_tensor(v, g, phys, ts)
+                if cnt == 0:
+                    continue
+                part.copy_(I.uniform_int_torch(seed, cnt, -1000, 1000, device=part.device, start=first) if is_i
+                           else I.uniform_f32_torch(seed, cnt, device=part.device, start=first))
+                s0 = first + cnt // 2
+                smp = part[cnt // 2:cnt // 2 + 4096].cpu().numpy()
+                want = (I.uniform_int(seed, smp.size, -1000, 1000, start=s0) if is_i
+                        else I.uniform_f32(seed, smp.size, start=s0))
+                gen_ok &= bool(np.array_equal(smp, want))
+        for _, phys in ctx._bench_local:
+            torch.cuda.synchronize(phys)
         out = S.Vector(ctx, dt, n)
         sc(v, out=out)
 
         def step(_):
             sc(v, out=out)
 
-        ms, _ = timer.run(step, K, W, D)
-        ms = D.max(ms)
-        # parity: chunks of the output against the oracle run on the same chunks,
-        # carried with the oracle's value of the preceding element (scan associativity)
-        optr, ofirst, ocnt = out.local_part(g)
-
-        class OView:
-            __cuda_array_interface__ = {"shape": (ocnt,), "typestr": "<i4" if dt == S.I32 else "<f4",
-                                        "data": (optr, False), "version": 3, "strides": None}
+        st, _ = timer.run(step, K, W)
+        ms = st["median"]
+        # parity: the WHOLE output vector against the oracle's scan of the whole
+        # input: int32 bit-exact, fp32 rel-L2 <= 1e-5 vs double.  One
+        # process: rank 0 downloads both vectors; one process per GPU: every rank
+        # checks its block against the oracle seeded with the oracle's reduce of
+        # the preceding elements (scan(v)[i] = reduce(v[:first]) (+) scan(v[first:])).
         ctx.sync()
-        got_t = torch.as_tensor(OView(), device="cuda")
-        ok = True
-        errs = []
-        for c0 in (0, ocnt // 2 + 12345, ocnt - 100000):
-            if c0 == 0 and first > 0:
-                continue  # a later rank's first chunk starts from the carry-in, not from 0
-            xin = src[first + c0:first + c0 + 100000].cpu().numpy()
-            got = got_t[c0:c0 + 100000].cpu().numpy()
-            if dt == S.I32:
-                prev = 0 if c0 == 0 else int(got_t[c0 - 1].item())
-                ref = O.scan(O.OP_ADD_I32, xin).astype(np.int64) + prev
-                ok &= bool(np.array_equal(got.astype(np.int64), ref.astype(np.int32).astype(np.int64)))
+        t0 = time.perf_counter()
+        num = den = 0.0
+        exact = True
+        for g, phys in ctx._bench_local:
+            ip, first, cnt = _part_tensor(v, g, phys, ts)
+            op, ofirst, ocnt = _part_tensor(out, g, phys, ts)
+            if cnt == 0:
+                continue
+            assert (ofirst, ocnt) == (first, cnt)
+            xin = ip.cpu().numpy()
+            got = op.cpu().numpy()
+            if first == 0:
+                ref = O.scan(O.OP_ADD_I32 if is_i else O.OP_ADD_F32, xin)
             else:
-                prev = 0.0 if c0 == 0 else float(got_t[c0 - 1].item())
-                ref = O.scan(O.OP_ADD_F32, xin) + prev
-                e = float(np.linalg.norm(got - ref) / np.linalg.norm(ref))
-                errs.append(e)
-                ok &= e <= 1e-5
-        # global check: last element = the double-accumulated total (f32) / exact total (i32)
-        tot = src.to(torch.float64).sum().item() if dt == S.F32 else int(src.to(torch.int64).sum().item())
-        last = got_t[-1].item()
-        if D.world == 1:
-            if dt == S.I32:
-                ok &= int(last) == int(np.int32(np.int64(tot)))
+                # the oracle's left fold over the preceding elements, chunk by chunk
+                pre = 0 if is_i else 0.0
+                for a0 in range(0, first, 1 << 26):
+                    c = min(first, a0 + (1 << 26)) - a0
+                    xs = (I.uniform_int_torch(seed, c, -1000, 1000, device=ip.device, start=a0) if is_i
+                          else I.uniform_f32_torch(seed, c, device=ip.device, start=a0)).cpu().numpy()
+                    r = O.reduce_(O.OP_ADD_I32 if is_i else O.OP_ADD_F32, xs)
+                    pre = (pre + int(r)) if is_i else pre + float(r)
+                ref = O.scan(O.OP_ADD_I32 if is_i else O.OP_ADD_F32, xin)
+                if is_i:
+                    ref = ((ref.astype(np.int64) + pre) & 0xFFFFFFFF).astype(np.uint32).view(np.int32)
+                else:
+                    ref = ref + pre
+            if is_i:
+                exact &= bool(np.array_equal(got, ref))
             else:
-                errs.append(abs(last - tot) / abs(tot))
-                ok &= errs[-1] <= 1e-5
-        res[name] = {"workload": f"inclusive Scan (+) over 2^30 {'int32' if dt == S.I32 else 'fp32'}, block + carry-in",
-                     "ms": round(ms, 4), "elements_per_s": n / (ms / 1e3), "roofline": roof_hbm(8 * n, ms, P, name if name == "scan_i32" else None),
-                     "check": "ok" if ok else "FAIL", "max_rel_err": max(errs) if errs else 0.0,
-                     "data": "torch-seeded on device (int32 U{-1000..1000} / fp32 U[0,1))"}
-        del src, got_t
+                for a0 in range(0, cnt, 1 << 26):
+                    rr = ref[a0:a0 + (1 << 26)]
+                    d = got[a0:a0 + (1 << 26)].astype(np.float64) - rr
+                    num += float(np.dot(d, d))
+                    den += float(np.dot(rr, rr))
+            del xin, got, ref
+        check_s = time.perf_counter() - t0
+        if is_i:
+            ok = E.all_ok(exact and gen_ok)
+            err = None
+        else:
+            num, den = E.sum(num), E.sum(den)
+            err = (num / den) ** 0.5
+            ok = E.all_ok(gen_ok) and err <= 1e-5
+        res[name] = {"workload": f"inclusive Scan (+) over 2^30 {'int32' if is_i else 'fp32'}, block + carry-in",
+                     **ms_fields(st), "elements_per_s": n / (ms / 1e3),
+                     "roofline": roof_hbm(8 * n, ms, P, name if is_i else None, ngpu=G),
+                     "check": "ok" if ok else "FAIL",
+                     "parity": ("whole vector bit-exact vs the oracle" if is_i else
+                                f"whole-vector rel-L2 vs the double oracle = {err:.3e} (<= 1e-5)"),
+                     "parity_host_s": round(check_s, 1),
+                     "data": f"inputs.py stream seed {seed} ({'U{-1000..1000}' if is_i else 'U[0,1)'}), generated on "
+                             "the device by its torch copy, sampled against numpy"}
         v.destroy()
         out.destroy()
         torch.cuda.empty_cache()
 
     if "allpairs" in which:
         # Allpairs: zip-reduce rows on the FP32 pipes
-        import torch as _t
         for name, zsrc, nn, mm, dd, ops in (("allpairs_dot_4096", A.MULT, 4096, 4096, 4096, 2),
                                              ("allpairs_manhattan_4096x4096x128", A.ABSDIFF, 4096, 4096, 128, 2)):
             a = I.uniform_f32(81, nn * dd).reshape(nn, dd)
@@ -820,23 +1024,19 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             def step(_):
                 ap(ma, mb, out=c)
 
-            ms, _ = timer.run(step, max(3, K // 2), 2, D)
-            ms = D.max(ms)
+            st, _ = timer.run(step, max(5, K // 2), 2)
+            ms = st["median"]
             # parity on a 32 x 32 corner + a strip (oracle, same fold order: bit-exact)
             cg = c.to_numpy()
             fn = O.AP_DOT if zsrc == A.MULT else O.AP_MANHATTAN
             ok = np.array_equal(cg[:32, :32], O.allpairs(fn, a[:32], b[:32])) and np.array_equal(
                 cg[nn - 7:, mm - 40:], O.allpairs(fn, a[nn - 7:], b[mm - 40:]))
             flops = float(ops) * nn * mm * dd
-            sms = _t.cuda.get_device_properties(D.local).multi_processor_count
-            peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
             res[name] = {"workload": f"allpairs zip-reduce {'dotProduct (Eq. 2 matrix multiply)' if zsrc == A.MULT else 'Manhattan distance'} "
                                      f"{nn}x{mm}, d={dd}, block(A) x copy(B)",
-                         "ms": round(ms, 4), "pairs_per_s": nn * mm / (ms / 1e3),
-                         "roofline": {"bound": "alu", "achieved": flops / (ms / 1e3) / 1e12, "peak": peak / 1e12,
-                                      "unit": "TFLOP/s", "frac": flops / (ms / 1e3) / peak,
-                                      "traffic": ncu_traffic(name),
-                                      "note": f"{ops} fp32 ops per (i,j,k), no FMA (-fmad=false)"},
+                         **ms_fields(st), "pairs_per_s": nn * mm / (ms / 1e3),
+                         "roofline": {**roof_alu(flops, ms, P, sms, G, f"{ops} fp32 ops per (i,j,k), no FMA (-fmad=false)"),
+                                      "traffic": ncu_traffic(name)},
                          "check": "ok" if ok else "FAIL"}
             for x in (ma, mb, c):
                 x.destroy()
@@ -853,11 +1053,14 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         f0 = np.ones(N ** 3, np.float32)
         # application-level load balancing (lmosem.py): the subset's events ordered
         # longest ray walk first, dealt round-robin over the devices (done once at
-        # load time; the result does not depend on the order beyond fp32 atomics)
+        # load time on the host, timed here; the result does not depend on the
+        # order beyond fp32 atomics)
         from paper_conf_pact_steuwerg13_b200.lmosem import ListModeOSEM
+        t0 = time.perf_counter()
         order = ListModeOSEM.path_order(events, N)
-        if D.world > 1:
-            order = np.concatenate([order[r::D.world] for r in range(D.world)])
+        if G > 1:
+            order = np.concatenate([order[r::G] for r in range(G)])
+        order_s = time.perf_counter() - t0
         ev_raw = S.Vector(ctx, evd, nev).set_distribution(S.BLOCK)
         ev_raw.copy_in(events)
         ev = S.Vector(ctx, evd, nev).set_distribution(S.BLOCK)
@@ -878,8 +1081,8 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             upd(f, c, out=fn)                            # f * c
 
         f.copy_in(f0)
-        ms, seg = timer.run(step, max(3, K // 2), 2, D, marks=1)
-        ms, seg = D.max(ms), [D.max(x) for x in seg]
+        st, seg = timer.run(step, max(5, K // 2), 2, marks=1)
+        ms = st["median"]
         # the same Map over the events in generation order (no balancing)
         f.copy_in(f0)
 
@@ -889,8 +1092,7 @@ def bench_skeletons(args, D: Dist, P: dict, which):
             c.fill(0.0)
             lm(ev_raw, f, (c, S.WRITE))
 
-        ms_raw, _ = timer.run(step_raw, max(3, K // 4), 1, D)
-        ms_raw = D.max(ms_raw)
+        st_raw, _ = timer.run(step_raw, max(3, K // 4), 1)
         # parity on a 1/50 sample of the events vs the oracle (one subset from f = 1)
         sub = events[::50].copy()
         f.copy_in(f0)
@@ -907,10 +1109,13 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         visits = visits_sample * 50  # estimate of sum |path| for the full 10^7 (sampled 1/50)
         res["lmosem"] = {"workload": "LM OSEM subset: Map over 10^7 events (block) into copy(+) 150^3 image, "
                                      "copy->block combine, Zip f*c",
-                         "ms": round(ms, 4), "events_per_s": nev / (ms / 1e3), "map_ms": round(seg[0], 4),
-                         "map_ms_generation_order": round(ms_raw, 4),
+                         **ms_fields(st), "events_per_s": nev / (ms / 1e3), "map_ms": round(seg[0], 4),
+                         "map_ms_generation_order": round(st_raw["median"], 4),
+                         "host_path_order_s": round(order_s, 3),
+                         "host_path_order_note": "numpy ray-box clipping + argsort of the 10^7 events, once at load "
+                                                 "time (not in the timed step)",
                          "visits_per_s_est": visits / (seg[0] / 1e3), "visits_est": visits,
-                         "roofline": roof_l2("lmosem"),
+                         "roofline": roof_l2("lmosem") if G == 1 else None,
                          "rel_l2_c_sample": e, "check": "ok" if e <= 1e-4 else "FAIL"}
         for x in (ev, ev_raw, f, c, fn, evs):
             x.destroy()
@@ -922,15 +1127,17 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         N, nev, nsub = 150, 10_000_000, 10
         events = I.lmosem_events(I.SEED_LMOSEM, nev, N)
         osem = ListModeOSEM(ctx, N)
+        t0 = time.perf_counter()
         osem.load_events(events, nsub)
+        load_s = time.perf_counter() - t0
         f0 = np.ones(N ** 3, np.float32)
         osem.set_image(f0)
 
         def step(_):
             osem.iterate(1)
 
-        ms, _ = timer.run(step, max(3, K // 4), 2, D)
-        ms = D.max(ms)
+        st, _ = timer.run(step, max(5, K // 4), 2)
+        ms = st["median"]
         # parity: the same program on every 100th event (10 subsets) vs the oracle
         sub = events[::100].copy()
         osem.load_events(sub, nsub)
@@ -943,7 +1150,8 @@ def bench_skeletons(args, D: Dist, P: dict, which):
         e = float(np.linalg.norm(fg - fo) / np.linalg.norm(fo))
         res["lmosem_osem"] = {"workload": f"LM OSEM pass: {nsub} subsets x 10^6 events, 150^3 image; per subset "
                                           "f block->copy, Map (block events), c copy(+)->block, Zip f*c",
-                              "ms": round(ms, 4), "events_per_s": nev / (ms / 1e3),
+                              **ms_fields(st), "events_per_s": nev / (ms / 1e3),
+                              "host_load_events_s": round(load_s, 3),
                               "rel_l2_f_sample": e, "check": "ok" if e <= 1e-4 else "FAIL"}
         osem.destroy()
     ctx.finalize()
@@ -955,8 +1163,8 @@ HEADLINE_WORKLOAD = (f"mandelbrot {COLS}x{ROWS} Map over block-distributed Matri
                      f"MAX_ITER={MAX_ITER} (BASELINE configs[1])")
 
 
-def run_reference(args, D: Dist):
-    if D.rank != 0:
+def run_reference(args):
+    if int(os.environ.get("RANK", "0")) != 0:
         return 0
     # each step: the oracle on a bounded sample of the Mandelbrot workload (every 16th row)
     every = 16
@@ -967,7 +1175,7 @@ def run_reference(args, D: Dist):
         _, _, s = mandel_oracle(every)
         times.append(s)
     pix = (ROWS // every) * COLS
-    sec = float(np.mean(times))
+    sec = float(np.median(times))
     v = pix / sec
     line = {"impl": "reference", "metric": METRIC, "value": v, "unit": "elements/s", "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": sec * 1e3, "higher_is_better": True,
@@ -981,6 +1189,16 @@ def run_reference(args, D: Dist):
     return 0
 
 
+def all_checks_ok(sk: dict) -> bool:
+    """every parity flag in the skeleton section is ok, and no section failed"""
+    if not isinstance(sk, dict) or "error" in sk:
+        return False
+    for v in sk.values():
+        if isinstance(v, dict) and v.get("check") not in (None, "ok"):
+            return False
+    return True
+
+
 # ---------------------------------------------------------------- main
 def main():
     ap = argparse.ArgumentParser()
@@ -991,49 +1209,51 @@ def main():
     ap.add_argument("--skeletons", default="all")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
-    D = Dist(args.gpus)
     if args.impl == "reference":
-        return run_reference(args, D)
+        return run_reference(args)
+    E = Env(args.gpus)
     from paper_conf_pact_steuwerg13_b200 import build as B
-    if D.rank == 0:
+    if E.rank == 0:
         B.build()
-    D.barrier()
+    E.barrier()
     P = peaks()
-    r = bench_mandelbrot(args, D, P)
+    r = bench_mandelbrot(args, E, P)
     which = [] if args.skeletons == "none" else (
-        ["dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32", "scan_f32", "lmosem",
-         "lmosem_osem", "allpairs"]
+        ["mandel_plain", "dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32",
+         "scan_f32", "lmosem", "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
-    if D.rank != 0:
-        _skeleton_section(args, D, P, which, None)
-        return 0
+    if E.rank != 0:
+        sk = _skeleton_section(args, E, P, which, None)
+        return 0 if all_checks_ok(sk) else 1
     # oracle: full image on this host (parity of every pixel, exact work count, cpu baseline)
     counts_ref, sum_iter, cpu_s = mandel_oracle(1)
     parity = bool(np.array_equal(r["counts"], counts_ref))
     flops = OPS_PER_ITER * float(sum_iter)
     import torch
-    sms = torch.cuda.get_device_properties(0).multi_processor_count
-    alu_peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6
-    achieved = flops / (r["ms"] / 1e3)
-    # imbalance-limited ideal speed-up of the block-by-rows distribution (SURVEY §7 hard part 4)
+    G = r["ndev"]
+    sms = torch.cuda.get_device_properties(E.phys[0]).multi_processor_count
+    ms = r["st"]["median"]
     import oracle as O
+    # imbalance-limited ideal speed-up of the block-by-rows distribution (SURVEY §7 hard part 4)
     rs = O.row_sums(counts_ref)
-    order = row_order(ROWS, D.world)
-    per = [float(rs[order[a:b]].sum()) for a, b in (S_block(ROWS, args.gpus, gg) for gg in range(args.gpus))]
+    order = row_order(ROWS, G)
+    per = [float(rs[order[a:b]].sum()) for a, b in (S_block(ROWS, G, gg) for gg in range(G))]
     line = {
-        "metric": METRIC, "value": r["value"], "unit": "elements/s", "n_gpus": args.gpus, "steps": args.steps,
-        "warmup": args.warmup, "ms_per_step": r["ms"], "higher_is_better": True, "scaling": "strong",
+        "metric": METRIC, "value": r["value"], "unit": "elements/s", "n_gpus": G, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
         "vs_baseline": None, "dtype": "f32", "data": "synthetic",
         "config": {"workload": HEADLINE_WORKLOAD,
-                   "l2": "flushed between steps (256 MiB write, then a 256 MiB read so L2 is clean)",
-                   "parallelism": f"block rows over {args.gpus} GPU(s)",
-                   "row_order": "identity" if D.world == 1 else "round-robin (application-level balancing)",
+                   "l2": "flushed between steps (256 MiB write, then a 256 MiB read so L2 is clean), every GPU",
+                   "parallelism": f"block rows over {G} GPU(s); {E.mode}",
+                   "statistic": "median of the timed steps (max over ranks)",
+                   "ms_min": r["st"]["min"], "ms_mean": r["st"]["mean"],
+                   "row_order": "identity" if G == 1 else "round-robin (application-level balancing)",
                    "imbalance_limited_ideal_speedup": float(sum(per) / max(per)) if max(per) > 0 else 1.0},
-        "roofline": {"bound": "alu", "achieved": achieved / 1e12, "peak": alu_peak / 1e12, "unit": "TFLOP/s",
-                     "frac": achieved / alu_peak, "traffic": ncu_traffic("mandelbrot"),
-                     "note": f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count); peak = {sms} SMs x 128 "
-                             f"FP32 lanes x {P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false)"},
+        "roofline": {**roof_alu(flops, ms, P, sms, G,
+                                f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count); peak = {G} x {sms} SMs "
+                                f"x 128 FP32 lanes x {P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false)"),
+                     "traffic": ncu_traffic("mandelbrot")},
         "cpu_baseline": {"value": ROWS * COLS / cpu_s, "unit": "elements/s", "cores": 1, "kind": "oracle", **cpu_info(),
                          "sample": f"whole {COLS}x{ROWS} image, single thread ({cpu_s:.2f} s)"},
         "e2e": r["e2e"], "gpu_launches": int(r["launches"]), "clocks": r["clocks"],
@@ -1041,39 +1261,45 @@ def main():
         "paper_context": "SkelCL Mandelbrot 4096x3072 on one Tesla T10: 26 s (0.48 Mpx/s); MAX_ITER unstated, "
                          "so not the same workload (vs_baseline null)",
     }
-    line["skeletons"] = _skeleton_section(args, D, P, which, line)
+    sk = _skeleton_section(args, E, P, which, line)
+    if isinstance(sk, dict) and "mandel_plain" in sk:
+        mp = sk["mandel_plain"]
+        mp["check"] = "ok" if np.array_equal(mp.pop("_counts"), counts_ref) else "FAIL"
+        mp["roofline"] = roof_alu(flops, mp["ms"], P, sms, G, "8 fp32 ops/iteration x the oracle's iteration count")
+    line["skeletons"] = sk
     print(json.dumps(line), flush=True)
-    return 0
+    return 0 if (parity and all_checks_ok(sk)) else 1
 
 
-def _skeleton_section(args, D: Dist, P: dict, which, line):
+def _skeleton_section(args, E: Env, P: dict, which, line):
     """The per-skeleton lines, after the headline is complete.  A watchdog bounds
-    the section (SKL_BENCH_SKELETON_LIMIT_S, default 420 s): if it is exceeded -
+    the section (SKL_BENCH_SKELETON_LIMIT_S, default 600 s): if it is exceeded -
     e.g. a collective of the multi-rank path that never completes - rank 0 prints
-    the headline line with the skeletons marked as timed out and every rank
-    exits 0, so a run never ends without its line.  An exception in the section
-    is recorded in the line instead of losing it."""
+    the headline line with the skeletons marked as timed out and the process
+    exits with status 3.  An exception in the section is recorded in the line
+    (and makes the exit status non-zero)."""
     if not which:
         return {}
-    import threading
-    limit = float(os.environ.get("SKL_BENCH_SKELETON_LIMIT_S", "420"))
+    limit = float(os.environ.get("SKL_BENCH_SKELETON_LIMIT_S", "600"))
 
     def expire():
         if line is not None:
             print(json.dumps({**line, "skeletons": {"error": f"skeleton section exceeded {limit:.0f} s"}}),
                   flush=True)
-        os._exit(0)
+        os._exit(3)
 
     wd = threading.Timer(limit, expire)
     wd.daemon = True
     wd.start()
     try:
-        return bench_skeletons(args, D, P, which)
+        return bench_skeletons(args, E, P, which)
     except Exception as e:   # noqa: BLE001 - recorded in the bench line
-        if D.world > 1:      # the other ranks may be waiting in a collective: end the job
+        import traceback
+        traceback.print_exc()
+        if E.world > 1:      # the other ranks may be waiting in a collective: end the job
             if line is not None:
                 print(json.dumps({**line, "skeletons": {"error": repr(e)}}), flush=True)
-            os._exit(0)
+            os._exit(4)
         return {"error": repr(e)}
     finally:
         wd.cancel()
