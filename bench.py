@@ -743,7 +743,7 @@ def bench_skeletons(args, E: Env, P: dict, which):
                     st_warm, _ = timer.run(lambda _: graph.launch(), K, W, flush=False)
                     # the floor of this step in the same run: a graph of ONE
                     # one-element fill kernel between the same events
-                    tiny = S.Vector(ctx, S.F32, 1).set_distribution(S.BLOCK)
+                    tiny = S.Vector(ctx, S.F32, 1).set_distribution(S.BLOCK).fill(1.0)   # allocated before capture
                     gf = ctx.capture(lambda: tiny.fill(0.0))
                     st_floor, _ = timer.run(lambda _: gf.launch(), K, W, flush=False)
                     floor = {"ms": round(st_floor["median"], 4), "ms_min": round(st_floor["min"], 4),

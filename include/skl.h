@@ -136,6 +136,10 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * replicas in one kernel, no staging copy; logical devices of one GPU share one
  * launch; 2 = one kernel per device even then; 0 = slices exchanged into
  * staging, then folded; default 1),
+ * "mo_tma" (1 = a 2-D MapOverlap block stages its tile with one TMA copy,
+ * where TMA can describe the tile: 16-byte aligned rows, staged row <= 256
+ * units of up to 8 bytes, <= 256 rows; 0 = per-thread cp.async staging;
+ * default 1),
  * "mo_ws" (1 = 2-D MapOverlap tiles are staged by a TMA producer warp into a
  * ring of "mo_ws_stages" shared-memory buffers consumed by the other warps of
  * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged

@@ -40,11 +40,31 @@ union SklMoRes {
   SKL_TOUT e[SKL_CW];
   typename SklRaw<SKL_OUTB>::type raw;
 };
+// four byte results -> one 32-bit word with three byte permutes (PRMT); the
+// union's bytewise assembly took five shift/mask instructions per word
+__device__ __forceinline__ unsigned skl_pack4(unsigned b0, unsigned b1, unsigned b2, unsigned b3) {
+  return __byte_perm(__byte_perm(b0, b1, 0x3340), __byte_perm(b2, b3, 0x3340), 0x5410);
+}
 // store one thread's SKL_CW outputs of a row at o (ncols columns remain in the row)
 __device__ __forceinline__ void skl_mo_store(SKL_TOUT* o, const SklMoRes& v, bool full, long ncols) {
 #if SKL_OUT_PACK
   if (full) {
+#if SKL_SO == 1 && SKL_CW % 4 == 0
+    unsigned w[SKL_CW / 4];
+#pragma unroll
+    for (int k = 0; k < SKL_CW / 4; ++k)
+      w[k] = skl_pack4((unsigned char)v.e[4 * k], (unsigned char)v.e[4 * k + 1], (unsigned char)v.e[4 * k + 2],
+                       (unsigned char)v.e[4 * k + 3]);
+#if SKL_CW == 16
+    *(uint4*)o = make_uint4(w[0], w[1], w[2], w[3]);
+#elif SKL_CW == 8
+    *(uint2*)o = make_uint2(w[0], w[1]);
+#else
+    *(unsigned*)o = w[0];
+#endif
+#else
     *(typename SklRaw<SKL_OUTB>::type*)o = v.raw;
+#endif
     return;
   }
 #endif
@@ -198,6 +218,89 @@ skl_mo2d(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT* _
   (void)in_rows;
 }
 
+// TMA staging (option mo_tma, the default where a tensor map can describe the
+// part): one thread stages the block's whole (TH + 2d) x PITCH window with a
+// single cp.async.bulk.tensor.2d (out-of-matrix cells zero-filled by the copy
+// engine, NEAREST / non-zero neutral border tiles patched in shared memory),
+// the block waits on an mbarrier and applies f as skl_mo2d does.  The per-thread
+// staging walk (address arithmetic and one cp.async per 16 bytes, plus the
+// general path for border tiles) was ~40 % of the instructions of a byte stencil
+// (ncu of the identity u8 stencil: 258 instructions per warp for 32 outputs
+// per thread).  x coordinates are in 2^ushift-byte units.
+struct alignas(64) SklTmap {
+  unsigned long long opaque[16];
+};
+__device__ __forceinline__ void skl_mbar_wait(unsigned a, unsigned parity) {
+  unsigned done;
+  do {
+    asm volatile(
+        "{ .reg .pred p; mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2; selp.u32 %0, 1, 0, p; }"
+        : "=r"(done) : "r"(a), "r"(parity) : "memory");
+  } while (!done);
+}
+// Out-of-matrix cells of a TMA-staged tile (zero-filled) get the boundary mode's
+// value: NEAREST copies the nearest in-matrix row, then column (each coordinate
+// clamped independently, A20); NEUTRAL writes the neutral value.  All nthr
+// threads of the block (named barrier 1) take part.
+template <int NT>
+__device__ __forceinline__ void skl_mo_fix(SKL_TIN* tile, const SklMoGeo& G, int r0, int c0, SKL_TIN neutral) {
+  const int gr0 = r0 - SKL_D, gc0 = c0 - SKL_A;
+  const int top = gr0 < 0 ? -gr0 : 0, bot = G.Ri - gr0;  // rows [top, bot) are inside
+  const int left = gc0 < 0 ? -gc0 : 0, right = G.Ci - gc0;
+#if SKL_BOUNDARY == 1
+  if (top > 0 || bot < SKL_SROWS) {
+    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += NT) {
+      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+      if (i < top) tile[q] = tile[top * SKL_PITCH + j];
+      else if (i >= bot) tile[q] = tile[(bot - 1) * SKL_PITCH + j];
+    }
+    asm volatile("bar.sync 1, %0;" ::"n"(NT) : "memory");
+  }
+  if (left > 0 || right < SKL_PITCH) {
+    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += NT) {
+      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+      if (j < left) tile[q] = tile[i * SKL_PITCH + left];
+      else if (j >= right) tile[q] = tile[i * SKL_PITCH + right - 1];
+    }
+  }
+#else
+  for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += NT) {
+    const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
+    if (i < top || i >= bot || j < left || j >= right) tile[q] = neutral;
+  }
+#endif
+  asm volatile("bar.sync 1, %0;" ::"n"(NT) : "memory");
+}
+
+extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
+skl_mo2d_t(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, long in_row0, long out_row0, long R,
+           long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok, SKL_TOUT* __restrict__ push_up,
+           SKL_TOUT* __restrict__ push_down, long hd, int fix, int ushift) {
+  __shared__ __align__(128) SKL_TIN tile[SKL_SROWS * SKL_PITCH];
+  __shared__ __align__(8) unsigned long long bar;
+  constexpr unsigned TB = SKL_SROWS * SKL_PITCH * (unsigned)sizeof(SKL_TIN);
+  const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
+  const int r0 = G.rb + (int)blockIdx.y * SKL_TH;
+  const int c0 = (int)blockIdx.x * SKL_TW;
+  const unsigned b = (unsigned)__cvta_generic_to_shared(&bar);
+  if (threadIdx.x == 0) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b) : "memory");
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(b), "n"(TB) : "memory");
+    asm volatile(
+        "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::
+            "r"((unsigned)__cvta_generic_to_shared(tile)),
+        "l"((unsigned long long)&tmap), "r"(((c0 - SKL_A) * (int)sizeof(SKL_TIN)) >> ushift),
+        "r"(r0 - SKL_D - G.irow0), "r"(b)
+        : "memory");
+  }
+  __syncthreads();  // the barrier is initialised before anyone waits on it
+  skl_mbar_wait(b, 0);
+  if (fix && (r0 - SKL_D < 0 || r0 + SKL_TH + SKL_D > G.Ri || c0 - SKL_A < 0 || c0 + SKL_TW + SKL_A > G.Ci))
+    skl_mo_fix<SKL_BLOCK>(tile, G, r0, c0, neutral);
+  skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
+}
+
 // Persistent variant: a grid of resident blocks walks the tiles (t = blockIdx.x,
 // + gridDim.x, ...) with two shared-memory buffers, staging tile k+1 while
 // applying f to tile k, so the load latency of a tile hides behind the
@@ -241,61 +344,18 @@ skl_mo2d_p(const SKL_TIN* __restrict__ in, long in_row0, long in_rows, SKL_TOUT*
 // next tiles' loads are always in flight while f runs.  Border tiles whose
 // boundary mode is not "zero" (NEAREST, or NEUTRAL with a non-zero value) are
 // patched in shared memory by the consumers before f runs.
-struct alignas(64) SklTmap {
-  unsigned long long opaque[16];
-};
 #define SKL_WS_MAXS 8
 #ifndef SKL_WS_MINB
 #define SKL_WS_MINB 1
 #endif
-__device__ __forceinline__ void skl_mbar_wait(unsigned a, unsigned parity) {
-  unsigned done;
-  do {
-    asm volatile(
-        "{ .reg .pred p; mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2; selp.u32 %0, 1, 0, p; }"
-        : "=r"(done) : "r"(a), "r"(parity) : "memory");
-  } while (!done);
-}
 __device__ __forceinline__ void skl_bar_consumers() {
   asm volatile("bar.sync 1, %0;" ::"n"(SKL_BLOCK) : "memory");
-}
-
-// Out-of-matrix cells of a TMA-staged tile (zero-filled) get the boundary mode's
-// value: NEAREST copies the nearest in-matrix row, then column (each coordinate
-// clamped independently, A20); NEUTRAL writes the neutral value.
-__device__ __forceinline__ void skl_mo_fix(SKL_TIN* tile, const SklMoGeo& G, int r0, int c0, SKL_TIN neutral) {
-  const int gr0 = r0 - SKL_D, gc0 = c0 - SKL_A;
-  const int top = gr0 < 0 ? -gr0 : 0, bot = G.Ri - gr0;  // rows [top, bot) are inside
-  const int left = gc0 < 0 ? -gc0 : 0, right = G.Ci - gc0;
-#if SKL_BOUNDARY == 1
-  if (top > 0 || bot < SKL_SROWS) {
-    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
-      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
-      if (i < top) tile[q] = tile[top * SKL_PITCH + j];
-      else if (i >= bot) tile[q] = tile[(bot - 1) * SKL_PITCH + j];
-    }
-    skl_bar_consumers();
-  }
-  if (left > 0 || right < SKL_PITCH) {
-    for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
-      const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
-      if (j < left) tile[q] = tile[i * SKL_PITCH + left];
-      else if (j >= right) tile[q] = tile[i * SKL_PITCH + right - 1];
-    }
-  }
-#else
-  for (int q = threadIdx.x; q < SKL_SROWS * SKL_PITCH; q += SKL_BLOCK) {
-    const int i = q / SKL_PITCH, j = q - i * SKL_PITCH;
-    if (i < top || i >= bot || j < left || j >= right) tile[q] = neutral;
-  }
-#endif
-  skl_bar_consumers();
 }
 
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK + 32, SKL_WS_MINB)
 skl_mo2d_ws(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, long in_row0, long out_row0,
             long R, long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok, SKL_TOUT* __restrict__ push_up,
-            SKL_TOUT* __restrict__ push_down, long hd, int tiles_x, int ntiles, int nstages, int fix, int xscale) {
+            SKL_TOUT* __restrict__ push_down, long hd, int tiles_x, int ntiles, int nstages, int fix, int ushift) {
   extern __shared__ __align__(128) unsigned char skl_mo_dyn[];
   __shared__ __align__(8) unsigned long long bars[2 * SKL_WS_MAXS];
   constexpr unsigned TB = SKL_SROWS * SKL_PITCH * (unsigned)sizeof(SKL_TIN);
@@ -326,7 +386,7 @@ skl_mo2d_ws(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, lo
         asm volatile(
             "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], "
             "[%4];" ::"r"(base + TS * s),
-            "l"((unsigned long long)&tmap), "r"((c0 - SKL_A) * xscale), "r"(r0 - SKL_D - G.irow0),
+            "l"((unsigned long long)&tmap), "r"(((c0 - SKL_A) * (int)sizeof(SKL_TIN)) >> ushift), "r"(r0 - SKL_D - G.irow0),
             "r"(full0 + 8u * s)
             : "memory");
       }
@@ -341,7 +401,7 @@ skl_mo2d_ws(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, lo
     const int r0 = G.rb + (t / tiles_x) * SKL_TH, c0 = (t % tiles_x) * SKL_TW;
     const bool border = fix && (r0 - SKL_D < 0 || r0 + SKL_TH + SKL_D > G.Ri || c0 - SKL_A < 0 ||
                                 c0 + SKL_TW + SKL_A > G.Ci);
-    if (border) skl_mo_fix(tile, G, r0, c0, neutral);
+    if (border) skl_mo_fix<SKL_BLOCK>(tile, G, r0, c0, neutral);
     skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
     // generic-proxy writes of the patch must be ordered before the next TMA write
     if (border) asm volatile("fence.proxy.async.shared::cta;" ::: "memory");

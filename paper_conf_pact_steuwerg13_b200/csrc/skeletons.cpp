@@ -206,7 +206,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       defs += "#define SKL_PITCH " + std::to_string(tw + 2 * A) + "\n";
       defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_TH " + std::to_string(th) + "\n";
       defs += "#define SKL_CW " + std::to_string(cw) + "\n#define SKL_RH " + std::to_string(rh) + "\n";
-      defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n";
+      defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n#define SKL_SO " + std::to_string(so) + "\n";
       defs += "#define SKL_MO1D 0\n";
       // resident blocks per SM the register allocation must allow (default: 64
       // registers per thread for byte images - 87 registers halved the Sobel
@@ -927,14 +927,17 @@ static bool plan_halo_push(Ctx* ctx, Cont* o, size_t d, std::vector<void*>& up, 
   return true;
 }
 
-// TMA descriptor of a device's input part for skl_mo2d_ws: a 2-D tiled map over
-// rows x columns (row pitch C * elt bytes, a multiple of 16), box = the staged
-// window (pitch x srows elements).  Elements are described as 8/4/2/1-byte
-// units (the largest dividing elt; xscale units per element).  Returns false
-// when TMA cannot describe it (box wider than 256 units, no driver entry
-// point): the caller uses skl_mo2d.
+// TMA descriptor of a device's input part for skl_mo2d_t / skl_mo2d_ws: a 2-D
+// tiled map over rows x columns (row pitch C * elt bytes, a multiple of 16),
+// box = the staged window (pitch x srows elements).  The row is described in
+// 2^ushift-byte units: the widest of 8/4/2/1 bytes that divides the window's
+// width and offsets in bytes (every window starts at a multiple of 16 bytes:
+// tile widths and the halo width A are 16-byte multiples), so a byte image's
+// 544-byte window is 68 units, inside the 256-unit box limit.  Returns false
+// when TMA cannot describe it (box wider than 256 units or taller than 256
+// rows, no driver entry point): the caller uses skl_mo2d.
 static bool encode_tile_map(SklTensorMap* tm, const void* base, size_t elt, size_t C, size_t rows, size_t pitch,
-                            size_t srows, int* xscale) {
+                            size_t srows, int* ushift) {
   static PFN_cuTensorMapEncodeTiled_v12000 enc = nullptr;
   static bool tried = false;
   if (!tried) {
@@ -948,22 +951,24 @@ static bool encode_tile_map(SklTensorMap* tm, const void* base, size_t elt, size
       (void)cudaGetLastError();
   }
   if (!enc) return false;
-  const size_t unit = elt % 8 == 0 ? 8 : elt % 4 == 0 ? 4 : elt % 2 == 0 ? 2 : 1;
-  const size_t sc = elt / unit;
-  if (pitch * sc > 256 || srows > 256 || rows == 0 || rows >= (1ull << 31) || C * sc >= (1ull << 31)) return false;
+  const size_t wb = pitch * elt;  // window width in bytes (a multiple of 16)
+  const size_t unit = wb % 8 == 0 ? 8 : wb % 4 == 0 ? 4 : wb % 2 == 0 ? 2 : 1;
+  if ((C * elt) % unit != 0) return false;
+  const size_t units = wb / unit, cu = C * elt / unit;
+  if (units > 256 || srows > 256 || rows == 0 || rows >= (1ull << 31) || cu >= (1ull << 31)) return false;
   const CUtensorMapDataType dt = unit == 8 ? CU_TENSOR_MAP_DATA_TYPE_UINT64
                                  : unit == 4 ? CU_TENSOR_MAP_DATA_TYPE_UINT32
                                  : unit == 2 ? CU_TENSOR_MAP_DATA_TYPE_UINT16
                                              : CU_TENSOR_MAP_DATA_TYPE_UINT8;
-  const cuuint64_t dims[2] = {(cuuint64_t)(C * sc), (cuuint64_t)rows};
+  const cuuint64_t dims[2] = {(cuuint64_t)cu, (cuuint64_t)rows};
   const cuuint64_t strides[1] = {(cuuint64_t)(C * elt)};
-  const cuuint32_t box[2] = {(cuuint32_t)(pitch * sc), (cuuint32_t)srows};
+  const cuuint32_t box[2] = {(cuuint32_t)units, (cuuint32_t)srows};
   const cuuint32_t estr[2] = {1, 1};
   const CUresult r = enc((CUtensorMap*)tm, dt, 2, const_cast<void*>(base), dims, strides, box, estr,
                          CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE,
                          CU_TENSOR_MAP_L2_PROMOTION_L2_128B, CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   if (r != CUDA_SUCCESS) return false;
-  *xscale = (int)sc;
+  *ushift = unit == 8 ? 3 : unit == 4 ? 2 : unit == 2 ? 1 : 0;
   return true;
 }
 
@@ -1016,10 +1021,20 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       const dim3 grid((unsigned)ceil_div((size_t)C, (size_t)s->mo_tw),
                       (unsigned)ceil_div(r.size(), (size_t)s->mo_th));
       SklTensorMap tm;
-      int xscale = 1;
-      if (ctx->mo_ws && vec_ok &&
-          encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
-                          (size_t)(s->mo_th + 2 * s->d), &xscale)) {
+      int ushift = 0;
+      // fix: TMA-staged border tiles need patching unless the boundary value is zero
+      int fix = s->boundary == 1 ? 1 : 0;
+      for (unsigned char b : s->neutral) fix |= b != 0;
+      const bool tma = (ctx->mo_ws || (ctx->mo_tma && !ctx->mo_persist)) && vec_ok &&
+                       encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
+                                       (size_t)(s->mo_th + 2 * s->d), &ushift);
+      if (tma && !ctx->mo_ws) {
+        // one tile per block, staged by one TMA copy (skl_mo2d_t)
+        void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
+                         &pu, &pd, &hd, &fix, &ushift};
+        launch(ctx, g, s->prog, "skl_mo2d_t", grid, dim3(s->block), 0, targs);
+        ctx->n_tma++;
+      } else if (tma) {
         // TMA producer warp + consumer warps over a ring of staged tiles
         const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;
         const int nst = ctx->mo_ws_stages;
@@ -1028,11 +1043,8 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
         const int nthr = s->block + 32;
         const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_mo2d_ws", nthr, smem));
         const size_t pgrid = std::min((size_t)ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
-        // fix: border tiles need patching unless the boundary value is zero
-        int fix = s->boundary == 1 ? 1 : 0;
-        for (unsigned char b : s->neutral) fix |= b != 0;
         void* wargs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
-                         &pu, &pd, &hd, &tiles_x, &ntiles, (void*)&nst, &fix, &xscale};
+                         &pu, &pd, &hd, &tiles_x, &ntiles, (void*)&nst, &fix, &ushift};
         launch(ctx, g, s->prog, "skl_mo2d_ws", dim3((unsigned)pgrid), dim3((unsigned)nthr), smem, wargs);
         ctx->n_tma++;
       } else if (ctx->mo_persist) {
@@ -1062,7 +1074,8 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       defs += "#define SKL_A " + std::to_string(A) + "\n#define SKL_PITCH 0\n";
       defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_TH 1\n#define SKL_CW " +
               std::to_string(cw) + "\n#define SKL_RH 1\n#define SKL_MO1D 1\n#define SKL_OUTB " +
-              std::to_string((size_t)cw * ctx->type(s->tout).size) + "\n";
+              std::to_string((size_t)cw * ctx->type(s->tout).size) + "\n#define SKL_SO " +
+              std::to_string(ctx->type(s->tout).size) + "\n";
       const std::string user = "\n#line 1 \"user_source\"\n" + s->user_src + "\n#line 1 \"skeleton_template\"\n";
       s->prog1d = compile(ctx, defs + program_source(ctx, user + kernel_template("common.cuh") +
                                                                    kernel_template("mapoverlap.cuh")),

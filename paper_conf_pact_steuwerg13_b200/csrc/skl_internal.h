@@ -137,6 +137,7 @@ struct Ctx {
   int mo_rh = 0, mo_cw = 0;    // MapOverlap outputs per thread (rows x cols); 0 = auto
   int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
   int mo_persist = 0;          // MapOverlap 2-D: persistent blocks, double-buffered tiles
+  int mo_tma = 1;              // MapOverlap 2-D: one TMA copy stages a block's tile (skl_mo2d_t)
   int mo_ws = 0;               // MapOverlap 2-D: TMA producer warp + consumer warps (skl_mo2d_ws)
   int mo_ws_stages = 4;        //   shared-memory ring depth
   int mo_ws_minb = 0;          //   resident blocks per SM the registers must allow (0 = auto)

@@ -1,0 +1,142 @@
+"""GPU parity tests for the TMA-staged one-tile-per-block 2-D MapOverlap kernel
+(skl_mo2d_t, option mo_tma, the default where a tensor map describes the part;
+DESIGN.md 6.3): one cp.async.bulk.tensor copy stages a block's window, cells
+outside the matrix are zero-filled by the copy engine and patched for NEAREST
+and non-zero NEUTRAL (A20).  Bit-exact against the oracle at sizes
+spanning several tiles with ragged edges, every boundary mode, byte and float
+images, logical multi-device runs with the fused halo push; the per-thread
+cp.async kernel (mo_tma=0) gives the same results.  Also the separable Sobel
+user function (apps.SOBEL_SEPARABLE): full images and its square-root step for
+every m."""
+import re
+
+import numpy as np
+import pytest
+
+import oracle as O
+from gpu_util import require_gpu
+from paper_conf_pact_steuwerg13_b200 import apps as A
+from paper_conf_pact_steuwerg13_b200 import inputs as I
+from paper_conf_pact_steuwerg13_b200 import skl as S
+
+pytestmark = pytest.mark.gpu
+
+SHAPES_F32 = [(1, 4), (3, 16), (37, 52), (65, 132), (200, 300), (513, 1000)]
+SHAPES_U8 = [(1, 16), (3, 32), (37, 48), (65, 144), (200, 304), (513, 1008), (70, 1040)]
+
+
+def tma_ctx(ndev=1, **opts):
+    require_gpu()
+    c = S.Context(ndev, devices=[0] * ndev)
+    for k, v in opts.items():
+        c.set_option(k, v)
+    return c
+
+
+@pytest.mark.parametrize("shape", SHAPES_F32)
+@pytest.mark.parametrize("tma", [1, 0])
+def test_tma_f32_modes(shape, tma):
+    c = tma_ctx(mo_tma=tma, block_threads=128)
+    try:
+        x = I.image_f32(I.SEED_GAUSS, *shape)
+        m = S.Matrix.from_numpy(c, x)
+        before = c.counter("tma_launches")
+        for src, kind, d, bnd, nv in ((A.gaussian5(), O.OS_GAUSS5, 2, S.NEAREST, 0.0),
+                                      (A.gaussian5(), O.OS_GAUSS5, 2, S.NEUTRAL, 0.0),
+                                      (A.BOX3, O.OS_BOX3, 1, S.NEAREST, 0.0),
+                                      (A.SHIFTX, O.OS_SHIFT_X, 1, S.NEUTRAL, 7.0),
+                                      (A.SHIFTY, O.OS_SHIFT_Y, 1, S.NEAREST, 0.0)):
+            mo = S.MapOverlap(c, src, S.F32, S.F32, d, bnd, nv)
+            got = mo(m).to_numpy()
+            ref = O.mapoverlap2d(kind, x, d, O.OB_NEAREST if bnd == S.NEAREST else O.OB_NEUTRAL, nv)
+            assert np.array_equal(got, ref), (src, shape)
+        # rows of 16-byte multiples go through TMA when it is on
+        assert c.counter("tma_launches") - before == (5 if tma and (shape[1] * 4) % 16 == 0 else 0)
+    finally:
+        c.finalize()
+
+
+@pytest.mark.parametrize("shape", SHAPES_U8)
+@pytest.mark.parametrize("rh", [0, 4])
+def test_tma_u8(shape, rh):
+    c = tma_ctx(mo_rh=rh) if rh else tma_ctx()
+    try:
+        x = I.image_u8(I.SEED_SOBEL, *shape)
+        m = S.Matrix.from_numpy(c, x)
+        before = c.counter("tma_launches")
+        for src in (A.SOBEL, A.SOBEL_SEPARABLE):
+            sob = S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            assert np.array_equal(sob(m).to_numpy(), O.mapoverlap2d(O.OS_SOBEL, x, 1, O.OB_NEUTRAL, 0)), src
+        sx = S.MapOverlap(c, A.SHIFTX_U8, S.U8, S.U8, 1, S.NEAREST, 0)
+        assert np.array_equal(sx(m).to_numpy(), O.mapoverlap2d(O.OS_SHIFT_X, x, 1, O.OB_NEAREST, 0))
+        idn = S.MapOverlap(c, A.IDENT2D_U8, S.U8, S.U8, 1, S.NEUTRAL, 0)
+        assert np.array_equal(idn(m).to_numpy(), x)
+        assert c.counter("tma_launches") - before == 4
+    finally:
+        c.finalize()
+
+
+@pytest.mark.parametrize("ndev", [2, 3])
+@pytest.mark.parametrize("dt", ["f32", "u8"])
+def test_tma_overlap_distribution_and_halo_push(ndev, dt):
+    """parts with halo rows (the map starts at the part's first row), iterated
+    stencils whose halos are pushed by the kernel into the neighbours"""
+    c = tma_ctx(ndev)
+    try:
+        if dt == "f32":
+            x = I.image_f32(I.SEED_GAUSS, 301, 260)
+            st = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+            f = lambda r: O.mapoverlap2d(O.OS_GAUSS5, r, 2, O.OB_NEAREST, 0.0)  # noqa: E731
+        else:
+            x = I.image_u8(I.SEED_SOBEL, 301, 272)
+            st = S.MapOverlap(c, A.SOBEL_SEPARABLE, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            f = lambda r: O.mapoverlap2d(O.OS_SOBEL, r, 1, O.OB_NEUTRAL, 0)  # noqa: E731
+        a = S.Matrix.from_numpy(c, x)
+        b = st(a)
+        t = st(b)
+        b2 = st(t)
+        ref = x
+        for _ in range(3):
+            ref = f(ref)
+        assert np.array_equal(b2.to_numpy(), ref)
+        assert c.counter("tma_launches") >= 3 * ndev
+        assert c.counter("halo_push_bytes") > 0
+    finally:
+        c.finalize()
+
+
+def test_sobel_separable_root_step_every_m():
+    """the square-root step of apps.SOBEL_SEPARABLE, cut out of the user function's
+    own text and run as a Map over m = 0 .. 2^21 - 1 (h^2 + v^2 <= 2,080,800 <
+    2^21), against numpy's correctly rounded fp32 root: min(255, (int)sqrtf(m))"""
+    c = tma_ctx()
+    try:
+        src = A.SOBEL_SEPARABLE
+        body = src[src.index("  float fm"):src.index("}", src.index("return (uchar)(m >= 65025"))]
+        assert "rsqrt.approx" in body and "return (uchar)(m >= 65025 ? 255 : r);" in body
+        fn = "uchar root(int m) {\n" + body + "}"
+        n = 1 << 21
+        m = np.arange(n, dtype=np.int32)
+        got = S.Map(c, fn, S.I32, S.U8)(S.Vector.from_numpy(c, m)).to_numpy()
+        ref = np.minimum(np.sqrt(m.astype(np.float32)).astype(np.int64), 255).astype(np.uint8)
+        assert np.array_equal(got, ref)
+    finally:
+        c.finalize()
+
+
+def test_sobel_both_forms_full_image():
+    """8192^2 (the bench's workload): the separable user function and Listing
+    1.5 give the oracle's image bit for bit on row bands incl. both edges"""
+    c = tma_ctx()
+    try:
+        R = Cc = 8192
+        img = I.image_u8(I.SEED_SOBEL, R, Cc)
+        m = S.Matrix.from_numpy(c, img)
+        outs = [S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)(m).to_numpy() for src in (A.SOBEL, A.SOBEL_SEPARABLE)]
+        assert np.array_equal(outs[0], outs[1])
+        for r0 in (0, 4000, R - 64):
+            lo, hi = max(0, r0 - 8), min(R, r0 + 72)
+            ref = O.mapoverlap2d(O.OS_SOBEL, img[lo:hi], 1, O.OB_NEUTRAL, 0)
+            assert np.array_equal(outs[1][r0:r0 + 64], ref[r0 - lo:r0 - lo + 64])
+    finally:
+        c.finalize()
