@@ -286,45 +286,78 @@ skl_combine(const SKL_T* __restrict__ staging, skl_u64 stride, int nrep, SKL_T* 
 // result in place into its own replica - a reduce-scatter with the user's
 // operator in one kernel, no staging copy.  In place is safe: device g writes
 // only its own slice of its own replica, which no other device reads.
-// 512-thread blocks for the peer folds, one chunk per thread and step (40
-// registers; 2 chunks measured slower: 4 replicas 22.6 vs 34.8 us,
-// tools/combine_sweep.py)
+//
+// One pass, no grid-stride loop: thread t of block b owns the SKL_CUNR 16-byte
+// chunks b * SKL_CBLOCK * SKL_CUNR + u * SKL_CBLOCK + t (u < SKL_CUNR), issues
+// every replica's loads of all of them before the first fold (in groups of 4
+// replicas to bound registers) and stores the folded chunks.  Chunk indices are
+// 32-bit (the host checks the count).  The previous grid-stride loop with 64-bit
+// indices and a 64-bit float conversion per chunk executed ~350 instructions
+// per 16-byte chunk (ncu): issue-bound at 2.7 TB/s.
 #ifndef SKL_CBLOCK
 #error "SKL_CBLOCK (kCombineBlock, skl_internal.h) must be defined by the program source"
+#endif
+#ifndef SKL_CUNR
+#define SKL_CUNR 2
 #endif
 struct SklSrcs {
   const SKL_T* p[SKL_CMAXR];
 };
+// fold the SKL_CUNR chunks of this thread over every replica into a[]
 template <int V>
-__device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep, SKL_T* out, skl_u64 n_chunks) {
+__device__ __forceinline__ void skl_combine_fold(const SklSrcs& s, int nrep, unsigned i0, unsigned n_chunks,
+                                                 SklChunk<SKL_T, V> (&a)[SKL_CUNR]) {
   SklOp op;
-  for (skl_u64 i = (skl_u64)blockIdx.x * SKL_CBLOCK + threadIdx.x; i < n_chunks;
-       i += (skl_u64)gridDim.x * SKL_CBLOCK) {
-    SklChunk<SKL_T, V> x[SKL_CMAXR];
 #pragma unroll
-    for (int r = 0; r < SKL_CMAXR; ++r)
-      if (r < nrep) {
-        if (V > 1) x[r].q[0] = skl_ld16(s.p[r] + i * V);
-        else x[r].e[0] = s.p[r][i];
+  for (int g0 = 0; g0 < SKL_CMAXR; g0 += 4) {
+    if (g0 >= nrep) break;
+    SklChunk<SKL_T, V> x[SKL_CUNR][4];
+#pragma unroll
+    for (int u = 0; u < SKL_CUNR; ++u) {
+      const unsigned i = i0 + (unsigned)u * SKL_CBLOCK;
+      if (i < n_chunks) {
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+          if (g0 + j < nrep) {
+            if (V > 1) x[u][j].q[0] = skl_ld16(s.p[g0 + j] + (size_t)i * V);
+            else x[u][j].e[0] = s.p[g0 + j][i];
+          }
       }
-    SklChunk<SKL_T, V> a = x[0];
+    }
 #pragma unroll
-    for (int r = 1; r < SKL_CMAXR; ++r)
-      if (r < nrep) {
+    for (int u = 0; u < SKL_CUNR; ++u)
 #pragma unroll
-        for (int k = 0; k < V; ++k) a.e[k] = op(a.e[k], x[r].e[k]);
-      }
-    if (V > 1) skl_st16(out + i * V, a.q[0]);
-    else out[i] = a.e[0];
+      for (int j = 0; j < 4; ++j)
+        if (g0 + j < nrep) {
+          if (g0 + j == 0) {
+            a[u] = x[u][0];
+          } else {
+#pragma unroll
+            for (int k = 0; k < V; ++k) a[u].e[k] = op(a[u].e[k], x[u][j].e[k]);
+          }
+        }
+  }
+}
+template <int V>
+__device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep, SKL_T* out, unsigned n_chunks) {
+  const unsigned i0 = blockIdx.x * (unsigned)(SKL_CBLOCK * SKL_CUNR) + threadIdx.x;
+  SklChunk<SKL_T, V> a[SKL_CUNR];
+  skl_combine_fold<V>(s, nrep, i0, n_chunks, a);
+#pragma unroll
+  for (int u = 0; u < SKL_CUNR; ++u) {
+    const unsigned i = i0 + (unsigned)u * SKL_CBLOCK;
+    if (i >= n_chunks) break;
+    if (V > 1) skl_st16(out + (size_t)i * V, a[u].q[0]);
+    else out[i] = a[u].e[0];
   }
 }
 extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
 skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
 #if SKL_RVEC > 1
   if (vec) {
-    const skl_u64 nc = n / SKL_RVEC;
+    const unsigned nc = (unsigned)(n / SKL_RVEC);
     skl_combine_peer_run<SKL_RVEC>(s, nrep, out, nc);
-    const skl_u64 t0 = nc * SKL_RVEC;
+    const skl_u64 t0 = (skl_u64)nc * SKL_RVEC;
     if (blockIdx.x == 0 && threadIdx.x < n - t0) {
       SklOp op;
       const skl_u64 i = t0 + threadIdx.x;
@@ -338,7 +371,7 @@ skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
   }
 #endif
   (void)vec;
-  skl_combine_peer_run<1>(s, nrep, out, n);
+  skl_combine_peer_run<1>(s, nrep, out, (unsigned)n);
 }
 
 // The same fold for logical devices sharing one GPU, in ONE launch: bases[h] is
@@ -346,22 +379,15 @@ skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
 // to device e / chunk, whose replica receives the fold (chunk = the block
 // distribution's ceil(units / G) units in elements; a multiple of SKL_RVEC for
 // the 16-byte path).
-#ifndef SKL_CUNR
-#define SKL_CUNR 1
-#endif
-// SKL_CUNR chunks per thread and step: all their replica loads are issued
-// before the first store (the output aliases a replica, so the compiler cannot
-// hoist the next step's loads above this step's stores on its own)
-// Replica of the device owning element e: e / chunk through a float reciprocal
-// (within one of the true quotient for any e < 2^40 and <= 8 devices), fixed by
-// two exact compares - a 64-bit integer division is a ~100-instruction software
-// routine and made this kernel issue-bound - then selected with constant
+// Replica of the device owning chunk i (of V elements; chunk_v = chunk / V):
+// i / chunk_v through a float reciprocal (within one of the true quotient for
+// i < 2^31), fixed by two exact 32-bit compares, then selected with constant
 // indices (the pointer table stays in registers).
-__device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, skl_u64 e, skl_u64 chunk,
-                                                    float inv_chunk) {
-  int o = (int)((float)e * inv_chunk);
-  if ((skl_u64)o * chunk > e) --o;
-  if ((skl_u64)(o + 1) * chunk <= e) ++o;
+__device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, unsigned i, unsigned chunk_v,
+                                                    float inv) {
+  int o = (int)((float)i * inv);
+  if ((unsigned)o * chunk_v > i) --o;
+  if ((unsigned)(o + 1) * chunk_v <= i) ++o;
   o = o < 0 ? 0 : (o > nrep - 1 ? nrep - 1 : o);
   SKL_T* out = const_cast<SKL_T*>(s.p[0]);
 #pragma unroll
@@ -370,60 +396,27 @@ __device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, 
   return out;
 }
 template <int V>
-__device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, skl_u64 n_chunks, skl_u64 chunk) {
-  SklOp op;
-  const float inv_chunk = 1.0f / (float)chunk;
-  const skl_u64 stride = (skl_u64)gridDim.x * SKL_CBLOCK;
-  for (skl_u64 i0 = (skl_u64)blockIdx.x * SKL_CBLOCK + threadIdx.x; i0 < n_chunks; i0 += stride * SKL_CUNR) {
-    SklChunk<SKL_T, V> a[SKL_CUNR];
-    // replicas in groups of 4 (registers for 4, not SKL_CMAXR, replica chunks
-    // per step), folded left to right as each group arrives
+__device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, unsigned n_chunks, unsigned chunk_v) {
+  const unsigned i0 = blockIdx.x * (unsigned)(SKL_CBLOCK * SKL_CUNR) + threadIdx.x;
+  const float inv = 1.0f / (float)chunk_v;
+  SklChunk<SKL_T, V> a[SKL_CUNR];
+  skl_combine_fold<V>(s, nrep, i0, n_chunks, a);
 #pragma unroll
-    for (int g0 = 0; g0 < SKL_CMAXR; g0 += 4) {
-      if (g0 >= nrep) break;
-      SklChunk<SKL_T, V> x[SKL_CUNR][4];
-#pragma unroll
-      for (int u = 0; u < SKL_CUNR; ++u) {
-        const skl_u64 i = i0 + (skl_u64)u * stride;
-        if (i < n_chunks) {
-#pragma unroll
-          for (int j = 0; j < 4; ++j)
-            if (g0 + j < nrep) {
-              if (V > 1) x[u][j].q[0] = skl_ld16(s.p[g0 + j] + i * V);
-              else x[u][j].e[0] = s.p[g0 + j][i];
-            }
-        }
-      }
-#pragma unroll
-      for (int u = 0; u < SKL_CUNR; ++u)
-#pragma unroll
-        for (int j = 0; j < 4; ++j)
-          if (g0 + j < nrep) {
-            if (g0 + j == 0) {
-              a[u] = x[u][0];
-            } else {
-#pragma unroll
-              for (int k = 0; k < V; ++k) a[u].e[k] = op(a[u].e[k], x[u][j].e[k]);
-            }
-          }
-    }
-#pragma unroll
-    for (int u = 0; u < SKL_CUNR; ++u) {
-      const skl_u64 i = i0 + (skl_u64)u * stride;
-      if (i >= n_chunks) break;
-      SKL_T* out = skl_combine_owner(s, nrep, i * V, chunk, inv_chunk);
-      if (V > 1) skl_st16(out + i * V, a[u].q[0]);
-      else out[i] = a[u].e[0];
-    }
+  for (int u = 0; u < SKL_CUNR; ++u) {
+    const unsigned i = i0 + (unsigned)u * SKL_CBLOCK;
+    if (i >= n_chunks) break;
+    SKL_T* out = skl_combine_owner(s, nrep, i, chunk_v, inv);
+    if (V > 1) skl_st16(out + (size_t)i * V, a[u].q[0]);
+    else out[i] = a[u].e[0];
   }
 }
 extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
 skl_combine_all(const SklSrcs s, int nrep, skl_u64 n, skl_u64 chunk, int vec) {
 #if SKL_RVEC > 1
   if (vec) {
-    const skl_u64 nc = n / SKL_RVEC;
-    skl_combine_all_run<SKL_RVEC>(s, nrep, nc, chunk);
-    const skl_u64 t0 = nc * SKL_RVEC;
+    const unsigned nc = (unsigned)(n / SKL_RVEC);
+    skl_combine_all_run<SKL_RVEC>(s, nrep, nc, (unsigned)(chunk / SKL_RVEC));
+    const skl_u64 t0 = (skl_u64)nc * SKL_RVEC;
     if (blockIdx.x == 0 && threadIdx.x < n - t0) {
       SklOp op;
       const skl_u64 i = t0 + threadIdx.x;
@@ -431,11 +424,11 @@ skl_combine_all(const SklSrcs s, int nrep, skl_u64 n, skl_u64 chunk, int vec) {
 #pragma unroll
       for (int r = 1; r < SKL_CMAXR; ++r)
         if (r < nrep) a = op(a, s.p[r][i]);
-      skl_combine_owner(s, nrep, i, chunk, 1.0f / (float)chunk)[i] = a;
+      skl_combine_owner(s, nrep, (unsigned)i, (unsigned)chunk, 1.0f / (float)chunk)[i] = a;
     }
     return;
   }
 #endif
   (void)vec;
-  skl_combine_all_run<1>(s, nrep, n, chunk);
+  skl_combine_all_run<1>(s, nrep, (unsigned)n, (unsigned)chunk);
 }

@@ -150,7 +150,8 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
         defs += "#define SKL_LBW " + std::to_string(ctx->scan_lbw) + "\n";
         defs += "#define SKL_SUB " + std::to_string(s->scan_sub) + "\n";
       }
-      if (ctx->combine_unroll) defs += "#define SKL_CUNR " + std::to_string(ctx->combine_unroll) + "\n";
+      s->cunr = ctx->combine_unroll > 0 ? ctx->combine_unroll : 2;
+      defs += "#define SKL_CUNR " + std::to_string(s->cunr) + "\n";
       body = user + kernel_template("common.cuh") + kernel_template("op.cuh") +
              kernel_template("reduce.cuh") + (kind == K_SCAN ? kernel_template("scan.cuh") : "");
       break;
@@ -616,8 +617,9 @@ void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* d
   }
   unsigned long long n = nelem;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock),
-                                                           (size_t)ctx->D(g).sm_count * 4));
+  if (ceil_div(nelem, per) >= (1ull << 31)) fail(SKL_ERR_INVALID_ARG, "copy(+) combine: slice too large");
+  // one pass: every thread folds s->cunr chunks (no grid-stride loop)
+  const size_t grid = std::max<size_t>(1, ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock * (size_t)s->cunr));
   void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec};
   launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(kCombineBlock), 0, args);
 }
@@ -640,8 +642,8 @@ void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t 
   }
   unsigned long long n = nelem, ch = chunk_elems;
   const size_t per = vec ? 16 / st : 1;
-  const size_t grid = std::max<size_t>(1, std::min<size_t>(ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock),
-                                                           (size_t)ctx->D(g).sm_count * 4));
+  if (ceil_div(nelem, per) >= (1ull << 31)) fail(SKL_ERR_INVALID_ARG, "copy(+) combine: container too large");
+  const size_t grid = std::max<size_t>(1, ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock * (size_t)s->cunr));
   void* args[] = {(void*)&sp, &nrep, &n, &ch, &vec};
   launch(ctx, g, s->prog, "skl_combine_all", dim3((unsigned)grid), dim3(kCombineBlock), 0, args);
 }
@@ -1028,7 +1030,21 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       const bool tma = (ctx->mo_ws || (ctx->mo_tma && !ctx->mo_persist)) && vec_ok &&
                        encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
                                        (size_t)(s->mo_th + 2 * s->d), &ushift);
-      if (tma && !ctx->mo_ws) {
+      if (tma && !ctx->mo_ws && ctx->mo_tma == 2) {
+        // resident blocks walk runs of tiles down the tile columns, the next
+        // tile's TMA copy in flight while f runs on the current one (skl_mo2d_tp)
+        const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;
+        const size_t smem = 2 * ((tile_bytes + 127) / 128 * 128) + 128;
+        int tiles_y = (int)grid.y, ntiles = (int)(grid.x * grid.y);
+        const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_mo2d_tp", s->block, smem));
+        const size_t pgrid = std::min((size_t)ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
+        int per_block = (int)ceil_div((size_t)ntiles, pgrid);
+        const size_t nblk = ceil_div((size_t)ntiles, (size_t)per_block);
+        void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
+                         &pu, &pd, &hd, &fix, &ushift, &tiles_y, &ntiles, &per_block};
+        launch(ctx, g, s->prog, "skl_mo2d_tp", dim3((unsigned)nblk), dim3(s->block), smem, targs);
+        ctx->n_tma++;
+      } else if (tma && !ctx->mo_ws) {
         // one tile per block, staged by one TMA copy (skl_mo2d_t)
         void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
                          &pu, &pd, &hd, &fix, &ushift};

@@ -145,7 +145,7 @@ struct Ctx {
   int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
   int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
-  int combine_unroll = 0;      // copy(+) -> block fold: chunks per thread and step (0 = 1)
+  int combine_unroll = 0;      // copy(+) -> block folds: 16-byte chunks per thread (0 = 2)
   int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
                                // (0 = staged exchange then fold, 2 = one kernel per device even on one GPU)
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
@@ -270,7 +270,7 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
 constexpr int kXferMaxSegs = 32;
 // threads per block of the peer folds (skl_combine_peer / skl_combine_all); the
 // Reduce/Scan programs are compiled with SKL_CBLOCK set to this value
-constexpr int kCombineBlock = 512;
+constexpr int kCombineBlock = 256;
 struct XferSeg {
   const void* src;
   void* dst;
@@ -319,6 +319,7 @@ struct Skel {
   int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0;
   bool mo_1d = false;
   int scan_ch = 0;   // Scan: 16-byte chunks per thread (0 = generic path)
+  int cunr = 2;      // Reduce/Scan programs: 16-byte chunks per thread of the copy(+) folds (SKL_CUNR)
   int scan_sub = 4;  // Scan: tiles per look-back chunk (vector path)
   int scan_variant = 0;
   int scan_fstride = 16;  // Scan: status word spacing in 8-byte units

@@ -1,5 +1,6 @@
 """GPU parity tests for the TMA-staged one-tile-per-block 2-D MapOverlap kernel
-(skl_mo2d_t, option mo_tma, the default where a tensor map describes the part;
+(skl_mo2d_t, option mo_tma, the default where a tensor map describes the part,
+and its pipelined persistent form skl_mo2d_tp, mo_tma=2;
 DESIGN.md 6.3): one cp.async.bulk.tensor copy stages a block's window, cells
 outside the matrix are zero-filled by the copy engine and patched for NEAREST
 and non-zero NEUTRAL (A20).  Bit-exact against the oracle at sizes
@@ -34,7 +35,7 @@ def tma_ctx(ndev=1, **opts):
 
 
 @pytest.mark.parametrize("shape", SHAPES_F32)
-@pytest.mark.parametrize("tma", [1, 0])
+@pytest.mark.parametrize("tma", [1, 0, 2])
 def test_tma_f32_modes(shape, tma):
     c = tma_ctx(mo_tma=tma, block_threads=128)
     try:
@@ -57,9 +58,9 @@ def test_tma_f32_modes(shape, tma):
 
 
 @pytest.mark.parametrize("shape", SHAPES_U8)
-@pytest.mark.parametrize("rh", [0, 4])
-def test_tma_u8(shape, rh):
-    c = tma_ctx(mo_rh=rh) if rh else tma_ctx()
+@pytest.mark.parametrize("rh,tma", [(0, 1), (4, 1), (0, 2), (4, 2)])
+def test_tma_u8(shape, rh, tma):
+    c = tma_ctx(mo_rh=rh, mo_tma=tma) if rh else tma_ctx(mo_tma=tma)
     try:
         x = I.image_u8(I.SEED_SOBEL, *shape)
         m = S.Matrix.from_numpy(c, x)
@@ -78,10 +79,11 @@ def test_tma_u8(shape, rh):
 
 @pytest.mark.parametrize("ndev", [2, 3])
 @pytest.mark.parametrize("dt", ["f32", "u8"])
-def test_tma_overlap_distribution_and_halo_push(ndev, dt):
+@pytest.mark.parametrize("tma", [1, 2])
+def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
     """parts with halo rows (the map starts at the part's first row), iterated
     stencils whose halos are pushed by the kernel into the neighbours"""
-    c = tma_ctx(ndev)
+    c = tma_ctx(ndev, mo_tma=tma)
     try:
         if dt == "f32":
             x = I.image_f32(I.SEED_GAUSS, 301, 260)
