@@ -202,8 +202,7 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "mo_ws") {
       c->mo_ws = value ? 1 : 0;
     } else if (k == "mo_tma") {
-      if (value < 0 || value > 2) fail(SKL_ERR_INVALID_ARG, "mo_tma in [0,2]");
-      c->mo_tma = (int)value;
+      c->mo_tma = value ? 1 : 0;
     } else if (k == "mo_ws_stages") {
       if (value < 2 || value > 8) fail(SKL_ERR_INVALID_ARG, "mo_ws_stages in [2,8]");
       c->mo_ws_stages = (int)value;

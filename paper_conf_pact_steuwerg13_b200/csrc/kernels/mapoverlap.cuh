@@ -301,61 +301,6 @@ skl_mo2d_t(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, lon
   skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
 }
 
-// TMA staging, pipelined (mo_tma=2): resident blocks each walk a run of tiles
-// down a column of the tile grid (the halo rows a tile re-reads were just loaded
-// for the tile above it: L2 hits), with two shared-memory buffers: while the
-// block applies f to tile k, one thread has already issued the TMA copy of tile
-// k+1 into the other buffer, so the tile load latency (29 % of the warps' stall
-// samples of skl_mo2d_t on the Gaussian, ncu) overlaps the arithmetic.
-extern "C" __global__ void __launch_bounds__(SKL_BLOCK, 1)
-skl_mo2d_tp(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, long in_row0, long out_row0, long R,
-            long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok, SKL_TOUT* __restrict__ push_up,
-            SKL_TOUT* __restrict__ push_down, long hd, int fix, int ushift, int tiles_y, int ntiles, int per_block) {
-  extern __shared__ __align__(128) unsigned char skl_mo_dyn[];
-  __shared__ __align__(8) unsigned long long bars[2];
-  constexpr unsigned TB = SKL_SROWS * SKL_PITCH * (unsigned)sizeof(SKL_TIN);
-  constexpr unsigned TS = (TB + 127u) / 128u * 128u;
-  const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
-  const unsigned raw = (unsigned)__cvta_generic_to_shared(skl_mo_dyn);
-  const unsigned base = (raw + 127u) & ~127u;
-  const unsigned b0 = (unsigned)__cvta_generic_to_shared(bars);
-  const int t0 = (int)blockIdx.x * per_block;
-  const int t1 = min(ntiles, t0 + per_block);
-  if (t0 >= t1) return;
-  auto issue = [&](int t, int s) {
-    const int r0 = G.rb + (t % tiles_y) * SKL_TH, c0 = (t / tiles_y) * SKL_TW;
-    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(b0 + 8u * s), "n"(TB) : "memory");
-    asm volatile(
-        "cp.async.bulk.tensor.2d.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3}], [%4];" ::
-            "r"(base + TS * s),
-        "l"((unsigned long long)&tmap), "r"(((c0 - SKL_A) * (int)sizeof(SKL_TIN)) >> ushift),
-        "r"(r0 - SKL_D - G.irow0), "r"(b0 + 8u * s)
-        : "memory");
-  };
-  if (threadIdx.x == 0) {
-    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b0) : "memory");
-    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b0 + 8u) : "memory");
-    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-    issue(t0, 0);
-  }
-  __syncthreads();
-  for (int t = t0, k = 0; t < t1; ++t, ++k) {
-    const int s = k & 1;
-    // the other buffer was last read by tile k-1, finished at the barrier below
-    if (threadIdx.x == 0 && t + 1 < t1) issue(t + 1, s ^ 1);
-    skl_mbar_wait(b0 + 8u * s, (unsigned)(k >> 1) & 1u);
-    SKL_TIN* tile = (SKL_TIN*)(skl_mo_dyn + (base - raw) + TS * s);
-    const int r0 = G.rb + (t % tiles_y) * SKL_TH, c0 = (t / tiles_y) * SKL_TW;
-    const bool border =
-        fix && (r0 - SKL_D < 0 || r0 + SKL_TH + SKL_D > G.Ri || c0 - SKL_A < 0 || c0 + SKL_TW + SKL_A > G.Ci);
-    if (border) skl_mo_fix<SKL_BLOCK>(tile, G, r0, c0, neutral);
-    skl_mo_apply(tile, out, G, r0, c0, vec_ok, push_up, push_down);
-    // generic-proxy writes of the patch are ordered before the next TMA write
-    if (border) asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
-    __syncthreads();
-  }
-}
-
 // Persistent variant: a grid of resident blocks walks the tiles (t = blockIdx.x,
 // + gridDim.x, ...) with two shared-memory buffers, staging tile k+1 while
 // applying f to tile k, so the load latency of a tile hides behind the

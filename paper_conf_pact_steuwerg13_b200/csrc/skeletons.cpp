@@ -56,6 +56,9 @@ std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
 }
 
 std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
+std::string mo_rows_defs(int rh, int th) {
+  return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n";
+}
 
 // Scratch buffer per (skeleton, device), grown on demand.
 void* scratch(Skel* s, std::map<int, Scratch>& m, int g, size_t bytes, bool zero) {
@@ -178,35 +181,37 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       if (neutral) std::memcpy(s->neutral.data(), neutral, si);
       const int epc = (int)(16 / si);
       const int A = (int)ceil_div((size_t)d, (size_t)epc) * epc;
-      int cw, rh, tw, th;
-      // default register block: one 16-byte-wide run of outputs per row; 2 rows
-      // for byte images, 8 rows for wider elements (swept on B200, tools/sweep.py
-      // mo, profiles/sweeps/sweep15-17: Sobel u8 0.090 ms at 2 rows / 64
-      // registers; Gaussian f32 0.19 -> 0.146-0.159 ms at 8 rows / <= 128 registers)
-      cw = (int)(16 / std::min<size_t>(so, 16) > 0 ? 16 / std::min<size_t>(so, 16) : 1);
-      rh = si >= 4 ? 8 : 2;
+      // default register block: one 16-byte-wide run of outputs per row; 8 rows
+      // for wider elements, and for byte images 4 rows unless the function then
+      // spills at the 64-register budget (checked after compiling, below: then
+      // 2 rows).  Swept on B200 (tools/mo_probe.py, profiles/sweeps): identity u8
+      // 30.8 -> 26.6 us at 4 rows, the separable Sobel 75.9 -> 72.7 us, while
+      // Listing 1.5's Sobel (IEEE sqrtf subroutine) spills at 4 rows (77 -> 92 us);
+      // Gaussian f32 at 8 rows / <= 128 registers.
+      int cw = (int)(16 / std::min<size_t>(so, 16) > 0 ? 16 / std::min<size_t>(so, 16) : 1);
+      int rh = si >= 4 ? 8 : (si == 1 ? 4 : 2);
       if (ctx->mo_cw > 0) cw = ctx->mo_cw;  // register block per thread (tuning knobs)
       if (ctx->mo_rh > 0) rh = ctx->mo_rh;
+      s->mo_auto_rh = ctx->mo_rh == 0 && si == 1;
       if ((cw * (int)si) % 16 != 0 && (16 % (cw * (int)si)) != 0)
         fail(SKL_ERR_INVALID_ARG, "mo_cw x element size must divide or be a multiple of 16 bytes");
       const int nthr = ctx->block_threads;
-      tw = 32 * cw;
+      const int tw = 32 * cw;
       const int rows_thr = nthr / 32;
-      th = rows_thr * rh;
+      int th = rows_thr * rh;
       while (rh > 1 && (size_t)(th + 2 * d) * (size_t)(tw + 2 * A) * si > 44 * 1024) {
         rh /= 2;
         th = rows_thr * rh;
       }
       s->mo_tw = tw;
-      s->mo_th = th;
       s->mo_a = A;
       s->mo_pitch = tw + 2 * A;
+      s->mo_cw = cw;
       defs += "#define SKL_TIN " + tname(ctx, tin) + "\n#define SKL_TOUT " + tname(ctx, tout) + "\n";
       defs += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(boundary) + "\n";
       defs += "#define SKL_A " + std::to_string(A) + "\n";
       defs += "#define SKL_PITCH " + std::to_string(tw + 2 * A) + "\n";
-      defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_TH " + std::to_string(th) + "\n";
-      defs += "#define SKL_CW " + std::to_string(cw) + "\n#define SKL_RH " + std::to_string(rh) + "\n";
+      defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_CW " + std::to_string(cw) + "\n";
       defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n#define SKL_SO " + std::to_string(so) + "\n";
       defs += "#define SKL_MO1D 0\n";
       // resident blocks per SM the register allocation must allow (default: 64
@@ -219,6 +224,10 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       const int wsminb =
           ctx->mo_ws_minb > 0 ? ctx->mo_ws_minb : std::max(1, 65536 / ((nthr + 32) * (si >= 4 ? 128 : 64)));
       defs += "#define SKL_WS_MINB " + std::to_string(wsminb) + "\n";
+      s->mo_rh = rh;
+      s->mo_th = th;
+      s->mo_defs = defs;  // the row count goes in last (mo_rows_defs), so it can be halved
+      defs += mo_rows_defs(rh, th);
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;
@@ -228,6 +237,23 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
   }
   std::string log;
   s->prog = compile(ctx, defs + program_source(ctx, body), &log);
+  if (kind == K_MAPOVERLAP && s->mo_auto_rh && !ctx->offline && s->mo_rh > 2) {
+    // byte images: 4 rows per thread unless the function spills at the register
+    // budget (local memory in the TMA tile kernel), then 2 rows
+    cudaFuncAttributes fa{};
+    ctx->set_device(ctx->first_local);
+    cudaKernel_t k = nullptr;
+    if (cudaLibraryGetKernel(&k, s->prog->lib, "skl_mo2d_t") == cudaSuccess &&
+        cudaFuncGetAttributes(&fa, (const void*)k) == cudaSuccess) {
+      if (fa.localSizeBytes > 0) {
+        s->mo_rh /= 2;
+        s->mo_th /= 2;
+        s->prog = compile(ctx, s->mo_defs + mo_rows_defs(s->mo_rh, s->mo_th) + program_source(ctx, body), &log);
+      }
+    } else {
+      (void)cudaGetLastError();
+    }
+  }
   Skel* raw = s.release();
   ctx->skels.insert(raw);
   return raw;
@@ -1030,21 +1056,7 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
       const bool tma = (ctx->mo_ws || (ctx->mo_tma && !ctx->mo_persist)) && vec_ok &&
                        encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
                                        (size_t)(s->mo_th + 2 * s->d), &ushift);
-      if (tma && !ctx->mo_ws && ctx->mo_tma == 2) {
-        // resident blocks walk runs of tiles down the tile columns, the next
-        // tile's TMA copy in flight while f runs on the current one (skl_mo2d_tp)
-        const size_t tile_bytes = (size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si;
-        const size_t smem = 2 * ((tile_bytes + 127) / 128 * 128) + 128;
-        int tiles_y = (int)grid.y, ntiles = (int)(grid.x * grid.y);
-        const int occ = std::max(1, occupancy(ctx, g, s->prog, "skl_mo2d_tp", s->block, smem));
-        const size_t pgrid = std::min((size_t)ntiles, (size_t)ctx->D(g).sm_count * (size_t)occ);
-        int per_block = (int)ceil_div((size_t)ntiles, pgrid);
-        const size_t nblk = ceil_div((size_t)ntiles, (size_t)per_block);
-        void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
-                         &pu, &pd, &hd, &fix, &ushift, &tiles_y, &ntiles, &per_block};
-        launch(ctx, g, s->prog, "skl_mo2d_tp", dim3((unsigned)nblk), dim3(s->block), smem, targs);
-        ctx->n_tma++;
-      } else if (tma && !ctx->mo_ws) {
+      if (tma && !ctx->mo_ws) {
         // one tile per block, staged by one TMA copy (skl_mo2d_t)
         void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
                          &pu, &pd, &hd, &fix, &ushift};

@@ -316,7 +316,9 @@ struct Skel {
   std::map<int, Scratch> scratch_stage;  // per device: cross-device partials / totals
   std::map<int, uint32_t> epoch;    // scan lookback epochs per device
   // MapOverlap tile geometry (compile-time constants of prog)
-  int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0;
+  int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0, mo_rh = 0, mo_cw = 0;
+  bool mo_auto_rh = false;  // byte images: row count chosen after compiling (spill check)
+  std::string mo_defs;      // program defines without the row count
   bool mo_1d = false;
   int scan_ch = 0;   // Scan: 16-byte chunks per thread (0 = generic path)
   int cunr = 2;      // Reduce/Scan programs: 16-byte chunks per thread of the copy(+) folds (SKL_CUNR)

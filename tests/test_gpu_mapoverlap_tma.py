@@ -1,6 +1,5 @@
 """GPU parity tests for the TMA-staged one-tile-per-block 2-D MapOverlap kernel
-(skl_mo2d_t, option mo_tma, the default where a tensor map describes the part,
-and its pipelined persistent form skl_mo2d_tp, mo_tma=2;
+(skl_mo2d_t, option mo_tma, the default where a tensor map describes the part;
 DESIGN.md 6.3): one cp.async.bulk.tensor copy stages a block's window, cells
 outside the matrix are zero-filled by the copy engine and patched for NEAREST
 and non-zero NEUTRAL (A20).  Bit-exact against the oracle at sizes
@@ -35,7 +34,7 @@ def tma_ctx(ndev=1, **opts):
 
 
 @pytest.mark.parametrize("shape", SHAPES_F32)
-@pytest.mark.parametrize("tma", [1, 0, 2])
+@pytest.mark.parametrize("tma", [1, 0])
 def test_tma_f32_modes(shape, tma):
     c = tma_ctx(mo_tma=tma, block_threads=128)
     try:
@@ -58,7 +57,7 @@ def test_tma_f32_modes(shape, tma):
 
 
 @pytest.mark.parametrize("shape", SHAPES_U8)
-@pytest.mark.parametrize("rh,tma", [(0, 1), (4, 1), (0, 2), (4, 2)])
+@pytest.mark.parametrize("rh,tma", [(0, 1), (2, 1), (4, 1), (0, 0)])
 def test_tma_u8(shape, rh, tma):
     c = tma_ctx(mo_rh=rh, mo_tma=tma) if rh else tma_ctx(mo_tma=tma)
     try:
@@ -72,14 +71,14 @@ def test_tma_u8(shape, rh, tma):
         assert np.array_equal(sx(m).to_numpy(), O.mapoverlap2d(O.OS_SHIFT_X, x, 1, O.OB_NEAREST, 0))
         idn = S.MapOverlap(c, A.IDENT2D_U8, S.U8, S.U8, 1, S.NEUTRAL, 0)
         assert np.array_equal(idn(m).to_numpy(), x)
-        assert c.counter("tma_launches") - before == 4
+        assert c.counter("tma_launches") - before == (4 if tma else 0)
     finally:
         c.finalize()
 
 
 @pytest.mark.parametrize("ndev", [2, 3])
 @pytest.mark.parametrize("dt", ["f32", "u8"])
-@pytest.mark.parametrize("tma", [1, 2])
+@pytest.mark.parametrize("tma", [1, 0])
 def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
     """parts with halo rows (the map starts at the part's first row), iterated
     stencils whose halos are pushed by the kernel into the neighbours"""
@@ -101,7 +100,7 @@ def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
         for _ in range(3):
             ref = f(ref)
         assert np.array_equal(b2.to_numpy(), ref)
-        assert c.counter("tma_launches") >= 3 * ndev
+        assert c.counter("tma_launches") >= (3 * ndev if tma else 0)
         assert c.counter("halo_push_bytes") > 0
     finally:
         c.finalize()
