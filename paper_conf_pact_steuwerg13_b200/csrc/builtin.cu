@@ -179,4 +179,46 @@ void launch_xfer_batch(Ctx* ctx, int g, const std::vector<XferSeg>& segs) {
   }
 }
 
+// Device barrier of the IPC transport (ipc.cpp): lane h < world stores the
+// epoch into rank h's signal slot for this rank (a system-scope release over
+// NVLink: everything this GPU wrote before is visible to rank h first), then
+// waits for rank h's epoch in this rank's slot h (acquire).  The grid is one
+// warp; a wait longer than 20 s (globaltimer) raises the host-mapped error flag
+// and returns instead of hanging the GPU.
+struct SklSigSlots {
+  unsigned long long* p[kIpcMaxRanks];
+};
+__global__ void __launch_bounds__(32) skl_ipc_barrier(SklSigSlots peers, int world, int rank,
+                                                      unsigned long long* mine, unsigned long long epoch,
+                                                      unsigned* err) {
+  const int h = threadIdx.x;
+  if (h >= world || h == rank) return;
+  asm volatile("fence.acq_rel.sys;" ::: "memory");
+  asm volatile("st.release.sys.global.u64 [%0], %1;" ::"l"(peers.p[h] + rank), "l"(epoch) : "memory");
+  unsigned long long t0;
+  asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t0));
+  while (true) {
+    unsigned long long v;
+    asm volatile("ld.acquire.sys.global.u64 %0, [%1];" : "=l"(v) : "l"(mine + h) : "memory");
+    if (v >= epoch) break;
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    if (t - t0 > 20000000000ull) {
+      atomicExch(err, 1u);
+      break;
+    }
+    __nanosleep(200);
+  }
+}
+
+void launch_ipc_barrier(Ctx* ctx, unsigned long long* const* peer_slots, int world, int rank,
+                        unsigned long long* mine, unsigned long long epoch, unsigned* err) {
+  SklSigSlots s{};
+  for (int h = 0; h < world && h < kIpcMaxRanks; ++h) s.p[h] = peer_slots[h];
+  Device& D = ctx->D(ctx->first_local);
+  skl_ipc_barrier<<<1, 32, 0, D.stream>>>(s, world, rank, mine, epoch, err);
+  SKL_CUDA(cudaGetLastError());
+  ctx->n_launch++;
+}
+
 }  // namespace skl

@@ -170,7 +170,7 @@ void shm_destroy(Ctx* ctx) {
 }  // namespace
 
 void nccl_get_unique_id(void* out128) {
-  if (shm_mode()) {
+  if (shm_mode() || ipc_requested()) {
     std::random_device rd;
     const std::string nm = "/skl_" + std::to_string((long long)getpid()) + "_" + std::to_string(rd()) +
                            std::to_string(rd());
@@ -189,6 +189,10 @@ void nccl_init(Ctx* ctx, const void* id128) {
     shm_init(ctx, id128);
     return;
   }
+  if (ipc_requested()) {
+    ipc_init(ctx, id128);
+    return;
+  }
   ncclUniqueId id;
   std::memcpy(&id, id128, sizeof(id));
   ctx->set_device(ctx->first_local);
@@ -199,6 +203,7 @@ void nccl_init(Ctx* ctx, const void* id128) {
 
 void nccl_destroy(Ctx* ctx) {
   shm_destroy(ctx);
+  ipc_destroy(ctx);
   if (ctx->nccl_comm) nccl()->commDestroy((ncclComm_t)ctx->nccl_comm);
   ctx->nccl_comm = nullptr;
 }
@@ -245,6 +250,31 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
     for (int g = 0; g < ctx->G; ++g)
       if (!batch[(size_t)g].empty()) launch_xfer_batch(ctx, g, batch[(size_t)g]);
     barrier_streams(ctx);
+    return;
+  }
+  if (ctx->ipc) {
+    // one process per GPU over NVLink peer memory: every rank publishes the
+    // addresses of the moves it sources (host exchange, in list order), the
+    // device barrier makes every source final on every GPU, then each rank
+    // pulls the moves into it with ONE batched copy kernel (peer loads), and a
+    // second barrier keeps the sources alive until every rank has read them
+    const int me = ctx->first_local;
+    std::vector<uint64_t> mine(tr.size(), 0);
+    for (size_t i = 0; i < tr.size(); ++i)
+      if (tr[i].src == me && tr[i].n) mine[i] = (uint64_t)(uintptr_t)p.src(tr[i]);
+    const auto all = ipc_exchange(ctx, mine);
+    ipc_barrier(ctx);
+    std::vector<XferSeg> segs;
+    for (size_t i = 0; i < tr.size(); ++i) {
+      const Transfer& t = tr[i];
+      const size_t bytes = t.n * unit_bytes;
+      if (bytes == 0 || t.dst != me) continue;
+      const void* src = t.src == me ? p.src(t) : ipc_translate(ctx, t.src, all[(size_t)t.src].at(i));
+      if (t.src != me) ctx->p2p += (long long)bytes;
+      segs.push_back(XferSeg{src, p.dst(t), bytes});
+    }
+    if (!segs.empty()) launch_xfer_batch(ctx, me, segs);
+    ipc_barrier(ctx);
     return;
   }
   if (ctx->shm_comm) {

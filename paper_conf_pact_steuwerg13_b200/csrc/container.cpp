@@ -407,6 +407,37 @@ static void combine_to_block(Cont* c) {
   // one process driving every device, each able to load from every replica,
   // <= 8 replicas: one fused exchange + fold kernel per device (peer loads), the
   // fold written in place into the device's own replica
+  if (ctx->ipc && ctx->combine_peer && ctx->xfer_kernel) {
+    // one process per GPU over NVLink: the same fused exchange + fold, every
+    // rank reading the peers' replicas through the IPC mappings
+    const int me = ctx->first_local;
+    const Part& p = c->parts[(size_t)me];
+    const bool ok = p.ptr && p.buf.contains(Range{0, U});
+    const auto all = ipc_exchange(ctx, {(uint64_t)(uintptr_t)p.ptr, (uint64_t)p.buf.lo, ok ? 1u : 0u});
+    bool all_ok = G <= 8;
+    for (int h = 0; h < G; ++h) all_ok = all_ok && all[(size_t)h].at(2) == 1;
+    if (all_ok) {
+      NvtxRange nr("skl_combine_peer");
+      const Range r = block_range(U, G, me);
+      ipc_barrier(ctx);  // every replica is final before any rank reads it
+      if (!r.empty()) {
+        std::vector<const void*> srcs((size_t)G);
+        for (int h = 0; h < G; ++h)
+          srcs[(size_t)h] = (const char*)ipc_translate(ctx, h, all[(size_t)h][0]) + (r.lo - all[(size_t)h][1]) * ub;
+        ctx->p2p += (long long)((size_t)(G - 1) * r.size() * ub);
+        run_combine_peer(c->combine, me, srcs.data(), G, part_ptr(c, me, r.lo), r.size() * c->cols);
+      }
+      ipc_barrier(ctx);  // no rank overwrites its replica while a peer still reads it
+      if (r.empty()) free_part(c, me);
+      c->dist = blk;
+      c->diverged = false;
+      c->dev_valid = true;
+      c->halo_valid = false;
+      c->halo_ready = 0;
+      set_valid(c, blk, false);
+      return;
+    }
+  }
   bool fused = ctx->combine_peer && ctx->xfer_kernel && !ctx->dist_mode && ctx->nlocal == G && G <= 8;
   for (int g = 0; fused && g < G; ++g)
     for (int h = 0; h < G; ++h)

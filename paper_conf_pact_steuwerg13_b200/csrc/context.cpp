@@ -214,7 +214,7 @@ void ctx_destroy(Ctx* c) {
       extern void program_unload(Program*);
       program_unload(kv.second.get());
     }
-  if (c->nccl_comm || c->shm_comm) nccl_destroy(c);
+  if (c->nccl_comm || c->shm_comm || c->ipc) nccl_destroy(c);
   for (auto& d : c->dev) {
     cudaSetDevice(d.phys);
     if (d.ev) cudaEventDestroy(d.ev);
@@ -230,6 +230,9 @@ void* device_alloc(Ctx* ctx, int g, size_t bytes) {
   if (bytes == 0) bytes = 16;
   ctx->set_device(g);
   void* p = nullptr;
+  // one process per GPU over NVLink: every buffer a peer may read or write
+  // lives in the IPC heap (ipc.cpp); it takes precedence over a caller's allocator
+  if (ctx->ipc) return ipc_alloc(ctx, bytes);
   if (ctx->user_alloc) {
     // caller's allocator (e.g. torch's caching allocator), stream-ordered on
     // this device's stream
@@ -243,6 +246,12 @@ void* device_alloc(Ctx* ctx, int g, size_t bytes) {
 void device_free(Ctx* ctx, int g, void* p) {
   if (!p) return;
   ctx->set_device(g);
+  if (ctx->ipc) {
+    // the range is reused by later allocations, whose work is ordered after
+    // this stream's; peers read it only between device barriers
+    ipc_free(ctx, p);
+    return;
+  }
   if (ctx->user_free) {
     // the block may be reused at once on this stream: work other devices'
     // streams queued on it (peer copies) must be ordered before that reuse

@@ -934,8 +934,29 @@ void run_scan(Skel* s, Cont* in, Cont** out) {
 // exactly one producer, the adjacent device) and peer stores are possible.
 static bool plan_halo_push(Ctx* ctx, Cont* o, size_t d, std::vector<void*>& up, std::vector<void*>& down) {
   const int G = ctx->G;
-  if (!ctx->halo_push || ctx->dist_mode || G < 2 || ctx->nlocal != G || d == 0) return false;
-  if (o->dist.kind != DBLOCK) return false;
+  if (!ctx->halo_push || G < 2 || d == 0 || o->dist.kind != DBLOCK) return false;
+  if (ctx->ipc) {
+    // one process per GPU over NVLink: the neighbours' output parts, exchanged
+    // (collective: every rank takes the same decision from the same values)
+    up.assign((size_t)G, nullptr);
+    down.assign((size_t)G, nullptr);
+    const int me = ctx->first_local;
+    const Range want = need_range(o->units(), G, Dist{DOVERLAP, (int)d}, me);
+    const Part& p = o->parts[(size_t)me];
+    const bool ok = p.ptr && p.buf.contains(want);
+    const auto all = ipc_exchange(ctx, {(uint64_t)(uintptr_t)p.ptr, (uint64_t)p.buf.lo, ok ? 1u : 0u});
+    for (int g = 0; g < G; ++g)
+      if (core_range(o->units(), G, o->dist, g).size() < d || all[(size_t)g].at(2) == 0) return false;
+    const Range r = core_range(o->units(), G, o->dist, me);
+    const size_t ub = o->unit_bytes();
+    if (me > 0)
+      up[(size_t)me] = (char*)ipc_translate(ctx, me - 1, all[(size_t)me - 1][0]) + (r.lo - all[(size_t)me - 1][1]) * ub;
+    if (me + 1 < G)
+      down[(size_t)me] =
+          (char*)ipc_translate(ctx, me + 1, all[(size_t)me + 1][0]) + (r.hi - d - all[(size_t)me + 1][1]) * ub;
+    return true;
+  }
+  if (ctx->dist_mode || ctx->nlocal != G) return false;
   up.assign((size_t)G, nullptr);
   down.assign((size_t)G, nullptr);
   for (int g = 0; g < G; ++g) {
@@ -1021,7 +1042,10 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   const bool push = plan_halo_push(ctx, o, (size_t)d, push_up, push_down);
   long hd = push ? (long)d : 0;
   // the pushes overwrite halo units the neighbours may still be reading
-  if (push) barrier_streams(ctx);
+  if (push) {
+    if (ctx->ipc) ipc_barrier(ctx);
+    else barrier_streams(ctx);
+  }
   auto push_ptrs = [&](int g, void** pu, void** pd) {
     *pu = push ? push_up[(size_t)g] : nullptr;
     *pd = push ? push_down[(size_t)g] : nullptr;
@@ -1132,7 +1156,9 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
   mark_written(o);
   if (push) {
     o->halo_ready = (size_t)d;
-    barrier_streams(ctx);  // the neighbours' next reads of their halos wait for the pushes
+    // the neighbours' next reads of their halos wait for the pushes
+    if (ctx->ipc) ipc_barrier(ctx);
+    else barrier_streams(ctx);
   }
   if (ctx->debug_bounds) check_debug_flag(ctx);
 }

@@ -118,6 +118,7 @@ struct Ctx {
   int rank = 0, world = 1;
   void* nccl_comm = nullptr;   // ncclComm_t
   void* shm_comm = nullptr;    // host shared-memory loopback transport (SKL_COMM=shm, tests)
+  void* ipc = nullptr;         // IPC heap + peer mappings + barriers (SKL_COMM=ipc, ipc.cpp)
   std::vector<Device> dev;     // local devices, index g - first_local
   std::vector<TypeInfo> types; // index = skl_type (builtins first)
   std::set<Cont*> conts;
@@ -280,6 +281,18 @@ void launch_xfer_batch(Ctx* ctx, int g, const std::vector<XferSeg>& segs);
 void barrier_streams(Ctx* ctx);  // every local stream waits for every other
 cudaEvent_t event_get(Ctx* ctx, int g);
 void event_put(Ctx* ctx, int g, cudaEvent_t e);
+// one process per GPU over NVLink peer memory (ipc.cpp, SKL_COMM=ipc)
+constexpr int kIpcMaxRanks = 8;
+bool ipc_requested();
+void ipc_init(Ctx* ctx, const void* id128);
+void ipc_destroy(Ctx* ctx);
+void* ipc_alloc(Ctx* ctx, size_t bytes);
+void ipc_free(Ctx* ctx, void* ptr);
+// collective: every rank passes its values, gets every rank's (host barrier)
+std::vector<std::vector<uint64_t>> ipc_exchange(Ctx* ctx, const std::vector<uint64_t>& mine);
+void* ipc_translate(Ctx* ctx, int rank, uint64_t va);  // rank's device address, mapped here
+void ipc_barrier(Ctx* ctx);  // device barrier of every rank's stream (collective)
+void ipc_check(Ctx* ctx);
 // NCCL (dlopen)
 void nccl_get_unique_id(void* out128);
 void nccl_init(Ctx* ctx, const void* id);

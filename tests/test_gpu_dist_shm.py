@@ -1,6 +1,8 @@
 """The one-process-per-GPU mode (skl_init_dist) with 2 and 3 ranks, run as
-processes on one GPU over the shared-memory loopback transport (SKL_COMM=shm;
-NCCL refuses two ranks on one device).  Everything above the transport is the
+processes on one GPU, over the shared-memory loopback transport (SKL_COMM=shm;
+NCCL refuses two ranks on one device) and over the NVLink peer-memory transport
+(SKL_COMM=ipc: IPC heap, in-kernel peer loads/stores, device barriers - on one
+GPU the "peers" are the other processes' allocations of the same device).  Everything above the transport is the
 multi-rank code path: rank-local parts, the canonical transfer lists executed
 by both ranks, cross-rank Reduce / Scan carry-in, halo exchange, copy(+) ->
 block combine, collective host reads.  Each rank checks the oracle."""
@@ -19,9 +21,9 @@ pytestmark = pytest.mark.gpu
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 
 
-def _worker(rank, world, nid, q):
+def _worker(rank, world, nid, q, comm="shm"):
     try:
-        os.environ["SKL_COMM"] = "shm"
+        os.environ["SKL_COMM"] = comm
         sys.path.insert(0, ROOT)
         sys.path.insert(0, os.path.join(ROOT, "tests"))
         import oracle as O
@@ -61,9 +63,23 @@ def _worker(rank, world, nid, q):
         # MapOverlap with a halo exchange between the ranks, twice (halo refresh)
         img = I.image_f32(I.SEED_GAUSS, 97, 61)
         gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+        h0 = ctx.counter("halo_push_bytes")
         g2 = gau(gau(S.Matrix.from_numpy(ctx, img)))
         r1 = O.mapoverlap2d(O.OS_GAUSS5, img, 2, O.OB_NEAREST, 0.0)
         assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
+        if comm == "ipc":   # the first stencil pushed its border rows into the neighbours' halos
+            assert ctx.counter("halo_push_bytes") > h0
+        # iterated Sobel (ping-pong, halos pushed / exchanged every iteration)
+        im8 = I.image_u8(I.SEED_SOBEL, 131, 80)
+        sob = S.MapOverlap(ctx, A.SOBEL_SEPARABLE, S.U8, S.U8, 1, S.NEUTRAL, 0)
+        a8 = S.Matrix.from_numpy(ctx, im8)
+        b8, t8 = sob(a8), None
+        ref8 = O.mapoverlap2d(O.OS_SOBEL, im8, 1, O.OB_NEUTRAL, 0)
+        for _ in range(3):
+            t8 = sob(b8, out=t8)
+            b8, t8 = t8, b8
+            ref8 = O.mapoverlap2d(O.OS_SOBEL, ref8, 1, O.OB_NEUTRAL, 0)
+        assert np.array_equal(b8.to_numpy(), ref8)
         # copy(+) -> block: each rank adds its own events into its replica (LM OSEM)
         N, nev = 10, 3000
         osem = ListModeOSEM(ctx, N)
@@ -90,11 +106,12 @@ def _worker(rank, world, nid, q):
 
 
 @pytest.mark.parametrize("world", [2, 3])
-def test_ranks_on_one_gpu_over_shm(world):
+@pytest.mark.parametrize("comm", ["shm", "ipc"])
+def test_ranks_on_one_gpu(world, comm):
     require_gpu()
     sys.path.insert(0, ROOT)
     from paper_conf_pact_steuwerg13_b200 import skl as S
-    os.environ["SKL_COMM"] = "shm"
+    os.environ["SKL_COMM"] = comm
     try:
         nid = S.Context.nccl_unique_id()
     finally:
@@ -102,7 +119,7 @@ def test_ranks_on_one_gpu_over_shm(world):
     assert nid.startswith(b"/skl_")
     ctxm = mp.get_context("spawn")
     q = ctxm.Queue()
-    procs = [ctxm.Process(target=_worker, args=(r, world, nid, q)) for r in range(world)]
+    procs = [ctxm.Process(target=_worker, args=(r, world, nid, q, comm)) for r in range(world)]
     for p in procs:
         p.start()
     results = {}
