@@ -142,8 +142,10 @@ class Env:
         if self.spmd:
             if gpus not in (1, self.world):
                 raise SystemExit(f"--gpus {gpus} does not match WORLD_SIZE {self.world}")
-            # SKL_COMM=shm (tests): several ranks may share one GPU
-            phys = local_rank % max(1, nvis) if os.environ.get("SKL_COMM", "") == "shm" else local_rank
+            # SKL_COMM=shm or SKL_BENCH_SHARE_GPU=1 (tests of this path on one GPU):
+            # several ranks may share a GPU
+            share = os.environ.get("SKL_COMM", "") == "shm" or os.environ.get("SKL_BENCH_SHARE_GPU") == "1"
+            phys = local_rank % max(1, nvis) if share else local_rank
             if phys >= nvis:
                 raise SystemExit(f"LOCAL_RANK {local_rank} but only {nvis} visible GPU(s)")
             self.G = self.world
@@ -164,8 +166,10 @@ class Env:
 
     @property
     def mode(self):
-        return "one process per GPU (torchrun, skl_init_dist)" if self.spmd else \
-            f"one process driving {self.G} GPU(s) (skl_init)"
+        if self.spmd:
+            comm = os.environ.get("SKL_COMM") or "ipc"
+            return f"one process per GPU (torchrun, skl_init_dist, transport {comm})"
+        return f"one process driving {self.G} GPU(s) (skl_init)"
 
     def barrier(self):
         if self.pg:
@@ -537,7 +541,7 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
     physical = E.G > 1
     c4 = make_context(E) if physical else make_context(E, logical=4)
     G = c4.ndev
-    where = f"{G} physical GPUs (NVLink)" if physical else f"{G} logical devices on one GPU"
+    where = (f"{G} physical GPUs (NVLink), {E.mode}" if physical else f"{G} logical devices on one GPU")
     timer = Timer(c4, E)
     N = 150
     nvox = N ** 3
@@ -563,7 +567,7 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
 
     p0 = c4.counter("p2p_bytes")
     st, seg = timer.run(step_bc, K, W, marks=2)
-    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    moved = E.sum(c4.counter("p2p_bytes") - p0) / (K + W)   # every rank's pulls (one process: all devices)
     v.set_distribution(S.COPY)
     ok = bool(np.array_equal(v.to_numpy(), img)) and moved >= (G - 1) * nvox * 4
     out["redist_block_to_copy"] = {
@@ -595,7 +599,7 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
     c4.set_option("combine_peer", 0)
     p0 = c4.counter("p2p_bytes")
     _, seg0 = timer.run(step_cb, K, W, marks=1)
-    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    moved = E.sum(c4.counter("p2p_bytes") - p0) / (K + W)
     ok = ok and bool(np.all(cv.to_numpy() == 1.0))
     c4.set_option("combine_peer", 1)
     traffic = (G + 1) * nvox * 4                   # fused: G replica slices in, 1 folded slice out
@@ -631,7 +635,7 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
 
     p0 = c4.counter("p2p_bytes")
     st, seg = timer.run(step_halo, K, W, marks=1)
-    moved = (c4.counter("p2p_bytes") - p0) / (K + W)
+    moved = E.sum(c4.counter("p2p_bytes") - p0) / (K + W)
     out["halo_refresh"] = {
         "workload": f"overlap(2) halo refresh of an 8192^2 fp32 Matrix after a stencil, {where} "
                     f"({2 * (G - 1)} transfers of 2 rows)",
@@ -663,8 +667,8 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
             "workload": f"10 x Gaussian 5x5 on {where}, halos "
                         + ("pushed by the stencil kernel into the neighbours (fused)" if push
                            else "refreshed by copies between iterations"),
-            **ms_fields(st), "p2p_bytes_per_step": (c4.counter("p2p_bytes") - p0) / reps,
-            "halo_push_bytes_per_step": (c4.counter("halo_push_bytes") - h0) / reps,
+            **ms_fields(st), "p2p_bytes_per_step": E.sum(c4.counter("p2p_bytes") - p0) / reps,
+            "halo_push_bytes_per_step": E.sum(c4.counter("halo_push_bytes") - h0) / reps,
             "check": "ok" if ok else "FAIL"}
     for x in (a, b, t):
         x.destroy()
@@ -811,7 +815,7 @@ def bench_skeletons(args, E: Env, P: dict, which):
                                         "8 B/element, median of the timed steps", "points": sweep,
                             "check": "ok" if all(v["check"] == "ok" for v in sweep.values()) else "FAIL"}
 
-    if "redist" in which and not E.spmd:
+    if "redist" in which and (not E.spmd or E.world > 1):
         res.update(bench_redist(E, K, W, P))
 
     for it_name in ("gauss_iter", "sobel_iter"):

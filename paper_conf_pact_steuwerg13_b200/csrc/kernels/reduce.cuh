@@ -351,26 +351,35 @@ __device__ __forceinline__ void skl_combine_peer_run(const SklSrcs& s, int nrep,
     else out[i] = a[u].e[0];
   }
 }
+// scalar fold of element i over every replica (heads and tails)
+__device__ __forceinline__ SKL_T skl_combine_one(const SklSrcs& s, int nrep, skl_u64 i) {
+  SklOp op;
+  SKL_T a = s.p[0][i];
+#pragma unroll
+  for (int r = 1; r < SKL_CMAXR; ++r)   // constant indices: the pointers stay in registers
+    if (r < nrep) a = op(a, s.p[r][i]);
+  return a;
+}
+// vec: every source and out share one misalignment; the first `head` elements
+// (up to the next 16-byte boundary) and the tail are folded one by one
 extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
-skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
+skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec, int head) {
 #if SKL_RVEC > 1
   if (vec) {
-    const unsigned nc = (unsigned)(n / SKL_RVEC);
-    skl_combine_peer_run<SKL_RVEC>(s, nrep, out, nc);
-    const skl_u64 t0 = (skl_u64)nc * SKL_RVEC;
-    if (blockIdx.x == 0 && threadIdx.x < n - t0) {
-      SklOp op;
-      const skl_u64 i = t0 + threadIdx.x;
-      SKL_T a = s.p[0][i];
+    const skl_u64 h = (skl_u64)head < n ? (skl_u64)head : n;
+    SklSrcs sv;
 #pragma unroll
-      for (int r = 1; r < SKL_CMAXR; ++r)   // constant indices: the pointers stay in registers
-        if (r < nrep) a = op(a, s.p[r][i]);
-      out[i] = a;
-    }
+    for (int r = 0; r < SKL_CMAXR; ++r) sv.p[r] = s.p[r] + h;
+    const unsigned nc = (unsigned)((n - h) / SKL_RVEC);
+    skl_combine_peer_run<SKL_RVEC>(sv, nrep, out + h, nc);
+    const skl_u64 t0 = h + (skl_u64)nc * SKL_RVEC;
+    if (blockIdx.x == 0 && threadIdx.x < h) out[threadIdx.x] = skl_combine_one(s, nrep, threadIdx.x);
+    if (blockIdx.x == 0 && threadIdx.x < n - t0) out[t0 + threadIdx.x] = skl_combine_one(s, nrep, t0 + threadIdx.x);
     return;
   }
 #endif
   (void)vec;
+  (void)head;
   skl_combine_peer_run<1>(s, nrep, out, (unsigned)n);
 }
 
@@ -379,15 +388,15 @@ skl_combine_peer(const SklSrcs s, int nrep, SKL_T* out, skl_u64 n, int vec) {
 // to device e / chunk, whose replica receives the fold (chunk = the block
 // distribution's ceil(units / G) units in elements; a multiple of SKL_RVEC for
 // the 16-byte path).
-// Replica of the device owning chunk i (of V elements; chunk_v = chunk / V):
-// i / chunk_v through a float reciprocal (within one of the true quotient for
-// i < 2^31), fixed by two exact 32-bit compares, then selected with constant
-// indices (the pointer table stays in registers).
-__device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, unsigned i, unsigned chunk_v,
+// Replica of the device owning element e: e / chunk through a float reciprocal
+// (within one of the true quotient for e < 2^31), fixed by two exact 32-bit
+// compares, then selected with constant indices (the pointer table stays in
+// registers).
+__device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, unsigned e, unsigned chunk,
                                                     float inv) {
-  int o = (int)((float)i * inv);
-  if ((unsigned)o * chunk_v > i) --o;
-  if ((unsigned)(o + 1) * chunk_v <= i) ++o;
+  int o = (int)((float)e * inv);
+  if ((unsigned)o * chunk > e) --o;
+  if ((unsigned)(o + 1) * chunk <= e) ++o;
   o = o < 0 ? 0 : (o > nrep - 1 ? nrep - 1 : o);
   SKL_T* out = const_cast<SKL_T*>(s.p[0]);
 #pragma unroll
@@ -396,18 +405,30 @@ __device__ __forceinline__ SKL_T* skl_combine_owner(const SklSrcs& s, int nrep, 
   return out;
 }
 template <int V>
-__device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, unsigned n_chunks, unsigned chunk_v) {
+__device__ __forceinline__ void skl_combine_all_run(const SklSrcs& s, int nrep, unsigned n_chunks, unsigned chunk) {
   const unsigned i0 = blockIdx.x * (unsigned)(SKL_CBLOCK * SKL_CUNR) + threadIdx.x;
-  const float inv = 1.0f / (float)chunk_v;
+  const float inv = 1.0f / (float)chunk;
   SklChunk<SKL_T, V> a[SKL_CUNR];
   skl_combine_fold<V>(s, nrep, i0, n_chunks, a);
 #pragma unroll
   for (int u = 0; u < SKL_CUNR; ++u) {
     const unsigned i = i0 + (unsigned)u * SKL_CBLOCK;
     if (i >= n_chunks) break;
-    SKL_T* out = skl_combine_owner(s, nrep, i, chunk_v, inv);
-    if (V > 1) skl_st16(out + (size_t)i * V, a[u].q[0]);
-    else out[i] = a[u].e[0];
+    // owners of the chunk's first and last element (chunk = the block
+    // distribution's unit count in elements; it need not be a multiple of V)
+    const unsigned e0 = i * V;
+    SKL_T* o0 = skl_combine_owner(s, nrep, e0, chunk, inv);
+    if (V == 1) {
+      o0[e0] = a[u].e[0];
+      continue;
+    }
+    SKL_T* o1 = skl_combine_owner(s, nrep, e0 + V - 1, chunk, inv);
+    if (o0 == o1) {
+      skl_st16(o0 + e0, a[u].q[0]);
+    } else {  // the chunk straddles two devices' slices
+#pragma unroll
+      for (int k = 0; k < V; ++k) skl_combine_owner(s, nrep, e0 + k, chunk, inv)[e0 + k] = a[u].e[k];
+    }
   }
 }
 extern "C" __global__ void __launch_bounds__(SKL_CBLOCK)
@@ -415,16 +436,11 @@ skl_combine_all(const SklSrcs s, int nrep, skl_u64 n, skl_u64 chunk, int vec) {
 #if SKL_RVEC > 1
   if (vec) {
     const unsigned nc = (unsigned)(n / SKL_RVEC);
-    skl_combine_all_run<SKL_RVEC>(s, nrep, nc, (unsigned)(chunk / SKL_RVEC));
+    skl_combine_all_run<SKL_RVEC>(s, nrep, nc, (unsigned)chunk);
     const skl_u64 t0 = (skl_u64)nc * SKL_RVEC;
     if (blockIdx.x == 0 && threadIdx.x < n - t0) {
-      SklOp op;
       const skl_u64 i = t0 + threadIdx.x;
-      SKL_T a = s.p[0][i];
-#pragma unroll
-      for (int r = 1; r < SKL_CMAXR; ++r)
-        if (r < nrep) a = op(a, s.p[r][i]);
-      skl_combine_owner(s, nrep, (unsigned)i, (unsigned)chunk, 1.0f / (float)chunk)[i] = a;
+      skl_combine_owner(s, nrep, (unsigned)i, (unsigned)chunk, 1.0f / (float)chunk)[i] = skl_combine_one(s, nrep, i);
     }
     return;
   }

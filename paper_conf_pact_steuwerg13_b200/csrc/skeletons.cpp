@@ -636,17 +636,21 @@ void run_combine_peer(Skel* s, int g, const void* const* srcs, int nrep, void* d
     const void* p[8];
   } sp{};
   const size_t st = ctx->type(s->tin).size;
-  int vec = 16 % st == 0 && st < 16 && aligned16(dst);
+  // 16-byte path when every source and the destination share one offset within
+  // 16 bytes (a block slice that starts mid-word: its head is folded scalar)
+  const uintptr_t mis = (uintptr_t)dst & 15u;
+  int vec = 16 % st == 0 && st < 16 && mis % st == 0;
   for (int r = 0; r < nrep; ++r) {
     sp.p[r] = srcs[r];
-    vec = vec && aligned16(srcs[r]);
+    vec = vec && ((uintptr_t)srcs[r] & 15u) == mis;
   }
+  int head = vec ? (int)(((16 - mis) & 15u) / st) : 0;
   unsigned long long n = nelem;
   const size_t per = vec ? 16 / st : 1;
   if (ceil_div(nelem, per) >= (1ull << 31)) fail(SKL_ERR_INVALID_ARG, "copy(+) combine: slice too large");
   // one pass: every thread folds s->cunr chunks (no grid-stride loop)
   const size_t grid = std::max<size_t>(1, ceil_div(ceil_div(nelem, per), (size_t)kCombineBlock * (size_t)s->cunr));
-  void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec};
+  void* args[] = {(void*)&sp, &nrep, &dst, &n, &vec, &head};
   launch(ctx, g, s->prog, "skl_combine_peer", dim3((unsigned)grid), dim3(kCombineBlock), 0, args);
 }
 
@@ -661,7 +665,9 @@ void run_combine_all(Skel* s, int g, const void* const* bases, int nrep, size_t 
     const void* p[8];
   } sp{};
   const size_t st = ctx->type(s->tin).size;
-  int vec = 16 % st == 0 && st < 16 && chunk_elems % (16 / st) == 0;
+  // 16-byte loads whenever the replicas are 16-byte aligned; a chunk that
+  // straddles two devices' slices is stored element by element
+  int vec = 16 % st == 0 && st < 16;
   for (int r = 0; r < nrep; ++r) {
     sp.p[r] = bases[r];
     vec = vec && aligned16(bases[r]);
