@@ -34,9 +34,9 @@ def tma_ctx(ndev=1, **opts):
 
 
 @pytest.mark.parametrize("shape", SHAPES_F32)
-@pytest.mark.parametrize("tma", [1, 0])
-def test_tma_f32_modes(shape, tma):
-    c = tma_ctx(mo_tma=tma, block_threads=128)
+@pytest.mark.parametrize("tma,kt", [(1, 2), (1, 1), (1, 4), (0, 2)])
+def test_tma_f32_modes(shape, tma, kt):
+    c = tma_ctx(mo_tma=tma, mo_kt=kt, block_threads=128)
     try:
         x = I.image_f32(I.SEED_GAUSS, *shape)
         m = S.Matrix.from_numpy(c, x)
@@ -57,9 +57,9 @@ def test_tma_f32_modes(shape, tma):
 
 
 @pytest.mark.parametrize("shape", SHAPES_U8)
-@pytest.mark.parametrize("rh,tma", [(0, 1), (2, 1), (4, 1), (0, 0)])
-def test_tma_u8(shape, rh, tma):
-    c = tma_ctx(mo_rh=rh, mo_tma=tma) if rh else tma_ctx(mo_tma=tma)
+@pytest.mark.parametrize("rh,tma,kt", [(0, 1, 2), (2, 1, 1), (4, 1, 3), (0, 0, 2)])
+def test_tma_u8(shape, rh, tma, kt):
+    c = tma_ctx(mo_rh=rh, mo_tma=tma, mo_kt=kt) if rh else tma_ctx(mo_tma=tma, mo_kt=kt)
     try:
         x = I.image_u8(I.SEED_SOBEL, *shape)
         m = S.Matrix.from_numpy(c, x)

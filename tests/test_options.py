@@ -10,7 +10,7 @@ from paper_conf_pact_steuwerg13_b200 import skl as S
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 VALID = {"ap_tile": 2, "scan_chunks": 8, "mo_ws_stages": 3, "ap_bk": 32, "block_threads": 128,
-         "scan_variant": 6, "combine_peer": 2, "combine_unroll": 4}
+         "scan_variant": 6, "combine_peer": 2, "combine_unroll": 4, "mo_kt": 3}
 
 
 def documented_keys():
