@@ -140,7 +140,8 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * where TMA can describe the tile: 16-byte aligned rows, staged row <= 256
  * units of up to 8 bytes, <= 256 rows; 0 = per-thread cp.async staging;
  * default 1), "mo_kt" (TMA kernel: tiles per block, stacked vertically, all
- * copies issued when the block starts; 1..4, default 2),
+ * copies issued when the block starts; 1..4, or 0 = automatic: 2 for functions
+ * needing >= 64 registers, else 1; default 0),
  * "mo_ws" (1 = 2-D MapOverlap tiles are staged by a TMA producer warp into a
  * ring of "mo_ws_stages" shared-memory buffers consumed by the other warps of
  * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged

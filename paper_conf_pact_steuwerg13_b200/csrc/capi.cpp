@@ -204,7 +204,7 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "mo_tma") {
       c->mo_tma = value ? 1 : 0;
     } else if (k == "mo_kt") {
-      if (value < 1 || value > 4) fail(SKL_ERR_INVALID_ARG, "mo_kt in [1,4]");
+      if (value < 0 || value > 4) fail(SKL_ERR_INVALID_ARG, "mo_kt in [0,4]");
       c->mo_kt = (int)value;
     } else if (k == "mo_ws_stages") {
       if (value < 2 || value > 8) fail(SKL_ERR_INVALID_ARG, "mo_ws_stages in [2,8]");

@@ -214,8 +214,6 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_CW " + std::to_string(cw) + "\n";
       defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n#define SKL_SO " + std::to_string(so) + "\n";
       defs += "#define SKL_MO1D 0\n";
-      s->mo_kt = ctx->mo_kt;
-      defs += "#define SKL_MO_KT " + std::to_string(s->mo_kt) + "\n";
       // resident blocks per SM the register allocation must allow (default: 64
       // registers per thread for byte images - 87 registers halved the Sobel
       // occupancy and cost 30 % - and 128 for wider elements)
@@ -1089,13 +1087,30 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                        encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
                                        (size_t)(s->mo_th + 2 * s->d), &ushift);
       if (tma && !ctx->mo_ws) {
-        // s->mo_kt vertically stacked tiles per block, each staged by one TMA copy
-        // issued up front (skl_mo2d_t)
+        // kt vertically stacked tiles per block, each staged by one TMA copy
+        // issued up front (skl_mo2d_t).  Default (mo_kt = 0): 2 tiles when the
+        // function is heavy (>= 64 registers: the tile wait is worth hiding behind
+        // its arithmetic), else 1 (more, smaller blocks for light functions).
+        // B200 (tools/mo_probe.py): Gaussian 127 -> 117 us and separable Sobel
+        // 69.6 -> 65.6 us at 2 tiles; identity u8 26.7 us at 1 vs 28.7 at 2.
+        int kt = ctx->mo_kt;
+        if (kt == 0) {
+          if (s->mo_regs == 0) {
+            cudaFuncAttributes fa{};
+            cudaKernel_t kk = nullptr;
+            if (cudaLibraryGetKernel(&kk, s->prog->lib, "skl_mo2d_t") == cudaSuccess &&
+                cudaFuncGetAttributes(&fa, (const void*)kk) == cudaSuccess)
+              s->mo_regs = fa.numRegs;
+            else
+              (void)cudaGetLastError();
+          }
+          kt = s->mo_regs >= 64 ? 2 : 1;
+        }
         const size_t ts = ((size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si + 127) / 128 * 128;
-        const size_t smem = s->mo_kt > 1 ? (size_t)s->mo_kt * ts + 128 : 0;
-        const dim3 tgrid(grid.x, (unsigned)ceil_div(r.size(), (size_t)s->mo_th * (size_t)s->mo_kt));
+        const size_t smem = (size_t)kt * ts + 128;
+        const dim3 tgrid(grid.x, (unsigned)ceil_div(r.size(), (size_t)s->mo_th * (size_t)kt));
         void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
-                         &pu, &pd, &hd, &fix, &ushift};
+                         &pu, &pd, &hd, &fix, &ushift, &kt};
         launch(ctx, g, s->prog, "skl_mo2d_t", tgrid, dim3(s->block), smem, targs);
         ctx->n_tma++;
       } else if (tma) {

@@ -139,7 +139,7 @@ struct Ctx {
   int mo_minb = 0;             // MapOverlap min resident blocks per SM (0 = 64-register cap)
   int mo_persist = 0;          // MapOverlap 2-D: persistent blocks, double-buffered tiles
   int mo_tma = 1;              // MapOverlap 2-D: one TMA copy stages a block's tile (skl_mo2d_t)
-  int mo_kt = 2;               //   tiles per block (stacked vertically, all copies issued up front)
+  int mo_kt = 0;               //   tiles per block (stacked vertically, copies issued up front; 0 = auto)
   int mo_ws = 0;               // MapOverlap 2-D: TMA producer warp + consumer warps (skl_mo2d_ws)
   int mo_ws_stages = 4;        //   shared-memory ring depth
   int mo_ws_minb = 0;          //   resident blocks per SM the registers must allow (0 = auto)
@@ -330,7 +330,8 @@ struct Skel {
   std::map<int, Scratch> scratch_stage;  // per device: cross-device partials / totals
   std::map<int, uint32_t> epoch;    // scan lookback epochs per device
   // MapOverlap tile geometry (compile-time constants of prog)
-  int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0, mo_rh = 0, mo_cw = 0, mo_kt = 1;
+  int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0, mo_rh = 0, mo_cw = 0;
+  int mo_regs = 0;          // registers of the TMA tile kernel (picks the tiles per block)
   bool mo_auto_rh = false;  // byte images: row count chosen after compiling (spill check)
   std::string mo_defs;      // program defines without the row count
   bool mo_1d = false;
