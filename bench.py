@@ -3,7 +3,7 @@
 task statement; DESIGN.md §7 "Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,dot_sweep,sobel,gauss,gauss_iter,sobel_iter,redist,
+                    [--skeletons all|none|dot,dot_sweep,sobel,sobel_sep,gauss,gauss_iter,sobel_iter,redist,
                                  scan_i32,scan_f32,lmosem,lmosem_osem,allpairs,mandel_plain]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
@@ -867,14 +867,17 @@ def bench_skeletons(args, E: Env, P: dict, which):
         for x in (a, b, t):
             x.destroy()
 
-    if "sobel" in which or "gauss" in which:
+    if "sobel" in which or "gauss" in which or "sobel_sep" in which:
         R = Cc = 8192
-        for name in ("sobel", "gauss"):
+        for name in ("sobel", "sobel_sep", "gauss"):
             if name not in which:
                 continue
-            if name == "sobel":
+            if name in ("sobel", "sobel_sep"):
+                # Listing 1.5 as printed, and the same operator rewritten by a user
+                # for speed with bit-identical results (apps.SOBEL_SEPARABLE)
                 img = I.image_u8(I.SEED_SOBEL, R, Cc)
-                mo = S.MapOverlap(ctx, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0)
+                mo = S.MapOverlap(ctx, A.SOBEL if name == "sobel" else A.SOBEL_SEPARABLE, S.U8, S.U8, 1,
+                                  S.NEUTRAL, 0)
                 bpp, okind = 2, O.OS_SOBEL
             else:
                 img = I.image_f32(I.SEED_GAUSS, R, Cc)
@@ -899,12 +902,15 @@ def bench_skeletons(args, E: Env, P: dict, which):
             starts = {0, 4000, R - 64} | ({(R + G - 1) // G * (G // 2) - 32} if G > 1 else set())
             for r0 in sorted(starts):
                 blo, bhi = max(0, r0 - 8), min(R, r0 + 72)
-                ref = (O.mapoverlap2d(okind, img[blo:bhi], 1, O.OB_NEUTRAL, 0) if name == "sobel"
+                ref = (O.mapoverlap2d(okind, img[blo:bhi], 1, O.OB_NEUTRAL, 0) if name != "gauss"
                        else O.mapoverlap2d(okind, img[blo:bhi], 2, O.OB_NEAREST, 0.0))
                 a0 = r0 - blo
                 ok &= bool(np.array_equal(full[r0:r0 + 64], ref[a0:a0 + 64]))
-            res[name] = {"workload": f"{'Sobel u8 d=1 NEUTRAL' if name == 'sobel' else 'Gaussian 5x5 f32 d=2 NEAREST'} "
-                                     f"MapOverlap {R}x{Cc}, overlap distribution",
+            desc = {"sobel": "Sobel u8 d=1 NEUTRAL (Listing 1.5 as printed)",
+                    "sobel_sep": "Sobel u8 d=1 NEUTRAL, separable user function with an exact "
+                                 "rsqrt-based integer root (apps.SOBEL_SEPARABLE, bit-identical)",
+                    "gauss": "Gaussian 5x5 f32 d=2 NEAREST"}[name]
+            res[name] = {"workload": f"{desc} MapOverlap {R}x{Cc}, overlap distribution",
                          **ms_fields(st), "elements_per_s": R * Cc / (ms / 1e3),
                          "roofline": roof_hbm(bpp * R * Cc, ms, P, name, ngpu=G), "check": "ok" if ok else "FAIL"}
             res[name]["roofline_issue"] = roof_issue(name, ms, P, sms) if G == 1 else None
@@ -1223,7 +1229,7 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, E, P)
     which = [] if args.skeletons == "none" else (
-        ["mandel_plain", "dot", "dot_sweep", "sobel", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32",
+        ["mandel_plain", "dot", "dot_sweep", "sobel", "sobel_sep", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32",
          "scan_f32", "lmosem", "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))

@@ -272,30 +272,41 @@ __device__ __forceinline__ void skl_mo_fix(SKL_TIN* tile, const SklMoGeo& G, int
   asm volatile("bar.sync 1, %0;" ::"n"(NT) : "memory");
 }
 
-// kt (<= SKL_MO_KTMAX) tiles per block, stacked vertically: thread 0 issues all
-// their TMA copies at once, so the later tiles arrive while f runs on the first
-// (the tile wait was 29 % of the Gaussian's stall samples with one tile per
-// block); every tile has its own buffer (dynamic shared memory) and mbarrier.
-#define SKL_MO_KTMAX 4
+// SKL_MO_KT tiles per block, stacked vertically (compile-time; option mo_kt):
+// thread 0 issues all their TMA copies at once, so the later tiles arrive while
+// f runs on the first (the tile wait was 29 % of the Gaussian's stall samples
+// with one tile per block); every tile has its own buffer and mbarrier.  (A
+// run-time tile count around the inlined f made ptxas spill the byte stencils
+// heavily - 4x slower - so the count is a compile-time constant.)
+#ifndef SKL_MO_KT
+#define SKL_MO_KT 1
+#endif
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK, SKL_MO_MINB)
 skl_mo2d_t(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, long in_row0, long out_row0, long R,
            long C, long r_begin, long r_end, SKL_TIN neutral, int vec_ok, SKL_TOUT* __restrict__ push_up,
-           SKL_TOUT* __restrict__ push_down, long hd, int fix, int ushift, int kt) {
+           SKL_TOUT* __restrict__ push_down, long hd, int fix, int ushift) {
   constexpr unsigned TB = SKL_SROWS * SKL_PITCH * (unsigned)sizeof(SKL_TIN);
   constexpr unsigned TS = (TB + 127u) / 128u * 128u;
-  extern __shared__ __align__(128) unsigned char skl_mo_dyn[];  // kt x TS (+128 to align)
+#if SKL_MO_KT == 1
+  __shared__ __align__(128) SKL_TIN skl_tile0[SKL_SROWS * SKL_PITCH];
+  unsigned char* smem = (unsigned char*)skl_tile0;
+#else
+  extern __shared__ __align__(128) unsigned char skl_mo_dyn[];  // SKL_MO_KT x TS (+128 to align)
   unsigned char* smem = skl_mo_dyn + ((128u - ((unsigned)__cvta_generic_to_shared(skl_mo_dyn) & 127u)) & 127u);
-  __shared__ __align__(8) unsigned long long bars[SKL_MO_KTMAX];
+#endif
+  __shared__ __align__(8) unsigned long long bars[SKL_MO_KT];
   const SklMoGeo G{(int)R, (int)C, (int)r_begin, (int)r_end, (int)in_row0, (int)out_row0, (int)hd};
-  const int rt0 = G.rb + (int)blockIdx.y * (SKL_TH * kt);
+  const int rt0 = G.rb + (int)blockIdx.y * (SKL_TH * SKL_MO_KT);
   const int c0 = (int)blockIdx.x * SKL_TW;
   const unsigned b0 = (unsigned)__cvta_generic_to_shared(bars);
   const unsigned sbase = (unsigned)__cvta_generic_to_shared(smem);
   if (threadIdx.x == 0) {
-    for (int k = 0; k < kt; ++k)
+#pragma unroll
+    for (int k = 0; k < SKL_MO_KT; ++k)
       asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b0 + 8u * k) : "memory");
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-    for (int k = 0; k < kt; ++k) {
+#pragma unroll
+    for (int k = 0; k < SKL_MO_KT; ++k) {
       const int r0 = rt0 + k * SKL_TH;
       if (r0 >= G.re) break;
       asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(b0 + 8u * k), "n"(TB) : "memory");
@@ -309,7 +320,7 @@ skl_mo2d_t(const __grid_constant__ SklTmap tmap, SKL_TOUT* __restrict__ out, lon
   }
   __syncthreads();  // the barriers are initialised before anyone waits on them
 #pragma unroll 1
-  for (int k = 0; k < kt; ++k) {
+  for (int k = 0; k < SKL_MO_KT; ++k) {
     const int r0 = rt0 + k * SKL_TH;
     if (r0 >= G.re) break;
     SKL_TIN* tile = (SKL_TIN*)(smem + TS * k);

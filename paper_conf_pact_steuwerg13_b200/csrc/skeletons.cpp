@@ -56,8 +56,9 @@ std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
 }
 
 std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
-std::string mo_rows_defs(int rh, int th) {
-  return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n";
+std::string mo_rows_defs(int rh, int th, int kt) {
+  return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n#define SKL_MO_KT " +
+         std::to_string(kt) + "\n";
 }
 
 // Scratch buffer per (skeleton, device), grown on demand.
@@ -226,8 +227,9 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       defs += "#define SKL_WS_MINB " + std::to_string(wsminb) + "\n";
       s->mo_rh = rh;
       s->mo_th = th;
-      s->mo_defs = defs;  // the row count goes in last (mo_rows_defs), so it can be halved
-      defs += mo_rows_defs(rh, th);
+      s->mo_kt = ctx->mo_kt > 0 ? ctx->mo_kt : 1;
+      s->mo_defs = defs;  // rows and tiles per block go in last (mo_rows_defs): chosen after compiling
+      defs += mo_rows_defs(rh, th, s->mo_kt);
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;
@@ -237,21 +239,40 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
   }
   std::string log;
   s->prog = compile(ctx, defs + program_source(ctx, body), &log);
-  if (kind == K_MAPOVERLAP && s->mo_auto_rh && !ctx->offline && s->mo_rh > 2) {
-    // byte images: 4 rows per thread unless the function spills at the register
-    // budget (local memory in the TMA tile kernel), then 2 rows
-    cudaFuncAttributes fa{};
-    ctx->set_device(ctx->first_local);
-    cudaKernel_t k = nullptr;
-    if (cudaLibraryGetKernel(&k, s->prog->lib, "skl_mo2d_t") == cudaSuccess &&
-        cudaFuncGetAttributes(&fa, (const void*)k) == cudaSuccess) {
-      if (fa.localSizeBytes > 0) {
-        s->mo_rh /= 2;
-        s->mo_th /= 2;
-        s->prog = compile(ctx, s->mo_defs + mo_rows_defs(s->mo_rh, s->mo_th) + program_source(ctx, body), &log);
-      }
-    } else {
+  if (kind == K_MAPOVERLAP && !ctx->offline) {
+    // geometry chosen after compiling, from the TMA tile kernel's resources
+    // (tools/mo_probe.py on B200):
+    //  * tiles per block (mo_kt = 0): 2 for functions that need >= 64 registers -
+    //    the second tile's copy lands while f runs on the first - else 1
+    //    (Gaussian 127 -> 117 us, separable Sobel 69.6 -> 65.6 us at 2 tiles;
+    //    identity u8 26.7 us at 1 vs 28.7 at 2);
+    //  * byte images: 4 rows per thread unless the kernel then needs more local
+    //    memory than the 16-byte call frame of the IEEE sqrt subroutine (spills
+    //    at the 64-register budget: Listing 1.5's Sobel at 4 rows and 1 tile,
+    //    77 -> 92 us), else 2 rows.
+    auto attrs = [&](cudaFuncAttributes* fa) {
+      ctx->set_device(ctx->first_local);
+      cudaKernel_t k = nullptr;
+      if (cudaLibraryGetKernel(&k, s->prog->lib, "skl_mo2d_t") == cudaSuccess &&
+          cudaFuncGetAttributes(fa, (const void*)k) == cudaSuccess)
+        return true;
       (void)cudaGetLastError();
+      return false;
+    };
+    auto recompile = [&](int rh, int kt) {
+      s->mo_th = s->mo_th / s->mo_rh * rh;
+      s->mo_rh = rh;
+      s->mo_kt = kt;
+      s->prog = compile(ctx, s->mo_defs + mo_rows_defs(rh, s->mo_th, kt) + program_source(ctx, body), &log);
+    };
+    cudaFuncAttributes fa{};
+    if (attrs(&fa)) {
+      const bool heavy = fa.numRegs >= 64;
+      if (ctx->mo_kt == 0 && heavy) {
+        recompile(s->mo_rh, 2);
+        if (!attrs(&fa)) fa.localSizeBytes = 0;
+      }
+      if (s->mo_auto_rh && s->mo_rh > 2 && fa.localSizeBytes > 16) recompile(2, s->mo_kt);
     }
   }
   Skel* raw = s.release();
@@ -1087,30 +1108,14 @@ void run_mapoverlap(Skel* s, Cont* in, Cont** out) {
                        encode_tile_map(&tm, pin, si, (size_t)C, (size_t)in_rows, (size_t)s->mo_pitch,
                                        (size_t)(s->mo_th + 2 * s->d), &ushift);
       if (tma && !ctx->mo_ws) {
-        // kt vertically stacked tiles per block, each staged by one TMA copy
-        // issued up front (skl_mo2d_t).  Default (mo_kt = 0): 2 tiles when the
-        // function is heavy (>= 64 registers: the tile wait is worth hiding behind
-        // its arithmetic), else 1 (more, smaller blocks for light functions).
-        // B200 (tools/mo_probe.py): Gaussian 127 -> 117 us and separable Sobel
-        // 69.6 -> 65.6 us at 2 tiles; identity u8 26.7 us at 1 vs 28.7 at 2.
-        int kt = ctx->mo_kt;
-        if (kt == 0) {
-          if (s->mo_regs == 0) {
-            cudaFuncAttributes fa{};
-            cudaKernel_t kk = nullptr;
-            if (cudaLibraryGetKernel(&kk, s->prog->lib, "skl_mo2d_t") == cudaSuccess &&
-                cudaFuncGetAttributes(&fa, (const void*)kk) == cudaSuccess)
-              s->mo_regs = fa.numRegs;
-            else
-              (void)cudaGetLastError();
-          }
-          kt = s->mo_regs >= 64 ? 2 : 1;
-        }
+        // s->mo_kt vertically stacked tiles per block, each staged by one TMA copy
+        // issued up front (skl_mo2d_t); the count is chosen at creation
+        const int kt = s->mo_kt;
         const size_t ts = ((size_t)(s->mo_th + 2 * s->d) * (size_t)s->mo_pitch * si + 127) / 128 * 128;
-        const size_t smem = (size_t)kt * ts + 128;
+        const size_t smem = kt > 1 ? (size_t)kt * ts + 128 : 0;
         const dim3 tgrid(grid.x, (unsigned)ceil_div(r.size(), (size_t)s->mo_th * (size_t)kt));
         void* targs[] = {(void*)&tm, &pout, &in_row0, &out_row0, &R, &C, &rb, &re, s->neutral.data(), &vec_ok,
-                         &pu, &pd, &hd, &fix, &ushift, &kt};
+                         &pu, &pd, &hd, &fix, &ushift};
         launch(ctx, g, s->prog, "skl_mo2d_t", tgrid, dim3(s->block), smem, targs);
         ctx->n_tma++;
       } else if (tma) {

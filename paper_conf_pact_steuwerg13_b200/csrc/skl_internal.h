@@ -331,7 +331,7 @@ struct Skel {
   std::map<int, uint32_t> epoch;    // scan lookback epochs per device
   // MapOverlap tile geometry (compile-time constants of prog)
   int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0, mo_rh = 0, mo_cw = 0;
-  int mo_regs = 0;          // registers of the TMA tile kernel (picks the tiles per block)
+  int mo_kt = 1;            // TMA tile kernel: tiles per block (SKL_MO_KT)
   bool mo_auto_rh = false;  // byte images: row count chosen after compiling (spill check)
   std::string mo_defs;      // program defines without the row count
   bool mo_1d = false;

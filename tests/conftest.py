@@ -12,6 +12,13 @@ GOLDEN = os.path.join(ROOT, "tests", "golden")
 def pytest_configure(config):
     config.addinivalue_line("markers", "gpu: needs a B200 (run via gpurun)")
     config.addinivalue_line("markers", "slow: long-running")
+    # the library's on-disk cubin cache (SKL_CACHE_DIR), in a directory fresh for
+    # this session: the many short-lived contexts of the tests compile each
+    # (skeleton, types, options) program once instead of once per context; a
+    # test that sets its own directory (test_abi's cache test) still can
+    if "SKL_CACHE_DIR" not in os.environ:
+        import tempfile
+        os.environ["SKL_CACHE_DIR"] = tempfile.mkdtemp(prefix="skl_test_cache_")
 
 
 def read_golden(name):
