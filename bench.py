@@ -607,7 +607,8 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
         "workload": f"copy(+) -> block of a 150^3 fp32 Vector, {where} "
                     "(exchange fused into the device-order fold: every slice read straight from the replicas)",
         "ms": round(seg[1], 4), "algorithmic_bytes": traffic,
-        "roofline": roof_hbm(traffic, seg[1], P, ngpu=G if physical else 1),
+        "roofline": roof_hbm(traffic, seg[1], P, "redist_copy_add_to_block" if not physical else None,
+                             ngpu=G if physical else 1),
         "staged": {"ms": round(seg0[1], 4), "bytes_moved": moved,
                    "note": "slices exchanged into staging, then folded (combine_peer=0)",
                    "roofline": roof_hbm(2 * moved + traffic, seg0[1], P, ngpu=G if physical else 1)},

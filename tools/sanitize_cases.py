@@ -149,7 +149,42 @@ def tma_and_hybrid(G):
     ctx.finalize()
 
 
+def tma_tile_cases(G):
+    """the default TMA tile kernel (skl_mo2d_t, 1 and 2 tiles per block, border
+    patching, parts with halo rows, fused halo push) on G logical devices, both
+    Sobel forms, and the one-pass copy(+) fold on slices that start mid-word"""
+    for kt in (1, 2):
+        ctx = S.Context(G, devices=[0] * G)
+        ctx.set_option("mo_kt", kt)
+        n0 = ctx.counter("tma_launches")
+        img8 = I.image_u8(5, 70, 144)
+        for src in (A.SOBEL, A.SOBEL_SEPARABLE):
+            sob = S.MapOverlap(ctx, src, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            s1 = sob(sob(S.Matrix.from_numpy(ctx, img8)))
+            r8 = O.mapoverlap2d(O.OS_SOBEL, O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0), 1, O.OB_NEUTRAL, 0)
+            assert np.array_equal(s1.to_numpy(), r8)
+        imgf = I.image_f32(6, 150, 272)
+        ctx.set_option("block_threads", 128)
+        gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+        g2 = gau(gau(S.Matrix.from_numpy(ctx, imgf)))
+        r1 = O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0)
+        assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
+        assert ctx.counter("tma_launches") - n0 == 6 * G
+        n = 3001
+        addf = S.Reduce(ctx, A.ADD, S.F32)
+        cv = S.Vector(ctx, S.F32, n).set_distribution(S.COPY, 0, addf).fill(0.0)
+        idx = S.Vector.from_numpy(ctx, np.arange(n, dtype=np.int32)).set_distribution(S.BLOCK)
+        touch = S.Map(ctx, "void touch(int i, float* c) { c[i] = 1.0f + (float)(i % 5); }", S.I32, S.VOID,
+                      extra=[S.F32 | S.PTR])
+        touch(idx, (cv, S.WRITE))
+        cv.set_distribution(S.BLOCK)
+        assert np.array_equal(cv.to_numpy(), (1.0 + np.arange(n) % 5).astype(np.float32))
+        ctx.finalize()
+
+
 if __name__ == "__main__":
+    tma_tile_cases(1)
+    tma_tile_cases(3)
     one_device({})
     one_device({"scan_variant": 3, "map_interleave": 1, "block_threads": 128})
     logical_devices(3)
