@@ -41,10 +41,13 @@ NcclApi* nccl() {
   static NcclApi a;
   static std::once_flag once;
   std::call_once(once, [] {
+    // the copy already in the process first (torch's bundled NCCL when torch was
+    // imported): one NCCL build per process, never two side by side
+    a.h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD);
     const char* names[] = {"libnccl.so.2", "/usr/lib/x86_64-linux-gnu/libnccl.so.2", "libnccl.so"};
     for (const char* n : names) {
-      a.h = dlopen(n, RTLD_NOW | RTLD_GLOBAL);
       if (a.h) break;
+      a.h = dlopen(n, RTLD_NOW | RTLD_GLOBAL);
     }
     if (!a.h) return;
     a.getUniqueId = (decltype(a.getUniqueId))dlsym(a.h, "ncclGetUniqueId");
