@@ -183,8 +183,9 @@ void launch_xfer_batch(Ctx* ctx, int g, const std::vector<XferSeg>& segs) {
 // epoch into rank h's signal slot for this rank (a system-scope release over
 // NVLink: everything this GPU wrote before is visible to rank h first), then
 // waits for rank h's epoch in this rank's slot h (acquire).  The grid is one
-// warp; a wait longer than 20 s (globaltimer) raises the host-mapped error flag
-// and returns instead of hanging the GPU.
+// warp; a wait longer than 60 s (globaltimer) raises the host-mapped error flag
+// and returns instead of hanging the GPU (60 s: a peer may still be draining a
+// deep queue of earlier work before it reaches its barrier).
 struct SklSigSlots {
   unsigned long long* p[kIpcMaxRanks];
 };
@@ -203,7 +204,7 @@ __global__ void __launch_bounds__(32) skl_ipc_barrier(SklSigSlots peers, int wor
     if (v >= epoch) break;
     unsigned long long t;
     asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
-    if (t - t0 > 20000000000ull) {
+    if (t - t0 > 60000000000ull) {
       atomicExch(err, 1u);
       break;
     }

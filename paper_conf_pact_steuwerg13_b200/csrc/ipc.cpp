@@ -19,7 +19,7 @@
 //     signal slot (st.release.sys over NVLink) and spins on its own slots
 //     (ld.acquire.sys) - the producers of a collective's inputs are complete on
 //     every GPU before any rank reads them, and every read is complete before a
-//     rank reuses the memory.  A spin gives up after 20 s and raises a sticky
+//     rank reuses the memory.  A spin gives up after 60 s and raises a sticky
 //     host-visible error (SKL_ERR_NCCL at the next collective) instead of
 //     hanging the GPU.
 // Several ranks may share one GPU (processes time-slice it): the tests run 2-3
