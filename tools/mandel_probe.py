@@ -1,0 +1,77 @@
+"""Mandelbrot headline probe on one GPU: the per-pixel blocktest user function
+vs the two-pixel packed-fp32x2 user function (apps.mandelbrot_pairs), several
+launch configurations, each timed (CUDA events, L2 flushed, median of 20) and
+checked bit for bit against the oracle on the whole 4096x3072 image.
+
+  MANDEL_CFGS="kind,block,unroll,interleave,B;..."   kind: single | pairs
+"""
+import os
+import sys
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import torch  # noqa: E402
+
+import oracle as O  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import apps as A  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import inputs as I  # noqa: E402
+from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
+
+ROWS, COLS, MAX = 3072, 4096, 1000
+
+
+def timeit(fn, flush, reps=20, warm=3):
+    for _ in range(warm):
+        fn()
+    torch.cuda.synchronize()
+    torch.cuda._sleep(int(reps * 4e5))
+    ts = []
+    for _ in range(reps):
+        flush.zero_()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record()
+        fn()
+        b.record()
+        ts.append((a, b))
+    torch.cuda.synchronize()
+    return float(np.median([a.elapsed_time(b) for a, b in ts]))
+
+
+def main():
+    flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
+    grid = I.mandel_grid(ROWS, COLS)
+    ref, tot = O.mandelbrot(grid, MAX)
+    cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;pairs,1024,1,1,12;pairs,512,1,1,12;pairs,256,1,1,12")
+    for cfg in cfgs.split(";"):
+        kind, bt, un, il, B = cfg.split(",")
+        c = S.Context(1)
+        st = torch.cuda.Stream()
+        torch.cuda.set_stream(st)
+        c.set_stream(0, st.cuda_stream)
+        c.set_option("block_threads", int(bt))
+        c.set_option("map_unroll", int(un))
+        c.set_option("map_interleave", int(il))
+        if kind == "single":
+            m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
+            x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(grid)
+            o = S.Matrix(c, S.U32, ROWS, COLS)
+        else:
+            p2 = c.struct_type("Pix2", A.PIX2_DECL, 16, 16)
+            c2 = c.struct_type("Cnt2", A.CNT2_DECL, 8, 8)
+            m = S.Map(c, A.mandelbrot_pairs(MAX, int(B)), p2, c2)
+            x = S.Matrix(c, p2, ROWS, COLS // 2).copy_in(grid)
+            o = S.Matrix(c, c2, ROWS, COLS // 2)
+        m(x, out=o)
+        ms = timeit(lambda: m(x, out=o), flush)
+        got = o.to_numpy(np.uint32).reshape(ROWS, COLS)
+        ok = bool(np.array_equal(got, ref))
+        print(f"mandel {cfg}: {ms:.4f} ms  {8 * tot / (ms / 1e3) / 1e12:.2f} TFLOP/s (8 ops/iter)  bitexact={ok}",
+              flush=True)
+        c.finalize()
+
+
+if __name__ == "__main__":
+    main()
