@@ -1,9 +1,12 @@
 """Mandelbrot headline probe on one GPU: the per-pixel blocktest user function
-vs the two-pixel packed-fp32x2 user function (apps.mandelbrot_pairs), several
-launch configurations, each timed (CUDA events, L2 flushed, median of 20) and
-checked bit for bit against the oracle on the whole 4096x3072 image.
+in several launch configurations, each timed (CUDA events, L2 flushed, median
+of 20) and checked bit for bit against the oracle on the whole 4096x3072 image.
+(The two-pixel packed fp32x2 variant measured with it in round 2 -
+profiles/sweeps/sweep_r02_mandel_pairs.log - is in the history of
+paper_conf_pact_steuwerg13_b200/apps.py, commit "Mandelbrot user function for
+two neighbouring pixels".)
 
-  MANDEL_CFGS="kind,block,unroll,interleave,B;..."   kind: single | pairs
+  MANDEL_CFGS="single,block,unroll,interleave,B;..."
 """
 import os
 import sys
@@ -44,7 +47,7 @@ def main():
     flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
     grid = I.mandel_grid(ROWS, COLS)
     ref, tot = O.mandelbrot(grid, MAX)
-    cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;pairs,1024,1,1,12;pairs,512,1,1,12;pairs,256,1,1,12")
+    cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;single,512,1,1,12")
     for cfg in cfgs.split(";"):
         kind, bt, un, il, B = cfg.split(",")
         c = S.Context(1)
@@ -54,16 +57,9 @@ def main():
         c.set_option("block_threads", int(bt))
         c.set_option("map_unroll", int(un))
         c.set_option("map_interleave", int(il))
-        if kind == "single":
-            m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
-            x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(grid)
-            o = S.Matrix(c, S.U32, ROWS, COLS)
-        else:
-            p2 = c.struct_type("Pix2", A.PIX2_DECL, 16, 16)
-            c2 = c.struct_type("Cnt2", A.CNT2_DECL, 8, 8)
-            m = S.Map(c, A.mandelbrot_pairs(MAX, int(B)), p2, c2)
-            x = S.Matrix(c, p2, ROWS, COLS // 2).copy_in(grid)
-            o = S.Matrix(c, c2, ROWS, COLS // 2)
+        m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
+        x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(grid)
+        o = S.Matrix(c, S.U32, ROWS, COLS)
         m(x, out=o)
         ms = timeit(lambda: m(x, out=o), flush)
         got = o.to_numpy(np.uint32).reshape(ROWS, COLS)
