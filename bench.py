@@ -157,10 +157,13 @@ class Env:
             dist.init_process_group("gloo")
             self.pg = dist
         else:
-            if gpus > nvis:
+            # SKL_BENCH_LOGICAL=1 (tests of this path on one GPU): N logical devices
+            # on GPU 0, labelled as such; otherwise N physical GPUs
+            self.logical = os.environ.get("SKL_BENCH_LOGICAL") == "1"
+            if gpus > nvis and not self.logical:
                 raise SystemExit(f"--gpus {gpus} but only {nvis} visible GPU(s)")
             self.G = gpus
-            self.local = [(g, g) for g in range(gpus)]
+            self.local = [(g, 0 if self.logical else g) for g in range(gpus)]
             torch.cuda.set_device(0)
         self.phys = [p for _, p in self.local]
 
@@ -169,6 +172,8 @@ class Env:
         if self.spmd:
             comm = os.environ.get("SKL_COMM") or "ipc"
             return f"one process per GPU (torchrun, skl_init_dist, transport {comm})"
+        if getattr(self, "logical", False):
+            return f"one process driving {self.G} LOGICAL devices on one GPU (skl_init; testing only)"
         return f"one process driving {self.G} GPU(s) (skl_init)"
 
     def barrier(self):
@@ -381,7 +386,7 @@ def bench_mandelbrot(args, E: Env, P: dict):
     def step(_):
         m(cin, out=out)
 
-    clk = ClockSampler(E.phys)
+    clk = ClockSampler(sorted(set(E.phys)))
     clk.start()
     st, _ = timer.run(step, args.steps, args.warmup)
     clocks = clk.stop()
@@ -541,7 +546,7 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
     physical = E.G > 1
     c4 = make_context(E) if physical else make_context(E, logical=4)
     G = c4.ndev
-    where = (f"{G} physical GPUs (NVLink), {E.mode}" if physical else f"{G} logical devices on one GPU")
+    where = (f"{G} devices, {E.mode}" if physical else f"{G} logical devices on one GPU")
     timer = Timer(c4, E)
     N = 150
     nvox = N ** 3
