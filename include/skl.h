@@ -89,11 +89,21 @@ skl_status skl_type_size(skl_ctx* ctx, skl_type t, size_t* size);
  * distribution machinery runs on a 1-GPU box.
  *
  * skl_init_dist: one process per GPU (torchrun).  Global device g is rank g;
- * `nccl_id` is the 128-byte ncclUniqueId from skl_nccl_unique_id() on rank 0,
- * broadcast by the caller.  Exchanges between ranks use NCCL send/recv over
- * NVLink (libnccl.so.2 is loaded on first use).  Every rank must issue the same
- * sequence of calls (SPMD): host-visible results and redistributions are
- * collective.                                                                  */
+ * `nccl_id` is the 128-byte id from skl_nccl_unique_id() on rank 0, broadcast
+ * by the caller.  The transport between the ranks is chosen by the environment
+ * variable SKL_COMM (identical on every rank):
+ *   "ipc" (default; the ranks of one node): device memory comes from an IPC
+ *     heap, each rank maps the peers' buffers with CUDA IPC, and every exchange
+ *     (redistribution, halo push, copy(+) fold, Reduce partials, Scan carries)
+ *     runs as in-kernel peer loads/stores ordered by device barriers; the id is
+ *     the name of a POSIX shared-memory control block; a barrier that waits
+ *     more than 60 s fails the next call with SKL_ERR_NCCL instead of hanging;
+ *   "nccl": NCCL send/recv of the same transfer lists (libnccl.so.2 - the copy
+ *     already loaded in the process, if any - is loaded on first use; the id is
+ *     an ncclUniqueId);
+ *   "shm": a host shared-memory loopback (tests, several ranks on one GPU).
+ * Every rank must issue the same sequence of calls (SPMD): host-visible results
+ * and redistributions are collective.                                          */
 skl_status skl_init(int ndev, const int* devices, skl_ctx** out);
 skl_status skl_init_dist(int rank, int world, int cuda_device, const void* nccl_id, skl_ctx** out);
 skl_status skl_nccl_unique_id(void* out128);
@@ -114,6 +124,8 @@ skl_status skl_sync(skl_ctx* ctx);
  * restores the default.                                                        */
 typedef void* (*skl_alloc_fn)(size_t bytes, int cuda_device, void* cuda_stream, void* user);
 typedef void (*skl_free_fn)(void* ptr, int cuda_device, void* cuda_stream, void* user);
+/* (With the "ipc" transport of skl_init_dist every buffer comes from the IPC
+ * heap, which peers must be able to map; a caller's allocator is not used.)    */
 skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn release, void* user);
 /* Options: "block_threads" (work-group size; default 256),
  * "debug_bounds" (1 = get() range-checked, A21), "map_unroll" (chunks per

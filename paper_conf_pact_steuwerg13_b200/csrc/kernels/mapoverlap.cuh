@@ -191,6 +191,22 @@ __device__ __forceinline__ void skl_mo_apply(const SKL_TIN* tile, SKL_TOUT* __re
     }
     return;
   }
+#if SKL_OUT_PACK
+  if (full && rt + SKL_RH <= re) {
+    // every row of this thread in range and whole packed stores (all threads
+    // but those of a device's last tile row or the matrix's last columns): no
+    // per-row guard or partial-store path in the loop
+#pragma unroll
+    for (int i = 0; i < SKL_RH; ++i) {
+      const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
+      SklMoRes res;
+#pragma unroll
+      for (int j = 0; j < SKL_CW; ++j) res.e[j] = SKL_FUNC((SKL_TIN*)(p + j));
+      skl_mo_store(o + (long)i * Ci, res, true, SKL_CW);
+    }
+    return;
+  }
+#endif
 #pragma unroll
   for (int i = 0; i < SKL_RH; ++i) {
     const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;
