@@ -81,6 +81,9 @@ __device__ __forceinline__ void skl_mo_store(SKL_TOUT* o, const SklMoRes& v, boo
 #ifndef SKL_MO_MINB
 #define SKL_MO_MINB 1
 #endif
+#ifndef SKL_MO_HEAVY
+#define SKL_MO_HEAVY 0
+#endif
 
 // Geometry of one launch: 32-bit row / column arithmetic (the host guarantees
 // R, C < 2^31); 64-bit only where a row index is scaled to an element offset.
@@ -191,11 +194,14 @@ __device__ __forceinline__ void skl_mo_apply(const SKL_TIN* tile, SKL_TOUT* __re
     }
     return;
   }
-#if SKL_OUT_PACK
+#if SKL_OUT_PACK && SKL_MO_HEAVY
   if (full && rt + SKL_RH <= re) {
     // every row of this thread in range and whole packed stores (all threads
     // but those of a device's last tile row or the matrix's last columns): no
-    // per-row guard or partial-store path in the loop
+    // per-row guard or partial-store path in the loop.  Heavy functions only
+    // (the Gaussian 117 -> 109 us, Listing 1.5's Sobel 76 -> 74 us); for a
+    // light one the second copy of the loop cost more than the guards
+    // (identity u8 26.7 -> 27.7 us)
 #pragma unroll
     for (int i = 0; i < SKL_RH; ++i) {
       const SKL_TIN* p = tile + (SKL_D + ty * SKL_RH + i) * SKL_PITCH + SKL_A + tx * SKL_CW;

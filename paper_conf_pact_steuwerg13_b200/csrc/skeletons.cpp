@@ -56,9 +56,11 @@ std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
 }
 
 std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
+// rows per thread, tile rows, tiles per block; a block of 2+ tiles marks a heavy
+// function (>= 64 registers), which also gets the unguarded full-tile path
 std::string mo_rows_defs(int rh, int th, int kt) {
   return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n#define SKL_MO_KT " +
-         std::to_string(kt) + "\n";
+         std::to_string(kt) + "\n#define SKL_MO_HEAVY " + (kt > 1 ? "1" : "0") + "\n";
 }
 
 // Scratch buffer per (skeleton, device), grown on demand.
