@@ -4,6 +4,8 @@ flushed), each checked against the oracle on row bands.
 
   python tools/mo_probe.py [names] [--once]      names: ident_u8,sobel,sobel_sep,ident_f32,gauss
   MO_OPTS="key=value,..."  library options (skl_set_option) for every context
+  MO_PER_EVENT=k           k launches between one event pair (time per launch = total / k)
+  MO_NOFLUSH=1             no L2 flush before the timed launches
 
 --once runs each kernel a single time (for ncu -k regex:skl_mo launch lists).
 """
@@ -33,14 +35,15 @@ def opts():
     return out
 
 
-def timeit(fn, flush, reps=20, warm=3):
+def timeit(fn, flush, reps=20, warm=3, flush_on=True):
     for _ in range(warm):
         fn()
     torch.cuda.synchronize()
     torch.cuda._sleep(int(reps * 4e5))
     ts = []
     for _ in range(reps):
-        flush.zero_()
+        if flush_on:
+            flush.zero_()
         a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         a.record()
         fn()
@@ -88,7 +91,12 @@ def main():
             torch.cuda.synchronize()
             print(f"{name}: ran once", flush=True)
         else:
-            ms = timeit(lambda: mo(mi, out=out), flush)
+            per = int(os.environ.get("MO_PER_EVENT", "1"))   # launches between one event pair
+
+            def many():
+                for _ in range(per):
+                    mo(mi, out=out)
+            ms = timeit(many, flush, flush_on=os.environ.get("MO_NOFLUSH") != "1") / per
             full = out.to_numpy()
             ok = True
             for r0 in (0, 4000, R - 64):
