@@ -1267,8 +1267,11 @@ def main():
                    "row_order": "identity" if G == 1 else "round-robin (application-level balancing)",
                    "imbalance_limited_ideal_speedup": float(sum(per) / max(per)) if max(per) > 0 else 1.0},
         "roofline": {**roof_alu(flops, ms, P, sms, G,
-                                f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count); peak = {G} x {sms} SMs "
-                                f"x 128 FP32 lanes x {P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false)"),
+                                f"8 fp32 ops/iteration x {sum_iter} iterations (oracle count: the A22 loop's 3 mul, "
+                                f"4 add/sub and the escape-test add); peak = {G} x {sms} SMs x 128 FP32 lanes x "
+                                f"{P['sm_max_mhz']:.0f} MHz (no FMA: -fmad=false).  The tuned user function executes 7 "
+                                f"per iteration inside escape-free blocks (the test once per block), so its executed-op "
+                                f"rate is about 7/8 of 'achieved'"),
                      "traffic": ncu_traffic("mandelbrot")},
         "cpu_baseline": {"value": ROWS * COLS / cpu_s, "unit": "elements/s", "cores": 1, "kind": "oracle", **cpu_info(),
                          "sample": f"whole {COLS}x{ROWS} image, single thread ({cpu_s:.2f} s)"},
