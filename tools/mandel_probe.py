@@ -6,7 +6,8 @@ profiles/sweeps/sweep_r02_mandel_pairs.log - is in the history of
 paper_conf_pact_steuwerg13_b200/apps.py, commit "Mandelbrot user function for
 two neighbouring pixels".)
 
-  MANDEL_CFGS="single,block,unroll,interleave,B;..."
+  MANDEL_CFGS="single,block,unroll,interleave,B[,THxTW];..."   THxTW: pixels stored in
+  TH x TW warp tiles (application-level layout, restored on download)
 """
 import os
 import sys
@@ -49,7 +50,12 @@ def main():
     ref, tot = O.mandelbrot(grid, MAX)
     cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;single,512,1,1,12")
     for cfg in cfgs.split(";"):
-        kind, bt, un, il, B = cfg.split(",")
+        kind, bt, un, il, B = cfg.split(",")[:5]
+        tile = cfg.split(",")[5] if len(cfg.split(",")) > 5 else ""
+        perm = np.arange(ROWS * COLS)
+        if tile:
+            th, tw = (int(v) for v in tile.split("x"))
+            perm = perm.reshape(ROWS // th, th, COLS // tw, tw).transpose(0, 2, 1, 3).reshape(-1)
         c = S.Context(1)
         st = torch.cuda.Stream()
         torch.cuda.set_stream(st)
@@ -58,11 +64,13 @@ def main():
         c.set_option("map_unroll", int(un))
         c.set_option("map_interleave", int(il))
         m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
-        x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(grid)
+        x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(np.ascontiguousarray(grid.reshape(-1, 2)[perm]))
         o = S.Matrix(c, S.U32, ROWS, COLS)
         m(x, out=o)
         ms = timeit(lambda: m(x, out=o), flush)
-        got = o.to_numpy(np.uint32).reshape(ROWS, COLS)
+        got = np.empty(ROWS * COLS, np.uint32)
+        got[perm] = o.to_numpy(np.uint32).reshape(-1)
+        got = got.reshape(ROWS, COLS)
         ok = bool(np.array_equal(got, ref))
         print(f"mandel {cfg}: {ms:.4f} ms  {8 * tot / (ms / 1e3) / 1e12:.2f} TFLOP/s (8 ops/iter)  bitexact={ok}",
               flush=True)
