@@ -353,19 +353,25 @@ def mandel_map(ctx, plain: bool = False):
         # the A22 loop as written (apps.mandelbrot), default Map configuration
         return S.Map(ctx, A.mandelbrot(MAX_ITER), S.F32X2, S.U32)
     # user-side tuning (the paper's optional work-group size):
-    # 1024-thread blocks, one 4-pixel chunk per thread, warp-interleaved pixels
-    # (lanes of a warp iterate neighbouring pixels: less idle-lane time); the
-    # customising function tests the escape on the end state of each block of 12
-    # iterations (the orbit grows monotonically after an escape) and replays a
-    # suspicious block exactly (bit-identical counts; apps.mandelbrot_blocktest).
-    # Swept: profiles/sweeps/sweep18-19, sweep24.
-    ctx.set_option("block_threads", 1024)
+    # 128-thread blocks, ONE pixel per thread, warp-interleaved pixels (lanes of
+    # a warp iterate neighbouring pixels: less idle-lane time) - many small blocks
+    # let the block scheduler balance the data-dependent cost, also when a GPU's
+    # share is small (8 GPUs: 384 rows); the customising function tests the
+    # escape on the end state of each block of 12 iterations (the orbit grows
+    # monotonically after an escape) and replays a suspicious block exactly
+    # (bit-identical counts; apps.mandelbrot_blocktest).  Swept:
+    # profiles/sweeps/sweep18-19, sweep24, sweep_r02_mandel_share.log (1024
+    # threads x 4 pixels 0.764 ms -> 128 x 1 0.716 ms; one GPU's share at 8 GPUs
+    # 0.127 -> 0.117 ms).
+    ctx.set_option("block_threads", 128)
     ctx.set_option("map_unroll", 1)
     ctx.set_option("map_interleave", 1)
+    ctx.set_option("map_il_elems", 1)
     m = S.Map(ctx, A.mandelbrot_blocktest(MAX_ITER, 12), S.F32X2, S.U32)
     ctx.set_option("block_threads", 256)
     ctx.set_option("map_unroll", 4)
     ctx.set_option("map_interleave", 0)
+    ctx.set_option("map_il_elems", 0)
     return m
 
 

@@ -135,7 +135,9 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * border units into the neighbours' halo units, so the next overlap read
  * exchanges nothing; default 1), "map_interleave" (1 = lane l of a
  * warp handles elements base + 32 j + l: for customising functions whose cost
- * varies per element, e.g. Mandelbrot; default 0), "ap_fast" (Allpairs
+ * varies per element, e.g. Mandelbrot; default 0), "map_il_elems" (elements
+ * per lane of the interleaved kernel; 0 = one 16-byte chunk's worth; default 0),
+ * "ap_fast" (Allpairs
  * zip-reduce 128 x 128 tiles for 4-byte inputs with d % 4 == 0; default 1),
  * "ap_hybrid" (1 = when the 128 x 128 tiles leave the last wave less than half
  * full, that wave runs as 128 x 64 halves; default 1), "ap_tile" (0 = automatic,

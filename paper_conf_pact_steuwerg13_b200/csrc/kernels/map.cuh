@@ -21,6 +21,9 @@
 #define SKL_XARGS
 #endif
 
+#ifndef SKL_ILJ
+#define SKL_ILJ (SKL_UNROLL * SKL_VEC)
+#endif
 #define SKL_QIN ((SKL_VEC * sizeof(SKL_TIN)) / 16)
 #if SKL_ZIP
 #define SKL_QIN2 ((SKL_VEC * sizeof(SKL_TIN2)) / 16)
@@ -150,7 +153,7 @@ skl_map_sc(const SKL_TIN* __restrict__ in SKL_IN2_PARAM SKL_OUT_PARAM, skl_u64 n
 // counts).  Each load / store instruction still covers a contiguous run.
 extern "C" __global__ void __launch_bounds__(SKL_BLOCK)
 skl_map_il(const SKL_TIN* __restrict__ in SKL_IN2_PARAM SKL_OUT_PARAM, skl_u64 n SKL_XPARAMS) {
-  constexpr int J = SKL_UNROLL * SKL_VEC;
+  constexpr int J = SKL_ILJ;  // elements per lane (option map_il_elems; default one chunk)
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const skl_u64 base = ((skl_u64)blockIdx.x * (SKL_BLOCK / 32) + warp) * (32 * J) + lane;
   SKL_TIN a[J];

@@ -118,6 +118,8 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       else defs += "#define SKL_TOUT " + tname(ctx, tout) + "\n#define SKL_OUT_VOID 0\n";
       defs += "#define SKL_VEC " + std::to_string(vec) + "\n";
       defs += "#define SKL_UNROLL " + std::to_string(ctx->map_unroll) + "\n";
+      s->ilj = ctx->map_il_elems > 0 ? ctx->map_il_elems : (int)(ctx->map_unroll * vec);
+      defs += "#define SKL_ILJ " + std::to_string(s->ilj) + "\n";
       std::string xp, xa;
       for (size_t k = 0; k < s->extra.size(); ++k) {
         const int t = s->extra[k];
@@ -490,7 +492,7 @@ static void run_elementwise(Skel* s, Cont* in, Cont* in2, Cont** out, const skl_
     size_t grid;
     const char* kname;
     if (s->interleave) {
-      grid = std::max<size_t>(1, ceil_div(n, per_block * vec));
+      grid = std::max<size_t>(1, ceil_div(n, (size_t)s->block * (size_t)s->ilj));
       kname = "skl_map_il";
     } else if (vec_ok) {
       grid = std::max<size_t>(1, ceil_div(n / vec, per_block));

@@ -146,6 +146,7 @@ struct Ctx {
   int lazy_fusion = 1;         // defer Zip/Map without an output (fused into a Reduce)
   int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
+  int map_il_elems = 0;        //   elements per lane of the interleaved kernel (0 = one chunk)
   int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
   int combine_unroll = 0;      // copy(+) -> block folds: 16-byte chunks per thread (0 = 2)
   int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
@@ -344,6 +345,7 @@ struct Skel {
   bool ap_zr = false;     // Allpairs: zip-reduce form
   int block = 256;   // threads per block the program was compiled for
   int unroll = 4;    // Map/Zip chunks per thread the program was compiled for
+  int ilj = 4;       // Map/Zip interleaved kernel: elements per lane (SKL_ILJ)
   bool interleave = false;  // Map/Zip: launch the warp-interleaved kernel
   std::map<Skel*, Program*> fused;  // Reduce: fused programs per producing Zip/Map
   std::map<Skel*, Skel*> composed;  // Map g: g∘f per producing Zip/Map f (nullptr: not composable)

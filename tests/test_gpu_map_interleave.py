@@ -16,14 +16,16 @@ pytestmark = pytest.mark.gpu
 SIZES = [1, 31, 33, 1000, 4097, (1 << 20) + 3]
 
 
-@pytest.fixture(scope="module", params=[(256, 1), (1024, 1), (128, 4)], ids=lambda p: f"b{p[0]}u{p[1]}")
+@pytest.fixture(scope="module", params=[(256, 1, 0), (1024, 1, 0), (128, 4, 0), (128, 1, 1), (64, 1, 3)],
+                ids=lambda p: f"b{p[0]}u{p[1]}j{p[2]}")
 def ctx(request):
     require_gpu()
-    bt, un = request.param
+    bt, un, j = request.param
     c = S.Context(1)
     c.set_option("map_interleave", 1)
     c.set_option("block_threads", bt)
     c.set_option("map_unroll", un)
+    c.set_option("map_il_elems", j)   # elements per lane (0 = one chunk)
     yield c
     c.finalize()
 

@@ -8,6 +8,9 @@ two neighbouring pixels".)
 
   MANDEL_CFGS="single,block,unroll,interleave,B[,THxTW];..."   THxTW: pixels stored in
   TH x TW warp tiles (application-level layout, restored on download)
+  MANDEL_ILJ=j     elements per lane of the interleaved Map kernel (map_il_elems)
+  MANDEL_EVERY=k   only rows 0, k, 2k, ... (one GPU's share of the image at k GPUs
+                   with the bench's round-robin row dealing)
 """
 import os
 import sys
@@ -46,7 +49,10 @@ def timeit(fn, flush, reps=20, warm=3):
 
 def main():
     flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
-    grid = I.mandel_grid(ROWS, COLS)
+    global ROWS
+    every = int(os.environ.get("MANDEL_EVERY", "1"))
+    grid = np.ascontiguousarray(I.mandel_grid(ROWS, COLS)[::every])
+    ROWS = grid.shape[0]
     ref, tot = O.mandelbrot(grid, MAX)
     cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;single,512,1,1,12")
     for cfg in cfgs.split(";"):
@@ -63,6 +69,8 @@ def main():
         c.set_option("block_threads", int(bt))
         c.set_option("map_unroll", int(un))
         c.set_option("map_interleave", int(il))
+        if os.environ.get("MANDEL_ILJ"):
+            c.set_option("map_il_elems", int(os.environ["MANDEL_ILJ"]))
         m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
         x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(np.ascontiguousarray(grid.reshape(-1, 2)[perm]))
         o = S.Matrix(c, S.U32, ROWS, COLS)
