@@ -1066,9 +1066,14 @@ def bench_skeletons(args, E: Env, P: dict, which):
     if "lmosem" in which:
         N, nev = 150, 10_000_000
         evd = ctx.struct_type("Event", A.EVENT_DECL, A.EVENT_SIZE, 4)
-        ctx.set_option("map_unroll", 1)   # divergent per-event work: one chunk per thread
+        # divergent per-event work: one event per thread (as lmosem.py)
+        ctx.set_option("map_unroll", 1)
+        ctx.set_option("map_interleave", 1)
+        ctx.set_option("map_il_elems", 1)
         lm = S.Map(ctx, A.lmosem_map(N), evd, S.VOID, extra=[S.F32 | S.PTR, S.F32 | S.PTR])
         ctx.set_option("map_unroll", 4)
+        ctx.set_option("map_interleave", 0)
+        ctx.set_option("map_il_elems", 0)
         upd = S.Zip(ctx, A.LMOSEM_UPDATE, S.F32, S.F32, S.F32)
         addf = S.Reduce(ctx, A.ADD, S.F32)
         events = I.lmosem_events(I.SEED_LMOSEM, nev, N)
