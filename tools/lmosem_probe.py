@@ -23,7 +23,7 @@ order = ListModeOSEM.path_order(events, N)
 sorted_ev = np.ascontiguousarray(events[order])
 sub = events[::50].copy()
 c_ref = O.lmosem(sub, N, np.ones(N ** 3, np.float32))[0]
-for cfg in os.environ.get("LM_CFGS", "256,1,0,0;128,1,0,0;128,1,1,1;256,1,1,1;64,1,1,1").split(";"):
+for cfg in os.environ.get("LM_CFGS", "256,1,0,0;128,1,0,0;128,1,1,1;256,1,1,1;64,1,1,1").split(";"):  # noqa: E501
     bt, un, il, j = (int(v) for v in cfg.split(","))
     ctx = S.Context(1)
     st = torch.cuda.Stream()
