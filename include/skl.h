@@ -145,7 +145,12 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * "xfer_kernel" (1 = with several devices in this process, the moves of a
  * redistribution or halo refresh into one GPU run as one batched copy kernel
  * (peer loads over NVLink between GPUs); 0 = one cudaMemcpy(Peer)Async per
- * move; default 1), "combine_peer" (copy(+) -> block with every device in
+ * move; default 1), "xfer_chunks" (host <-> device transfers of >= 4 MB per
+ * part go in this many chunks on copy-engine streams, so a Map computes chunk k
+ * while chunk k+1 uploads and its output streams back per chunk; 1..64,
+ * default 8), "xfer_taper" (1 = the last two chunks are 1/2 and 1/4 of the
+ * others, shortening the compute + download tail after the last upload;
+ * default 1), "combine_peer" (copy(+) -> block with every device in
  * this process: 1 = each device folds its slice straight out of the peers'
  * replicas in one kernel, no staging copy; logical devices of one GPU share one
  * launch; 2 = one kernel per device even then; 0 = slices exchanged into

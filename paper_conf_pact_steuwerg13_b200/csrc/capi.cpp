@@ -231,6 +231,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->combine_peer = (int)value;
     } else if (k == "xfer_kernel") {
       c->xfer_kernel = value ? 1 : 0;
+    } else if (k == "xfer_taper") {
+      c->xfer_taper = value ? 1 : 0;
     } else if (k == "xfer_chunks") {
       if (value < 1 || value > 64) fail(SKL_ERR_INVALID_ARG, "xfer_chunks in [1,64]");
       c->xfer_chunks = (int)value;

@@ -62,11 +62,23 @@ static int xfer_chunks(Ctx* ctx, size_t bytes) {
   return (int)std::min<size_t>((size_t)ctx->xfer_chunks, bytes / (1u << 20));
 }
 // chunk k of K of the unit range r (boundaries on multiples of 64 units, so
-// that chunk pointers keep the buffer's 16-byte alignment)
-static Range chunk_of(const Range& r, int k, int K) {
+// that chunk pointers keep the buffer's 16-byte alignment).  Tapered (default,
+// option xfer_taper): the last two chunks are 1/4 and 1/2 of the others, so the
+// work that follows the last upload - computing the last chunk and streaming
+// its result back - is short (the end-to-end step of a Map whose input and
+// output cross PCIe is the upload time plus that tail).
+static Range chunk_of(Ctx* ctx, const Range& r, int k, int K) {
+  // weights in quarters: 4 for every chunk but the last two (2, 1)
+  const bool taper = ctx->xfer_taper && K >= 4;
+  const size_t total = taper ? (size_t)4 * (size_t)(K - 2) + 3 : (size_t)K;
+  auto cum = [&](int i) -> size_t {  // weight of chunks [0, i)
+    if (!taper) return (size_t)i;
+    if (i <= K - 2) return (size_t)4 * (size_t)i;
+    return (size_t)4 * (size_t)(K - 2) + (i == K - 1 ? 2 : 3);
+  };
   auto cut = [&](int i) -> size_t {
     if (i >= K) return r.hi;
-    return r.lo + (r.size() * (size_t)i / (size_t)K) / 64 * 64;
+    return r.lo + (r.size() * cum(i) / total) / 64 * 64;
   };
   return Range{cut(k), cut(k + 1)};
 }
@@ -191,7 +203,7 @@ void host_upload(Cont* c, const void* host) {
       SKL_CUDA(cudaStreamWaitEvent(D.h2d, D.ev, 0));
       Part& p = c->parts[(size_t)g];
       for (int k = 0; k < K; ++k) {
-        const Range q = chunk_of(r, k, K);
+        const Range q = chunk_of(ctx, r, k, K);
         if (q.empty()) continue;
         SKL_CUDA(cudaMemcpyAsync(part_ptr(c, g, q.lo), (const char*)host + q.lo * ub, q.size() * ub,
                                  cudaMemcpyHostToDevice, D.h2d));

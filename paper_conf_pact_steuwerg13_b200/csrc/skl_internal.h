@@ -152,6 +152,7 @@ struct Ctx {
   int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
                                // (0 = staged exchange then fold, 2 = one kernel per device even on one GPU)
   int xfer_chunks = 8;         // host<->device transfers split into this many chunks per part
+  int xfer_taper = 1;          //   the last two chunks 1/2 and 1/4 of the others (short tail)
   int ap_fast = 1;             // Allpairs zip-reduce: 128-row tiles (4-byte inputs, d % 4 == 0)
   int ap_tile = 0;             // Allpairs tile columns: 0 = by wave fill, 8 = 128, 4 = 64, 2 = hybrid
   int ap_bk = 0;               // Allpairs 128-row kernels: k-slice depth (0 = 16)

@@ -312,8 +312,10 @@ def e2e():
     d2h = timeit(lambda: pin_out.copy_(dev_out, non_blocking=True))
     print(f"PCIe pinned H2D {grid.nbytes / 1e6:.0f} MB: {h2d:.3f} ms ({grid.nbytes / h2d / 1e6:.1f} GB/s); "
           f"D2H {R * Cc * 4 / 1e6:.0f} MB: {d2h:.3f} ms ({R * Cc * 4 / d2h / 1e6:.1f} GB/s)", flush=True)
-    for ch in (int(x) for x in os.environ.get("E2E_CHUNKS", "4,8,16,32").split(",")):
-        c = ctx_with({"xfer_chunks": ch, "block_threads": 1024, "map_unroll": 1, "map_interleave": 1})
+    for cfg in os.environ.get("E2E_CHUNKS", "4,8,16,32").split(","):
+        ch, taper = (int(v) for v in (cfg.split(":") + ["1"])[:2])   # "chunks[:taper]"
+        c = ctx_with({"xfer_chunks": ch, "xfer_taper": taper, "block_threads": 128, "map_unroll": 1,
+                      "map_interleave": 1, "map_il_elems": 1})
         m = S.Map(c, A.mandelbrot_blocktest(1000, 12), S.F32X2, S.U32)
         e_in = S.Matrix(c, S.F32X2, R, Cc).set_distribution(S.BLOCK)
         e_out = S.Matrix(c, S.U32, R, Cc)
@@ -325,7 +327,7 @@ def e2e():
 
         ms = timeit(step, reps=10)
         dev = timeit(lambda: m(e_in, out=e_out), reps=10)
-        print(f"e2e chunks={ch}: {ms:.3f} ms (kernel alone {dev:.3f} ms)", flush=True)
+        print(f"e2e chunks={ch} taper={taper}: {ms:.3f} ms (kernel alone {dev:.3f} ms)", flush=True)
         c.finalize()
 
 
