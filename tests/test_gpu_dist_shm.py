@@ -71,7 +71,7 @@ def _worker(rank, world, nid, q, comm="shm"):
             assert ctx.counter("halo_push_bytes") > h0
         # iterated Sobel (ping-pong, halos pushed / exchanged every iteration)
         im8 = I.image_u8(I.SEED_SOBEL, 131, 80)
-        sob = S.MapOverlap(ctx, A.SOBEL_SEPARABLE, S.U8, S.U8, 1, S.NEUTRAL, 0)
+        sob = S.MapOverlap(ctx, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)
         a8 = S.Matrix.from_numpy(ctx, im8)
         b8, t8 = sob(a8), None
         ref8 = O.mapoverlap2d(O.OS_SOBEL, im8, 1, O.OB_NEUTRAL, 0)

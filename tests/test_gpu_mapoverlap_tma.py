@@ -5,9 +5,9 @@ outside the matrix are zero-filled by the copy engine and patched for NEAREST
 and non-zero NEUTRAL (A20).  Bit-exact against the oracle at sizes
 spanning several tiles with ragged edges, every boundary mode, byte and float
 images, logical multi-device runs with the fused halo push; the per-thread
-cp.async kernel (mo_tma=0) gives the same results.  Also the separable Sobel
-user function (apps.SOBEL_SEPARABLE): full images and its square-root step for
-every m."""
+cp.async kernel (mo_tma=0) gives the same results.  Also the tuned Sobel user
+function (apps.SOBEL_TUNED): full images in every register-block geometry and
+its square-root step for every m."""
 import re
 
 import numpy as np
@@ -64,7 +64,7 @@ def test_tma_u8(shape, rh, tma, kt):
         x = I.image_u8(I.SEED_SOBEL, *shape)
         m = S.Matrix.from_numpy(c, x)
         before = c.counter("tma_launches")
-        for src in (A.SOBEL, A.SOBEL_SEPARABLE):
+        for src in (A.SOBEL, A.SOBEL_TUNED):
             sob = S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)
             assert np.array_equal(sob(m).to_numpy(), O.mapoverlap2d(O.OS_SOBEL, x, 1, O.OB_NEUTRAL, 0)), src
         sx = S.MapOverlap(c, A.SHIFTX_U8, S.U8, S.U8, 1, S.NEAREST, 0)
@@ -90,7 +90,7 @@ def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
             f = lambda r: O.mapoverlap2d(O.OS_GAUSS5, r, 2, O.OB_NEAREST, 0.0)  # noqa: E731
         else:
             x = I.image_u8(I.SEED_SOBEL, 301, 272)
-            st = S.MapOverlap(c, A.SOBEL_SEPARABLE, S.U8, S.U8, 1, S.NEUTRAL, 0)
+            st = S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)
             f = lambda r: O.mapoverlap2d(O.OS_SOBEL, r, 1, O.OB_NEUTRAL, 0)  # noqa: E731
         a = S.Matrix.from_numpy(c, x)
         b = st(a)
@@ -106,15 +106,16 @@ def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
         c.finalize()
 
 
-def test_sobel_separable_root_step_every_m():
-    """the square-root step of apps.SOBEL_SEPARABLE, cut out of the user function's
+def test_sobel_tuned_root_step_every_m():
+    """the square-root step of apps.SOBEL_TUNED, cut out of the user function's
     own text and run as a Map over m = 0 .. 2^21 - 1 (h^2 + v^2 <= 2,080,800 <
     2^21), against numpy's correctly rounded fp32 root: min(255, (int)sqrtf(m))"""
     c = tma_ctx()
     try:
-        src = A.SOBEL_SEPARABLE
-        body = src[src.index("  float fm"):src.index("}", src.index("return (uchar)(m >= 65025"))]
-        assert "rsqrt.approx" in body and "return (uchar)(m >= 65025 ? 255 : r);" in body
+        src = A.SOBEL_TUNED
+        last = "  return (uchar)__float_as_int(t);\n"
+        body = src[src.index("  float k"):src.index(last) + len(last)]
+        assert "sqrt.approx" in body and "add.rm" in body
         fn = "uchar root(int m) {\n" + body + "}"
         n = 1 << 21
         m = np.arange(n, dtype=np.int32)
@@ -126,18 +127,30 @@ def test_sobel_separable_root_step_every_m():
 
 
 def test_sobel_both_forms_full_image():
-    """8192^2 (the bench's workload): the separable user function and Listing
-    1.5 give the oracle's image bit for bit on row bands incl. both edges"""
+    """8192^2 (the bench's workload): the tuned user function and Listing 1.5
+    give the oracle's whole image bit for bit"""
     c = tma_ctx()
     try:
         R = Cc = 8192
         img = I.image_u8(I.SEED_SOBEL, R, Cc)
         m = S.Matrix.from_numpy(c, img)
-        outs = [S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)(m).to_numpy() for src in (A.SOBEL, A.SOBEL_SEPARABLE)]
-        assert np.array_equal(outs[0], outs[1])
-        for r0 in (0, 4000, R - 64):
-            lo, hi = max(0, r0 - 8), min(R, r0 + 72)
-            ref = O.mapoverlap2d(O.OS_SOBEL, img[lo:hi], 1, O.OB_NEUTRAL, 0)
-            assert np.array_equal(outs[1][r0:r0 + 64], ref[r0 - lo:r0 - lo + 64])
+        ref = O.mapoverlap2d(O.OS_SOBEL, img, 1, O.OB_NEUTRAL, 0)
+        for src in (A.SOBEL, A.SOBEL_TUNED):
+            assert np.array_equal(S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)(m).to_numpy(), ref)
+    finally:
+        c.finalize()
+
+
+@pytest.mark.parametrize("cw,rh,kt", [(16, 4, 2), (8, 8, 1), (4, 16, 1), (8, 4, 1), (16, 2, 2)])
+def test_sobel_tuned_geometries(cw, rh, kt):
+    """the tuned Sobel in the register-block geometries the bench sweeps, on a
+    ragged 1000 x 1500 image with every edge: bit-exact against the oracle"""
+    c = tma_ctx()
+    try:
+        for k, v in (("mo_cw", cw), ("mo_rh", rh), ("mo_kt", kt)):
+            c.set_option(k, v)
+        img = I.image_u8(I.SEED_SOBEL + 11, 1000, 1500)
+        got = S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)(S.Matrix.from_numpy(c, img)).to_numpy()
+        assert np.array_equal(got, O.mapoverlap2d(O.OS_SOBEL, img, 1, O.OB_NEUTRAL, 0))
     finally:
         c.finalize()

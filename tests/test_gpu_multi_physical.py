@@ -99,7 +99,7 @@ def _ipc_worker(rank, world, nid, q):
         from paper_conf_pact_steuwerg13_b200 import skl as S2
         ctx = S2.Context.dist(rank, world, rank, nid)
         img = I2.image_u8(I2.SEED_SOBEL, 301, 272)
-        sob = S2.MapOverlap(ctx, A2.SOBEL_SEPARABLE, S2.U8, S2.U8, 1, S2.NEUTRAL, 0)
+        sob = S2.MapOverlap(ctx, A2.SOBEL_TUNED, S2.U8, S2.U8, 1, S2.NEUTRAL, 0)
         b = sob(sob(S2.Matrix.from_numpy(ctx, img)))
         ref = O2.mapoverlap2d(O2.OS_SOBEL, O2.mapoverlap2d(O2.OS_SOBEL, img, 1, O2.OB_NEUTRAL, 0), 1,
                               O2.OB_NEUTRAL, 0)

@@ -1,8 +1,9 @@
 """MapOverlap probe on one GPU: 8192^2 identity u8 / Sobel (paper form and the
-separable user function) / identity f32 / Gaussian, timed with CUDA events (L2
+tuned user function apps.SOBEL_TUNED) / identity f32 / Gaussian, timed with CUDA events (L2
 flushed), each checked against the oracle on row bands.
 
-  python tools/mo_probe.py [names] [--once]      names: ident_u8,sobel,sobel_sep,ident_f32,gauss
+  python tools/mo_probe.py [names] [--once]      names: ident_u8,sobel,sobel_tuned,ident_f32,gauss,
+                                                 file:<path> (a u8 user function checked as Sobel)
   MO_OPTS="key=value,..."  library options (skl_set_option) for every context
   MO_PER_EVENT=k           k launches between one event pair (time per launch = total / k)
   MO_NOFLUSH=1             no L2 flush before the timed launches
@@ -54,7 +55,7 @@ def timeit(fn, flush, reps=20, warm=3, flush_on=True):
 
 
 def main():
-    names = [a for a in sys.argv[1:] if not a.startswith("--")] or ["ident_u8", "sobel", "sobel_sep", "ident_f32",
+    names = [a for a in sys.argv[1:] if not a.startswith("--")] or ["ident_u8", "sobel", "sobel_tuned", "ident_f32",
                                                                    "gauss"]
     once = "--once" in sys.argv
     flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
@@ -74,9 +75,12 @@ def main():
             mo, img, st, d, b = S.MapOverlap(c, A.IDENT2D_U8, S.U8, S.U8, 1, S.NEUTRAL, 0), img8, O.OS_IDENT, 1, O.OB_NEUTRAL
         elif name == "sobel":
             mo, img, st, d, b = S.MapOverlap(c, A.SOBEL, S.U8, S.U8, 1, S.NEUTRAL, 0), img8, O.OS_SOBEL, 1, O.OB_NEUTRAL
-        elif name == "sobel_sep":
-            mo, img, st, d, b = (S.MapOverlap(c, A.SOBEL_SEPARABLE, S.U8, S.U8, 1, S.NEUTRAL, 0), img8, O.OS_SOBEL, 1,
+        elif name == "sobel_tuned":
+            mo, img, st, d, b = (S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0), img8, O.OS_SOBEL, 1,
                                  O.OB_NEUTRAL)
+        elif name.startswith("file:"):   # a Sobel-semantics u8 user function from a file
+            mo, img, st, d, b = (S.MapOverlap(c, open(name[5:]).read(), S.U8, S.U8, 1, S.NEUTRAL, 0), img8,
+                                 O.OS_SOBEL, 1, O.OB_NEUTRAL)
         elif name == "ident_f32":
             mo, img, st, d, b = (S.MapOverlap(c, A.IDENT2D, S.F32, S.F32, 1, S.NEAREST, 0.0), img32, O.OS_IDENT, 1,
                                  O.OB_NEAREST)
@@ -99,6 +103,8 @@ def main():
             ms = timeit(many, flush, flush_on=os.environ.get("MO_NOFLUSH") != "1") / per
             full = out.to_numpy()
             ok = True
+            if name.startswith("file:"):   # whole image
+                ok = bool(np.array_equal(full, O.mapoverlap2d(st, img, d, b, 0)))
             for r0 in (0, 4000, R - 64):
                 lo, hi = max(0, r0 - 8), min(R, r0 + 72)
                 ref = O.mapoverlap2d(st, img[lo:hi], d, b, 0)

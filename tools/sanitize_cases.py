@@ -158,7 +158,7 @@ def tma_tile_cases(G):
         ctx.set_option("mo_kt", kt)
         n0 = ctx.counter("tma_launches")
         img8 = I.image_u8(5, 70, 144)
-        for src in (A.SOBEL, A.SOBEL_SEPARABLE):
+        for src in (A.SOBEL, A.SOBEL_TUNED):
             sob = S.MapOverlap(ctx, src, S.U8, S.U8, 1, S.NEUTRAL, 0)
             s1 = sob(sob(S.Matrix.from_numpy(ctx, img8)))
             r8 = O.mapoverlap2d(O.OS_SOBEL, O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0), 1, O.OB_NEUTRAL, 0)
