@@ -146,6 +146,12 @@ class Env:
             # several ranks may share a GPU
             share = os.environ.get("SKL_COMM", "") == "shm" or os.environ.get("SKL_BENCH_SHARE_GPU") == "1"
             phys = local_rank % max(1, nvis) if share else local_rank
+            if not share and nvis == 1 and self.world > 1:
+                # the launcher gave every rank only its own GPU: that is device 0
+                # here, and the peers' memory cannot be mapped by CUDA IPC, so the
+                # library's transport is NCCL unless one was chosen
+                phys = 0
+                os.environ.setdefault("SKL_COMM", "nccl")
             if phys >= nvis:
                 raise SystemExit(f"LOCAL_RANK {local_rank} but only {nvis} visible GPU(s)")
             self.G = self.world
