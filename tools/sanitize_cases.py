@@ -163,13 +163,20 @@ def tma_tile_cases(G):
             s1 = sob(sob(S.Matrix.from_numpy(ctx, img8)))
             r8 = O.mapoverlap2d(O.OS_SOBEL, O.mapoverlap2d(O.OS_SOBEL, img8, 1, O.OB_NEUTRAL, 0), 1, O.OB_NEUTRAL, 0)
             assert np.array_equal(s1.to_numpy(), r8)
+        # the tuned Sobel in the bench's 8 x 8 register block
+        for k, v in (("mo_rh", 8), ("mo_cw", 8)):
+            ctx.set_option(k, v)
+        sob = S.MapOverlap(ctx, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)
+        assert np.array_equal(sob(sob(S.Matrix.from_numpy(ctx, img8))).to_numpy(), r8)
+        for k in ("mo_rh", "mo_cw"):
+            ctx.set_option(k, 0)
         imgf = I.image_f32(6, 150, 272)
         ctx.set_option("block_threads", 128)
         gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
         g2 = gau(gau(S.Matrix.from_numpy(ctx, imgf)))
         r1 = O.mapoverlap2d(O.OS_GAUSS5, imgf, 2, O.OB_NEAREST, 0.0)
         assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
-        assert ctx.counter("tma_launches") - n0 == 6 * G
+        assert ctx.counter("tma_launches") - n0 == 8 * G
         n = 3001
         addf = S.Reduce(ctx, A.ADD, S.F32)
         cv = S.Vector(ctx, S.F32, n).set_distribution(S.COPY, 0, addf).fill(0.0)
