@@ -3,7 +3,7 @@
 task statement; DESIGN.md §7 "Measurement").
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-                    [--skeletons all|none|dot,dot_sweep,sobel,sobel_tuned,gauss,gauss_iter,sobel_iter,redist,
+                    [--skeletons all|none|dot,dot_sweep,ident_u8,sobel,sobel_tuned,gauss,gauss_iter,sobel_iter,redist,
                                  scan_i32,scan_f32,lmosem,lmosem_osem,allpairs,mandel_plain]
 
 Headline workload (BASELINE configs[1]): Mandelbrot 4096x3072, a Map over a
@@ -493,6 +493,7 @@ def ncu_traffic(workload: str):
 
 
 SOBEL_TUNED_GEOMETRY = {"mo_rh": 8, "mo_cw": 8, "mo_kt": 1}
+NCU_KEY = {"ident_u8": "ident_u8_stencil"}   # bench line -> profiles/ncu_traffic.json entry
 
 
 def roof_issue(workload: str, ms: float, P: dict, sms: int):
@@ -888,12 +889,18 @@ def bench_skeletons(args, E: Env, P: dict, which):
         for x in (a, b, t):
             x.destroy()
 
-    if "sobel" in which or "gauss" in which or "sobel_tuned" in which:
+    if any(n in which for n in ("sobel", "sobel_tuned", "gauss", "ident_u8")):
         R = Cc = 8192
-        for name in ("sobel", "sobel_tuned", "gauss"):
+        for name in ("ident_u8", "sobel", "sobel_tuned", "gauss"):
             if name not in which:
                 continue
-            if name in ("sobel", "sobel_tuned"):
+            if name == "ident_u8":
+                # the u8 skeleton alone (identity user function, Sobel's image and
+                # boundary): what the staging, tile walk and packed stores cost
+                img = I.image_u8(I.SEED_SOBEL, R, Cc)
+                mo = S.MapOverlap(ctx, A.IDENT2D_U8, S.U8, S.U8, 1, S.NEUTRAL, 0)
+                bpp, okind = 2, O.OS_IDENT
+            elif name in ("sobel", "sobel_tuned"):
                 # Listing 1.5 as printed, and the same operator rewritten by a user
                 # for speed with bit-identical results (apps.SOBEL_TUNED)
                 img = I.image_u8(I.SEED_SOBEL, R, Cc)
@@ -935,14 +942,21 @@ def bench_skeletons(args, E: Env, P: dict, which):
                        else O.mapoverlap2d(okind, img[blo:bhi], 2, O.OB_NEAREST, 0.0))
                 a0 = r0 - blo
                 ok &= bool(np.array_equal(full[r0:r0 + 64], ref[a0:a0 + 64]))
-            desc = {"sobel": "Sobel u8 d=1 NEUTRAL (Listing 1.5 as printed)",
+            desc = {"ident_u8": "identity u8 d=1 NEUTRAL (the skeleton alone)",
+                    "sobel": "Sobel u8 d=1 NEUTRAL (Listing 1.5 as printed)",
                     "sobel_tuned": "Sobel u8 d=1 NEUTRAL, Listing 1.5 rewritten for speed: difference "
                                    "form and an exact sqrt.approx floor (apps.SOBEL_TUNED, bit-identical)",
                     "gauss": "Gaussian 5x5 f32 d=2 NEAREST"}[name]
             res[name] = {"workload": f"{desc} MapOverlap {R}x{Cc}, overlap distribution",
                          **ms_fields(st), "elements_per_s": R * Cc / (ms / 1e3),
-                         "roofline": roof_hbm(bpp * R * Cc, ms, P, name, ngpu=G), "check": "ok" if ok else "FAIL"}
-            res[name]["roofline_issue"] = roof_issue(name, ms, P, sms) if G == 1 else None
+                         "roofline": roof_hbm(bpp * R * Cc, ms, P, NCU_KEY.get(name, name), ngpu=G),
+                         "check": "ok" if ok else "FAIL"}
+            dur = ncu_field(NCU_KEY.get(name, name), "duration_ns")
+            if dur and G == 1:
+                # the same kernel alone (ncu gpu__time_duration of the committed
+                # capture, cold L2): the event-timed step adds the launch / event floor
+                res[name]["roofline"]["kernel_alone_frac"] = round(bpp * R * Cc / (dur * 1e-9) / 1e9 / P["hbm_gbs"], 4)
+            res[name]["roofline_issue"] = roof_issue(NCU_KEY.get(name, name), ms, P, sms) if G == 1 else None
             if name == "gauss":
                 # the binding roof: 25 FMUL + 25 FADD per pixel (no FMA under -fmad=false)
                 res[name]["roofline_alu"] = roof_alu(50.0 * R * Cc, ms, P, sms, G, "50 fp32 ops/pixel (25 mul + 25 add)")
@@ -1263,7 +1277,7 @@ def main():
     P = peaks()
     r = bench_mandelbrot(args, E, P)
     which = [] if args.skeletons == "none" else (
-        ["mandel_plain", "dot", "dot_sweep", "sobel", "sobel_tuned", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32",
+        ["mandel_plain", "dot", "dot_sweep", "ident_u8", "sobel", "sobel_tuned", "gauss", "gauss_iter", "sobel_iter", "redist", "scan_i32",
          "scan_f32", "lmosem", "lmosem_osem", "allpairs"]
         if args.skeletons == "all"
         else args.skeletons.split(","))
