@@ -492,6 +492,18 @@ def ncu_traffic(workload: str):
     return ncu_field(workload, "bytes_per_launch")
 
 
+def try_capture(ctx, fn):
+    """fn's skeleton calls as one CUDA graph (multi-device capture), or None
+    where the context cannot capture (the one-process-per-GPU mode)"""
+    from paper_conf_pact_steuwerg13_b200 import skl as S
+    try:
+        return ctx.capture(fn)
+    except S.SklError as e:
+        if e.name != "UNSUPPORTED":
+            raise
+        return None
+
+
 SOBEL_TUNED_GEOMETRY = {"mo_rh": 8, "mo_cw": 8, "mo_kt": 1}
 NCU_KEY = {"ident_u8": "ident_u8_stencil"}   # bench line -> profiles/ncu_traffic.json entry
 
@@ -674,24 +686,35 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
     for push in (0, 1):
         c4.set_option("halo_push", push)
 
-        def step_it(_):
+        def run10():
             gau(a, out=b)
             for k in range(ITER - 1):
                 gau(b, out=t) if k % 2 == 0 else gau(t, out=b)
 
+        # bytes one step moves: counted while its calls are issued (a graph
+        # replay moves what its capture issued)
+        run10()
         p0, h0 = c4.counter("p2p_bytes"), c4.counter("halo_push_bytes")
+        run10()
+        p_step, h_step = E.sum(c4.counter("p2p_bytes") - p0), E.sum(c4.counter("halo_push_bytes") - h0)
+        graph = try_capture(c4, run10)
+
+        def step_it(_):
+            graph.launch() if graph else run10()
+
         Ki = max(3, K // 4)
         st, _ = timer.run(step_it, Ki, W)
-        reps = Ki + W
         fin = t if (ITER - 1) % 2 == 1 else b
         ok = bool(np.array_equal(fin.to_numpy()[lo:lo + len(sub)][chk], ref[chk]))
         out[f"gauss_iter10_g{G}_{'push' if push else 'refresh'}"] = {
             "workload": f"10 x Gaussian 5x5 on {where}, halos "
                         + ("pushed by the stencil kernel into the neighbours (fused)" if push
                            else "refreshed by copies between iterations"),
-            **ms_fields(st), "p2p_bytes_per_step": E.sum(c4.counter("p2p_bytes") - p0) / reps,
-            "halo_push_bytes_per_step": E.sum(c4.counter("halo_push_bytes") - h0) / reps,
+            "launch": "one CUDA graph per step" if graph else "skeleton calls",
+            **ms_fields(st), "p2p_bytes_per_step": p_step, "halo_push_bytes_per_step": h_step,
             "check": "ok" if ok else "FAIL"}
+        if graph:
+            graph.destroy()
     for x in (a, b, t):
         x.destroy()
     c4.finalize()
@@ -864,10 +887,16 @@ def bench_skeletons(args, E: Env, P: dict, which):
         t = S.Matrix(ctx, dt, R, Cc)
         ITER = 10
 
-        def step(_):
+        def run10():
             stn(a, out=b)
             for k in range(ITER - 1):
                 stn(b, out=t) if k % 2 == 0 else stn(t, out=b)
+
+        run10()
+        graph = try_capture(ctx, run10)
+
+        def step(_):
+            graph.launch() if graph else run10()
 
         st, _ = timer.run(step, max(5, K // 4), W)
         # parity: 64 rows around the device boundary nearest the middle (the
@@ -882,8 +911,11 @@ def bench_skeletons(args, E: Env, P: dict, which):
             r = O.mapoverlap2d(okind, r, dd, ob, nv)
         fin = (t if (ITER - 1) % 2 == 1 else b)
         ok = bool(np.array_equal(fin.to_numpy()[lo + 30:lo + 94], r[30:94]))
+        if graph:
+            graph.destroy()
         res[it_name.replace("_iter", "_iter10")] = {
             "workload": f"10 x {desc} MapOverlap {R}x{Cc}, ping-pong (halo exchange between iterations on >1 GPU)",
+            "launch": "one CUDA graph per step" if graph else "skeleton calls",
             **ms_fields(st), "ms_per_iteration": round(st["median"] / ITER, 4),
             "elements_per_s": ITER * R * Cc / (st["median"] / 1e3), "check": "ok" if ok else "FAIL"}
         for x in (a, b, t):

@@ -330,7 +330,11 @@ skl_status skl_scalar_get(skl_cont* scalar, void* value, size_t bytes);
  * scalar_get, host_data, sync) are not allowed inside.  Containers and
  * skeletons used by a graph must outlive it, keep their sizes and
  * distributions, and have been used once before capture (so that nothing is
- * allocated or compiled while capturing).  One local device only.            */
+ * allocated or compiled while capturing).  Several local devices (one process
+ * driving every GPU, or logical devices): the capture forks from the first
+ * device's stream into the others and joins them at the end, so one launch
+ * replays the whole multi-device sequence, halo exchanges included.  Not in
+ * the one-process-per-GPU mode (skl_init_dist): SKL_ERR_UNSUPPORTED.         */
 typedef struct skl_graph skl_graph;
 skl_status skl_capture_begin(skl_ctx* ctx);
 skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out);

@@ -575,14 +575,49 @@ struct skl_graph {
   cudaGraph_t graph;
   cudaGraphExec_t exec;
 };
+// Several local devices (one process driving every GPU, or logical devices):
+// the capture opens on the first device's stream and forks into the other
+// devices' streams through an event recorded there, so their calls - and the
+// cross-stream barriers between them - are recorded into the same graph; the
+// end joins every stream back before closing.  One graph launch then replays
+// the multi-device sequence (iterated stencils with their halo exchange): the
+// host cost of a call grows with the devices it launches on (~6 us each), more
+// than the GPU time of a stencil iteration on 8 GPUs.  Not in the one-process-
+// per-GPU mode: its device barriers carry epochs that a replay would repeat.
+static std::vector<cudaStream_t> capture_streams(Ctx* c) {
+  std::vector<cudaStream_t> out;
+  for (int g = c->first_local + 1; g < c->first_local + c->nlocal; ++g) {
+    cudaStream_t st = c->D(g).stream;
+    bool seen = st == c->D(c->first_local).stream;
+    for (cudaStream_t o : out) seen = seen || o == st;
+    if (!seen) out.push_back(st);
+  }
+  return out;
+}
+static int stream_device(Ctx* c, cudaStream_t st) {
+  for (int g = c->first_local; g < c->first_local + c->nlocal; ++g)
+    if (c->D(g).stream == st) return c->D(g).phys;
+  return c->D(c->first_local).phys;
+}
 skl_status skl_capture_begin(skl_ctx* ctx) {
   return guard([&] {
     Ctx* c = C(ctx);
-    if (c->nlocal != 1) fail(SKL_ERR_UNSUPPORTED, "graph capture needs exactly one local device");
+    if (c->dist_mode) fail(SKL_ERR_UNSUPPORTED, "graph capture in the one-process-per-GPU mode");
     if (c->capturing) fail(SKL_ERR_INVALID_ARG, "already capturing");
     c->set_device(c->first_local);
-    SKL_CUDA(cudaStreamBeginCapture(c->D(c->first_local).stream, cudaStreamCaptureModeRelaxed));
+    cudaStream_t origin = c->D(c->first_local).stream;
+    SKL_CUDA(cudaStreamBeginCapture(origin, cudaStreamCaptureModeRelaxed));
     c->capturing = true;
+    const auto others = capture_streams(c);
+    if (!others.empty()) {
+      if (!c->cap_fork) SKL_CUDA(cudaEventCreateWithFlags(&c->cap_fork, cudaEventDisableTiming));
+      SKL_CUDA(cudaEventRecord(c->cap_fork, origin));
+      for (cudaStream_t st : others) {
+        SKL_CUDA(cudaSetDevice(stream_device(c, st)));
+        SKL_CUDA(cudaStreamWaitEvent(st, c->cap_fork, 0));
+      }
+      c->set_device(c->first_local);
+    }
   });
 }
 skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out) {
@@ -590,9 +625,20 @@ skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out) {
     Ctx* c = C(ctx);
     if (!c->capturing || !out) fail(SKL_ERR_INVALID_ARG, "not capturing / NULL out");
     c->capturing = false;
+    cudaStream_t origin = c->D(c->first_local).stream;
+    const auto others = capture_streams(c);
+    if (c->cap_join.size() < others.size()) c->cap_join.resize(others.size(), nullptr);
+    for (size_t i = 0; i < others.size(); ++i) {
+      const int dev = stream_device(c, others[i]);
+      SKL_CUDA(cudaSetDevice(dev));
+      if (!c->cap_join[i]) SKL_CUDA(cudaEventCreateWithFlags(&c->cap_join[i], cudaEventDisableTiming));
+      SKL_CUDA(cudaEventRecord(c->cap_join[i], others[i]));
+      c->set_device(c->first_local);
+      SKL_CUDA(cudaStreamWaitEvent(origin, c->cap_join[i], 0));
+    }
     c->set_device(c->first_local);
     cudaGraph_t graph = nullptr;
-    SKL_CUDA(cudaStreamEndCapture(c->D(c->first_local).stream, &graph));
+    SKL_CUDA(cudaStreamEndCapture(origin, &graph));
     cudaGraphExec_t exec = nullptr;
     cudaError_t e = cudaGraphInstantiate(&exec, graph, 0);
     if (e != cudaSuccess) {
@@ -605,9 +651,32 @@ skl_status skl_capture_end(skl_ctx* ctx, skl_graph** out) {
 skl_status skl_graph_launch(skl_graph* gr) {
   return guard([&] {
     if (!gr) fail(SKL_ERR_INVALID_ARG, "NULL graph");
-    gr->ctx->set_device(gr->g);
-    SKL_CUDA(cudaGraphLaunch(gr->exec, gr->ctx->D(gr->g).stream));
-    gr->ctx->n_launch += 1;
+    Ctx* c = gr->ctx;
+    if (c->capturing) fail(SKL_ERR_INVALID_ARG, "graph launch while capturing");
+    cudaStream_t origin = c->D(gr->g).stream;
+    // a multi-device graph runs after the work already queued on every device
+    // stream, and later work on any of them runs after it
+    const auto others = capture_streams(c);
+    if (c->cap_join.size() < others.size()) c->cap_join.resize(others.size(), nullptr);
+    for (size_t i = 0; i < others.size(); ++i) {
+      SKL_CUDA(cudaSetDevice(stream_device(c, others[i])));
+      if (!c->cap_join[i]) SKL_CUDA(cudaEventCreateWithFlags(&c->cap_join[i], cudaEventDisableTiming));
+      SKL_CUDA(cudaEventRecord(c->cap_join[i], others[i]));
+      c->set_device(gr->g);
+      SKL_CUDA(cudaStreamWaitEvent(origin, c->cap_join[i], 0));
+    }
+    c->set_device(gr->g);
+    SKL_CUDA(cudaGraphLaunch(gr->exec, origin));
+    c->n_launch += 1;
+    if (!others.empty()) {
+      if (!c->cap_fork) SKL_CUDA(cudaEventCreateWithFlags(&c->cap_fork, cudaEventDisableTiming));
+      SKL_CUDA(cudaEventRecord(c->cap_fork, origin));
+      for (cudaStream_t st : others) {
+        SKL_CUDA(cudaSetDevice(stream_device(c, st)));
+        SKL_CUDA(cudaStreamWaitEvent(st, c->cap_fork, 0));
+      }
+      c->set_device(gr->g);
+    }
   });
 }
 skl_status skl_graph_destroy(skl_graph* gr) {

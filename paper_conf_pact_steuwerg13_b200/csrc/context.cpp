@@ -223,6 +223,9 @@ void ctx_destroy(Ctx* c) {
     if (d.d2h) cudaStreamDestroy(d.d2h);
     if (d.own) cudaStreamDestroy(d.own);
   }
+  if (c->cap_fork) cudaEventDestroy(c->cap_fork);
+  for (cudaEvent_t e : c->cap_join)
+    if (e) cudaEventDestroy(e);
   delete c;
 }
 

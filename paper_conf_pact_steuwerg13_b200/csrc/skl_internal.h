@@ -114,7 +114,9 @@ struct Ctx {
   int first_local = 0, nlocal = 1;
   bool dist_mode = false;      // one process per GPU, NCCL between ranks
   bool offline = false;        // no devices: compile only (skl_init_offline)
-  bool capturing = false;      // a CUDA graph capture is open on the device stream
+  bool capturing = false;      // a CUDA graph capture is open on the device stream(s)
+  cudaEvent_t cap_fork = nullptr;            // capture fork / join events (several devices)
+  std::vector<cudaEvent_t> cap_join;
   int rank = 0, world = 1;
   void* nccl_comm = nullptr;   // ncclComm_t
   void* shm_comm = nullptr;    // host shared-memory loopback transport (SKL_COMM=shm, tests)

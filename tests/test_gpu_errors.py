@@ -66,11 +66,22 @@ def test_empty_and_mismatch(ctx):
 
 
 def test_capture_rules():
+    """several local devices capture into one graph; nested captures and host
+    reads inside a capture are refused"""
     require_gpu()
     c2 = S.Context(2, devices=[0, 0])
     try:
+        g = c2.capture(lambda: None)
+        g.launch()
+        g.destroy()
+        v = S.Vector.from_numpy(c2, np.ones(100, np.float32)).set_distribution(S.BLOCK)
+        w = S.Map(c2, A.NEG, S.F32, S.F32)(v)          # lives on the devices only
         with pytest.raises(S.SklError) as e:
-            c2.capture(lambda: None)
-        assert e.value.name == "UNSUPPORTED"
+            c2.capture(lambda: c2.capture(lambda: None))
+        assert e.value.name == "INVALID_ARG"
+        with pytest.raises(S.SklError) as e:
+            c2.capture(lambda: w.to_numpy())
+        assert e.value.name == "INVALID_ARG"
+        assert np.array_equal(w.to_numpy(), -np.ones(100, np.float32))   # still usable
     finally:
         c2.finalize()
