@@ -761,7 +761,8 @@ def bench_skeletons(args, E: Env, P: dict, which):
         counts = np.empty((ROWS, COLS), np.uint32)
         counts[order] = o.to_numpy().reshape(ROWS, COLS)
         res["mandel_plain"] = {"workload": "Mandelbrot 4096x3072 MAX 1000, the plain A22 loop (apps.mandelbrot: "
-                                           "escape test every iteration), default Map (256 threads, 4 chunks)",
+                                           "escape test every iteration), the library's default Map for a function with a loop "
+                                           "(warp-interleaved, one element per lane, 256 threads)",
                                **ms_fields(st), "elements_per_s": ROWS * COLS / (st["median"] / 1e3),
                                "_counts": counts}
         for x in (cin, o):

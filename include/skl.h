@@ -137,6 +137,9 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * warp handles elements base + 32 j + l: for customising functions whose cost
  * varies per element, e.g. Mandelbrot; default 0), "map_il_elems" (elements
  * per lane of the interleaved kernel; 0 = one 16-byte chunk's worth; default 0),
+ * "map_auto" (1 = a Map/Zip whose customising source holds a loop - for /
+ * while / do - uses the interleaved kernel with one element per lane unless
+ * map_interleave / map_il_elems say otherwise; default 1),
  * "ap_fast" (Allpairs
  * zip-reduce 128 x 128 tiles for 4-byte inputs with d % 4 == 0; default 1),
  * "ap_hybrid" (1 = when the 128 x 128 tiles leave the last wave less than half

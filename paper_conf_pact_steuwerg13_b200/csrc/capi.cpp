@@ -201,6 +201,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
       c->mo_persist = value ? 1 : 0;
     } else if (k == "mo_ws") {
       c->mo_ws = value ? 1 : 0;
+    } else if (k == "map_auto") {
+      c->map_auto = value ? 1 : 0;
     } else if (k == "map_il_elems") {
       if (value < 0 || value > 64) fail(SKL_ERR_INVALID_ARG, "map_il_elems in [0,64]");
       c->map_il_elems = (int)value;

@@ -233,8 +233,8 @@ void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 
 // Reading A13: with no explicit entry, the customising function is the last
 // top-level function *defined* in the source ("float func(...)",
 // "float sum(...)", "float mult(...)": P:L254).
-std::string detect_entry(const std::string& src) {
-  // strip comments and string/char literals
+// the source without comments and string / char literals
+static std::string strip_source(const std::string& src) {
   std::string s;
   s.reserve(src.size());
   for (size_t i = 0; i < src.size(); ++i) {
@@ -257,6 +257,11 @@ std::string detect_entry(const std::string& src) {
       s += src[i];
     }
   }
+  return s;
+}
+
+std::string detect_entry(const std::string& src) {
+  const std::string s = strip_source(src);
   std::string last;
   int depth = 0;
   for (size_t i = 0; i < s.size(); ++i) {
@@ -339,4 +344,24 @@ bool read_and_clear_bounds_flags(Ctx* ctx) {
   }
   return hit;
 }
+// A customising function whose source holds a loop (for / while / do): its
+// per-element cost may vary (Mandelbrot's escape loop, a ray walk), so a Map /
+// Zip over it defaults to the warp-interleaved kernel with one element per
+// lane (option map_auto; the A22 loop: 1.13 -> 0.94 ms, sweep_r02_mandel_plain.log).
+bool has_loop(const std::string& src) {
+  const std::string s = strip_source(src);
+  for (size_t i = 0; i < s.size();) {
+    if (std::isalpha((unsigned char)s[i]) || s[i] == '_') {
+      size_t j = i;
+      while (j < s.size() && (std::isalnum((unsigned char)s[j]) || s[j] == '_')) ++j;
+      const std::string w = s.substr(i, j - i);
+      if (w == "for" || w == "while" || w == "do") return true;
+      i = j;
+    } else {
+      ++i;
+    }
+  }
+  return false;
+}
+
 }  // namespace skl

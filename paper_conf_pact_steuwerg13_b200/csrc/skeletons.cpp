@@ -100,7 +100,10 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
   // launch geometry is fixed at creation (compiled into the program)
   s->block = ctx->block_threads;
   s->unroll = ctx->map_unroll;
-  s->interleave = ctx->map_interleave != 0;
+  // Map / Zip over a function with a loop: interleaved, one element per lane
+  const bool auto_il = (kind == K_MAP || kind == K_ZIP) && ctx->map_interleave == 0 && ctx->map_auto &&
+                       has_loop(s->user_src);
+  s->interleave = ctx->map_interleave != 0 || auto_il;
   std::string defs = defs_common(ctx, s->entry, s->block);
   std::string body;
   switch (kind) {
@@ -118,7 +121,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       else defs += "#define SKL_TOUT " + tname(ctx, tout) + "\n#define SKL_OUT_VOID 0\n";
       defs += "#define SKL_VEC " + std::to_string(vec) + "\n";
       defs += "#define SKL_UNROLL " + std::to_string(ctx->map_unroll) + "\n";
-      s->ilj = ctx->map_il_elems > 0 ? ctx->map_il_elems : (int)(ctx->map_unroll * vec);
+      s->ilj = ctx->map_il_elems > 0 ? ctx->map_il_elems : (auto_il ? 1 : (int)(ctx->map_unroll * vec));
       defs += "#define SKL_ILJ " + std::to_string(s->ilj) + "\n";
       std::string xp, xa;
       for (size_t k = 0; k < s->extra.size(); ++k) {

@@ -149,6 +149,7 @@ struct Ctx {
   int halo_push = 1;           // MapOverlap stores its border rows into the neighbours' halos
   int map_interleave = 0;      // Map/Zip: warp-interleaved elements (divergent functions)
   int map_il_elems = 0;        //   elements per lane of the interleaved kernel (0 = one chunk)
+  int map_auto = 1;            //   functions with a loop: interleaved, one element per lane
   int xfer_kernel = 1;         // one process: redistribution moves as one batched kernel per device
   int combine_unroll = 0;      // copy(+) -> block folds: 16-byte chunks per thread (0 = 2)
   int combine_peer = 1;        // one process: copy(+) -> block folds straight from the peers' replicas
@@ -311,6 +312,7 @@ void launch(Ctx* ctx, int g, Program* prog, const char* kernel, dim3 grid, dim3 
 int max_smem_optin(Ctx* ctx, int g);
 int occupancy(Ctx* ctx, int g, Program* prog, const char* kernel, int block, size_t smem);
 std::string detect_entry(const std::string& src);
+bool has_loop(const std::string& src);
 std::string kernel_template(const char* name);  // embedded kernels/*.cuh
 
 // ------------------------------------------------------------------ skeletons

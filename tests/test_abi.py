@@ -219,3 +219,22 @@ def test_disk_cache_and_env_defaults(tmp_path, monkeypatch):
     c3 = S.Context.offline()
     assert "#define SKL_BLOCK 128" in S.Map(c3, src, S.F32, S.F32).source()
     c3.finalize()
+
+
+def test_map_over_a_loop_defaults_to_one_element_per_lane(offline):
+    """map_auto: a customising function with a loop (Mandelbrot's A22 escape
+    loop) compiles the interleaved kernel with one element per lane; a
+    straight-line function keeps the 16-byte chunks; comments and strings
+    mentioning loops do not count; map_auto 0 turns it off"""
+    def ilj(src, tin=S.F32, tout=S.F32):
+        s = S.Map(offline, src, tin, tout).source()
+        return int(s.split("#define SKL_ILJ ")[1].split()[0])
+    assert ilj(A.mandelbrot(100), S.F32X2, S.U32) == 1
+    assert ilj("float f(float x){ float s = 0.0f; for (int k = 0; k < 3; ++k) s = s + x; return s; }") == 1
+    assert ilj(A.NEG) > 1
+    assert ilj("float f(float x){ /* for while */ return x + 1.0f; } // do") > 1
+    offline.set_option("map_auto", 0)
+    try:
+        assert ilj(A.mandelbrot(100), S.F32X2, S.U32) > 1
+    finally:
+        offline.set_option("map_auto", 1)

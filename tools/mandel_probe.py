@@ -6,7 +6,8 @@ profiles/sweeps/sweep_r02_mandel_pairs.log - is in the history of
 paper_conf_pact_steuwerg13_b200/apps.py, commit "Mandelbrot user function for
 two neighbouring pixels".)
 
-  MANDEL_CFGS="single,block,unroll,interleave,B[,THxTW];..."   THxTW: pixels stored in
+  MANDEL_CFGS="kind,block,unroll,interleave,B[,THxTW];..."   kind: single (blocktest
+  user function, B iterations per block) or plain (the A22 loop); THxTW: pixels stored in
   TH x TW warp tiles (application-level layout, restored on download)
   MANDEL_ILJ=j     elements per lane of the interleaved Map kernel (map_il_elems)
   MANDEL_EVERY=k   only rows 0, k, 2k, ... (one GPU's share of the image at k GPUs
@@ -71,7 +72,8 @@ def main():
         c.set_option("map_interleave", int(il))
         if os.environ.get("MANDEL_ILJ"):
             c.set_option("map_il_elems", int(os.environ["MANDEL_ILJ"]))
-        m = S.Map(c, A.mandelbrot_blocktest(MAX, int(B)), S.F32X2, S.U32)
+        src = A.mandelbrot(MAX) if kind == "plain" else A.mandelbrot_blocktest(MAX, int(B))
+        m = S.Map(c, src, S.F32X2, S.U32)
         x = S.Matrix(c, S.F32X2, ROWS, COLS).copy_in(np.ascontiguousarray(grid.reshape(-1, 2)[perm]))
         o = S.Matrix(c, S.U32, ROWS, COLS)
         m(x, out=o)
