@@ -316,7 +316,10 @@ def e2e():
         ch, taper = (int(v) for v in (cfg.split(":") + ["1"])[:2])   # "chunks[:taper]"
         c = ctx_with({"xfer_chunks": ch, "xfer_taper": taper, "block_threads": 128, "map_unroll": 1,
                       "map_interleave": 1, "map_il_elems": 1})
-        m = S.Map(c, A.mandelbrot_blocktest(1000, 12), S.F32X2, S.U32)
+        # E2E_FN=cheap: a trivial function of the same types (the pipeline without compute)
+        src = ("uint cheap(float2 c){ return (uint)c.x; }" if os.environ.get("E2E_FN") == "cheap"
+               else A.mandelbrot_blocktest(1000, 12))
+        m = S.Map(c, src, S.F32X2, S.U32)
         e_in = S.Matrix(c, S.F32X2, R, Cc).set_distribution(S.BLOCK)
         e_out = S.Matrix(c, S.U32, R, Cc)
 
