@@ -12,6 +12,7 @@ two neighbouring pixels".)
   MANDEL_ILJ=j     elements per lane of the interleaved Map kernel (map_il_elems)
   MANDEL_EVERY=k   only rows 0, k, 2k, ... (one GPU's share of the image at k GPUs
                    with the bench's round-robin row dealing)
+  MANDEL_ORDER=center  those rows ordered nearest-the-middle first
 """
 import os
 import sys
@@ -52,7 +53,11 @@ def main():
     flush = torch.empty(64 << 20, dtype=torch.float32, device="cuda")
     global ROWS
     every = int(os.environ.get("MANDEL_EVERY", "1"))
-    grid = np.ascontiguousarray(I.mandel_grid(ROWS, COLS)[::every])
+    rows = np.arange(0, ROWS, every)
+    if os.environ.get("MANDEL_ORDER") == "center":
+        # the rows nearest the image's middle (the costliest) first
+        rows = rows[np.argsort(np.abs(rows - (ROWS - 1) / 2.0), kind="stable")]
+    grid = np.ascontiguousarray(I.mandel_grid(ROWS, COLS)[rows])
     ROWS = grid.shape[0]
     ref, tot = O.mandelbrot(grid, MAX)
     cfgs = os.environ.get("MANDEL_CFGS", "single,1024,1,1,12;single,512,1,1,12")
