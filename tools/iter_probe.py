@@ -1,7 +1,8 @@
 """Iterated Gaussian 8192^2 (10 iterations, ping-pong) on G logical devices of
 one GPU, replayed as one CUDA graph: event time per step, to separate the
 multi-device overhead (barriers, halo push, partial waves) from the stencil.
-ITER_G="1,2,4" ITER_PUSH=1 ITER_ONCE=1 (one replay each, for ncu launch lists)"""
+ITER_G="1,2,4" ITER_PUSH=1 ITER_PDL=1 ITER_ROWS=8192 ITER_ONCE=1 (one replay each, for ncu
+launch lists)"""
 import os
 import sys
 
@@ -13,7 +14,8 @@ from paper_conf_pact_steuwerg13_b200 import apps as A  # noqa: E402
 from paper_conf_pact_steuwerg13_b200 import inputs as I  # noqa: E402
 from paper_conf_pact_steuwerg13_b200 import skl as S  # noqa: E402
 
-R = C = 8192
+R = int(os.environ.get("ITER_ROWS", "8192"))
+C = 8192
 img = I.image_f32(I.SEED_GAUSS, R, C)
 once = os.environ.get("ITER_ONCE") == "1"
 for G in (int(g) for g in os.environ.get("ITER_G", "1,2,4").split(",")):
@@ -22,6 +24,7 @@ for G in (int(g) for g in os.environ.get("ITER_G", "1,2,4").split(",")):
     for g, st in enumerate(streams):
         c.set_stream(g, st.cuda_stream)
     c.set_option("halo_push", int(os.environ.get("ITER_PUSH", "1")))
+    c.set_option("pdl", int(os.environ.get("ITER_PDL", "1")))
     c.set_option("block_threads", 128)
     gau = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
     a = S.Matrix.from_numpy(c, img)
@@ -49,7 +52,8 @@ for G in (int(g) for g in os.environ.get("ITER_G", "1,2,4").split(",")):
             e1.record(streams[0])
             torch.cuda.synchronize()
             ts.append(e0.elapsed_time(e1))
-        print(f"G={G} push={os.environ.get('ITER_PUSH', '1')}: {np.median(ts[2:]):.4f} ms per 10 iterations",
+        print(f"G={G} push={os.environ.get('ITER_PUSH', '1')} pdl={os.environ.get('ITER_PDL', '1')} rows={R}: "
+              f"{np.median(ts[2:]):.4f} ms per 10 iterations",
               flush=True)
     g.destroy()
     c.finalize()
