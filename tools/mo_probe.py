@@ -67,7 +67,7 @@ def main():
         torch.cuda.set_stream(s)
         c.set_stream(0, s.cuda_stream)
         o = opts()
-        if name in ("gauss", "ident_f32") and "block_threads" not in o:
+        if (name in ("gauss", "ident_f32") or name.startswith("gfile:")) and "block_threads" not in o:
             o["block_threads"] = 128
         for k, v in o.items():
             c.set_option(k, v)
@@ -81,6 +81,9 @@ def main():
         elif name.startswith("file:"):   # a Sobel-semantics u8 user function from a file
             mo, img, st, d, b = (S.MapOverlap(c, open(name[5:]).read(), S.U8, S.U8, 1, S.NEUTRAL, 0), img8,
                                  O.OS_SOBEL, 1, O.OB_NEUTRAL)
+        elif name.startswith("gfile:"):   # an f32 user function from a file checked as the Gaussian
+            mo, img, st, d, b = (S.MapOverlap(c, open(name[6:]).read(), S.F32, S.F32, 2, S.NEAREST, 0.0), img32,
+                                 O.OS_GAUSS5, 2, O.OB_NEAREST)
         elif name == "ident_f32":
             mo, img, st, d, b = (S.MapOverlap(c, A.IDENT2D, S.F32, S.F32, 1, S.NEAREST, 0.0), img32, O.OS_IDENT, 1,
                                  O.OB_NEAREST)
@@ -103,7 +106,7 @@ def main():
             ms = timeit(many, flush, flush_on=os.environ.get("MO_NOFLUSH") != "1") / per
             full = out.to_numpy()
             ok = True
-            if name.startswith("file:"):   # whole image
+            if name.startswith(("file:", "gfile:")):   # whole image
                 ok = bool(np.array_equal(full, O.mapoverlap2d(st, img, d, b, 0)))
             for r0 in (0, 4000, R - 64):
                 lo, hi = max(0, r0 - 8), min(R, r0 + 72)
