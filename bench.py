@@ -753,7 +753,6 @@ def bench_skeletons(args, E: Env, P: dict, which):
     res = {}
     K, W = max(20, args.steps), max(3, args.warmup)
     G = ctx.ndev
-    one_dev = len(ctx._bench_local) == 1
     sms = torch.cuda.get_device_properties(E.phys[0]).multi_processor_count
 
     if "mandel_plain" in which:
@@ -794,7 +793,7 @@ def bench_skeletons(args, E: Env, P: dict, which):
             floor = None
             # the same step recorded once as a CUDA graph and replayed (removes the
             # host enqueue time that dominates at 2^20 elements)
-            graph = ctx.capture(lambda: step(None)) if one_dev else None
+            graph = try_capture(ctx, lambda: step(None))
             if graph is not None:
                 st, _ = timer.run(lambda _: graph.launch(), K, W)
                 if n == 1 << 20:   # 8 MiB fits L2: also the warm number (no flush)
