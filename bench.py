@@ -541,6 +541,17 @@ def roof_hbm(bytes_per_step: float, ms: float, P: dict, workload: str = None, ng
             "algorithmic_bytes": bytes_per_step}
 
 
+NVLINK_GBS = 900.0   # NVLink 5, per GPU per direction (nominal; no measured figure on this box)
+
+
+def roof_nvlink(bytes_moved: float, ms: float, ngpu: int):
+    """bytes that crossed between GPUs per step / device time, per GPU, against
+    the nominal NVLink 5 rate per direction (every GPU receives its share)"""
+    per = bytes_moved / max(1, ngpu) / (ms / 1e3) / 1e9
+    return {"bound": "nvlink", "achieved": round(per, 1), "peak": NVLINK_GBS, "unit": "GB/s per GPU",
+            "frac": round(per / NVLINK_GBS, 4), "peak_source": "nominal NVLink 5, 900 GB/s per direction"}
+
+
 def roof_alu(ops: float, ms: float, P: dict, sms: int, ngpu: int = 1, note: str = ""):
     peak = sms * FP32_LANES_PER_SM * P["sm_max_mhz"] * 1e6 * ngpu
     fl = ops / (ms / 1e3)
@@ -615,6 +626,8 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
         "workload": f"block -> copy of a 150^3 fp32 Vector (13.5 MB), {where}",
         "ms": round(seg[1], 4), "bytes_moved": moved,
         "roofline": roof_hbm(2 * moved, seg[1], P, ngpu=G if physical else 1), "check": "ok" if ok else "FAIL"}
+    if physical:
+        out["redist_block_to_copy"]["roofline_nvlink"] = roof_nvlink(moved, seg[1], G)
 
     # a10: copy(+) -> block (LM OSEM's c): every device scatters into its own
     # zeroed replica (a void Map with a WRITE extra argument, as the LM OSEM
@@ -654,6 +667,10 @@ def bench_redist(E: Env, K: int, W: int, P: dict) -> dict:
                    "note": "slices exchanged into staging, then folded (combine_peer=0)",
                    "roofline": roof_hbm(2 * moved + traffic, seg0[1], P, ngpu=G if physical else 1)},
         "check": "ok" if ok else "FAIL"}
+    if physical:
+        # the fused fold reads the G - 1 peer replicas' slices over NVLink: the
+        # same bytes the staged path moves
+        out["redist_copy_add_to_block"]["roofline_nvlink"] = roof_nvlink(moved, seg[1], G)
     for x in (w, v, cv, idx):
         x.destroy()
 

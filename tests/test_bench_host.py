@@ -43,6 +43,8 @@ def test_roofline_helpers():
     assert r["achieved"] == 6000.0 and r["peak"] == 12000.0 and r["frac"] == 0.5
     a = bench.roof_alu(148 * 128 * 2e9 * 1e-3, 1.0, P, 148)   # exactly the peak for 1 ms
     assert abs(a["frac"] - 1.0) < 1e-12
+    n = bench.roof_nvlink(8 * 450e6, 1.0, 8)                   # 450 MB into each of 8 GPUs in 1 ms
+    assert n["achieved"] == 450.0 and n["frac"] == 0.5 and n["bound"] == "nvlink"
 
 
 def test_reference_arm_line():
