@@ -1,3 +1,5 @@
+// Measured variant (profiles/sweeps/sweep_r02_gauss_pair.log): two outputs per call in
+// packed fp32x2; needed an experimental skeleton hook (SKL_PAIR_FUNC) that was removed.
 #define SKL_PAIR_FUNC gauss2
 __device__ float skl_pc[2] = {-0.0f, 1.0f};
 __device__ __forceinline__ unsigned long long skl_pk(float a, float b) {

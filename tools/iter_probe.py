@@ -1,7 +1,7 @@
 """Iterated Gaussian 8192^2 (10 iterations, ping-pong) on G logical devices of
 one GPU, replayed as one CUDA graph: event time per step, to separate the
 multi-device overhead (barriers, halo push, partial waves) from the stencil.
-ITER_G="1,2,4" ITER_PUSH=1 ITER_PDL=1 ITER_ROWS=8192 ITER_ONCE=1 (one replay each, for ncu
+ITER_G="1,2,4" ITER_PUSH=1 ITER_ROWS=8192 ITER_ONCE=1 (one replay each, for ncu
 launch lists)"""
 import os
 import sys
@@ -24,7 +24,6 @@ for G in (int(g) for g in os.environ.get("ITER_G", "1,2,4").split(",")):
     for g, st in enumerate(streams):
         c.set_stream(g, st.cuda_stream)
     c.set_option("halo_push", int(os.environ.get("ITER_PUSH", "1")))
-    c.set_option("pdl", int(os.environ.get("ITER_PDL", "1")))
     c.set_option("block_threads", 128)
     gau = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
     a = S.Matrix.from_numpy(c, img)
@@ -52,7 +51,7 @@ for G in (int(g) for g in os.environ.get("ITER_G", "1,2,4").split(",")):
             e1.record(streams[0])
             torch.cuda.synchronize()
             ts.append(e0.elapsed_time(e1))
-        print(f"G={G} push={os.environ.get('ITER_PUSH', '1')} pdl={os.environ.get('ITER_PDL', '1')} rows={R}: "
+        print(f"G={G} push={os.environ.get('ITER_PUSH', '1')} rows={R}: "
               f"{np.median(ts[2:]):.4f} ms per 10 iterations",
               flush=True)
     g.destroy()
