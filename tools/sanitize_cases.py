@@ -189,7 +189,43 @@ def tma_tile_cases(G):
         ctx.finalize()
 
 
+def graph_cases(G):
+    """an iterated Gaussian on G logical devices (one stream each) recorded as ONE
+    multi-device CUDA graph and replayed, halos pushed inside the graph; and a
+    Map over a function with a loop (the interleaved one-element-per-lane default)"""
+    import torch
+    ctx = S.Context(G, devices=[0] * G)
+    streams = [torch.cuda.Stream() for _ in range(G)]
+    for g, st in enumerate(streams):
+        ctx.set_stream(g, st.cuda_stream)
+    gau = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    img = I.image_f32(6, 97, 70)
+    a = S.Matrix.from_numpy(ctx, img)
+    b = S.Matrix(ctx, S.F32, 97, 70)
+    t = S.Matrix(ctx, S.F32, 97, 70)
+
+    def it():
+        gau(a, out=b)
+        gau(b, out=t)
+
+    it()
+    gr = ctx.capture(it)
+    t.fill(0.0)
+    gr.launch()
+    gr.launch()
+    ref = O.mapoverlap2d(O.OS_GAUSS5, O.mapoverlap2d(O.OS_GAUSS5, img, 2, O.OB_NEAREST, 0.0), 2, O.OB_NEAREST, 0.0)
+    assert np.array_equal(t.to_numpy(), ref)
+    gr.destroy()
+    grid = I.mandel_grid(24, 40)
+    m = S.Map(ctx, A.mandelbrot(200), S.F32X2, S.U32)
+    x = S.Matrix(ctx, S.F32X2, 24, 40).set_distribution(S.BLOCK).copy_in(np.ascontiguousarray(grid))
+    got = m(x).to_numpy(np.uint32).reshape(24, 40)
+    assert np.array_equal(got, O.mandelbrot(grid, 200)[0])
+    ctx.finalize()
+
+
 if __name__ == "__main__":
+    graph_cases(3)
     tma_tile_cases(1)
     tma_tile_cases(3)
     one_device({})
