@@ -76,6 +76,32 @@ def test_iterated_stencil_halo_push_across_gpus(phys_ctx):
     assert c.counter("halo_push_bytes") > 0
 
 
+def test_graph_of_iterated_stencil_across_gpus(phys_ctx):
+    """the iterated stencil recorded as one multi-device CUDA graph (kernels and
+    halo pushes on every GPU) and replayed"""
+    c = phys_ctx
+    img = I.image_f32(I.SEED_GAUSS + 1, 1024, 512)
+    gau = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+    a = S.Matrix.from_numpy(c, img)
+    b = S.Matrix(c, S.F32, 1024, 512)
+    t = S.Matrix(c, S.F32, 1024, 512)
+
+    def it():
+        gau(a, out=b)
+        gau(b, out=t)
+        gau(t, out=b)
+
+    it()
+    g = c.capture(it)
+    b.fill(0.0)
+    g.launch()
+    ref = img
+    for _ in range(3):
+        ref = O.mapoverlap2d(O.OS_GAUSS5, ref, 2, O.OB_NEAREST, 0.0)
+    assert np.array_equal(b.to_numpy(), ref)
+    g.destroy()
+
+
 def test_copy_add_to_block_across_gpus(phys_ctx):
     c = phys_ctx
     n = 150 ** 3
