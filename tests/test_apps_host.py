@@ -36,3 +36,14 @@ def test_sobel_tuned_difference_form_is_listing_1_5():
     assert np.array_equal(h0 + 2 * h1 + h2, h_paper)
     assert np.array_equal(v0 + 2 * v1 + v2, v_paper)
     assert "int h = h0 + 2 * h1 + h2, v = v0 + 2 * v1 + v2;" in A.SOBEL_TUNED
+
+
+def test_sobel_tuned_bias_addend_is_or():
+    """apps.SOBEL_TUNED forms the biased m as h*h + (v*v + 0x4B000000): for every
+    m <= 2 * 1020^2 the 32-bit sum has the bits of 0x4B000000 | m (m < 2^23), and
+    that word read as fp32 is 2^23 + m exactly"""
+    m = np.arange(2 * 1020 * 1020 + 1, dtype=np.uint32)
+    biased = (m + np.uint32(0x4B000000)).astype(np.uint32)
+    assert np.array_equal(biased, m | np.uint32(0x4B000000))
+    assert np.array_equal(biased.view(np.float32).astype(np.float64), m.astype(np.float64) + 2.0 ** 23)
+    assert "int m = h * h + (v * v + 0x4B000000);" in A.SOBEL_TUNED

@@ -108,7 +108,7 @@ def test_tma_overlap_distribution_and_halo_push(ndev, dt, tma):
 
 def test_sobel_tuned_root_step_every_m():
     """the square-root step of apps.SOBEL_TUNED, cut out of the user function's
-    own text and run as a Map over m = 0 .. 2^21 - 1 (h^2 + v^2 <= 2,080,800 <
+    own text (the bias added to m as the function adds it) and run as a Map over m = 0 .. 2^21 - 1 (h^2 + v^2 <= 2,080,800 <
     2^21), against numpy's correctly rounded fp32 root: min(255, (int)sqrtf(m))"""
     c = tma_ctx()
     try:
@@ -116,7 +116,10 @@ def test_sobel_tuned_root_step_every_m():
         last = "  return (uchar)__float_as_int(t);\n"
         body = src[src.index("  float k"):src.index(last) + len(last)]
         assert "sqrt.approx" in body and "add.rm" in body
-        fn = "uchar root(int m) {\n" + body + "}"
+        # the function's m carries the 2^23 exponent bias (added as the v*v
+        # multiply-add's addend); here it is added to the plain m
+        assert "int m = h * h + (v * v + 0x4B000000);" in src
+        fn = "uchar root(int m0) {\n  const int m = m0 + 0x4B000000;\n" + body + "}"
         n = 1 << 21
         m = np.arange(n, dtype=np.int32)
         got = S.Map(c, fn, S.I32, S.U8)(S.Vector.from_numpy(c, m)).to_numpy()
