@@ -163,7 +163,9 @@ skl_status skl_set_allocator(skl_ctx* ctx, skl_alloc_fn alloc, skl_free_fn relea
  * units of up to 8 bytes, <= 256 rows; 0 = per-thread cp.async staging;
  * default 1), "mo_kt" (TMA kernel: tiles per block, stacked vertically, all
  * copies issued when the block starts; 1..4, or 0 = automatic: 2 for functions
- * needing >= 64 registers, else 1; default 0),
+ * needing >= 64 registers, else 1; default 0), "mo_full" (2-D MapOverlap: 1 =
+ * threads whose rows and packed stores are all in range run an apply loop
+ * without per-row guards, 0 = never, -1 = with 2+ tiles per block; default -1),
  * "mo_ws" (1 = 2-D MapOverlap tiles are staged by a TMA producer warp into a
  * ring of "mo_ws_stages" shared-memory buffers consumed by the other warps of
  * resident blocks, where TMA can describe the tile: 16-byte aligned rows, staged

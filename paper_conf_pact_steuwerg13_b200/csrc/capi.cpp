@@ -211,6 +211,9 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value) {
     } else if (k == "mo_kt") {
       if (value < 0 || value > 4) fail(SKL_ERR_INVALID_ARG, "mo_kt in [0,4]");
       c->mo_kt = (int)value;
+    } else if (k == "mo_full") {
+      if (value < -1 || value > 1) fail(SKL_ERR_INVALID_ARG, "mo_full in {-1,0,1}");
+      c->mo_full = (int)value;
     } else if (k == "mo_ws_stages") {
       if (value < 2 || value > 8) fail(SKL_ERR_INVALID_ARG, "mo_ws_stages in [2,8]");
       c->mo_ws_stages = (int)value;

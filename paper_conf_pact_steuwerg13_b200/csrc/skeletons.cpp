@@ -58,9 +58,11 @@ std::string defs_common(Ctx* ctx, const std::string& entry, int block) {
 std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
 // rows per thread, tile rows, tiles per block; a block of 2+ tiles marks a heavy
 // function (>= 64 registers), which also gets the unguarded full-tile path
-std::string mo_rows_defs(int rh, int th, int kt) {
+// (option mo_full: 1 / 0 forces it on / off)
+std::string mo_rows_defs(Ctx* ctx, int rh, int th, int kt) {
+  const bool full = ctx->mo_full >= 0 ? ctx->mo_full == 1 : kt > 1;
   return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n#define SKL_MO_KT " +
-         std::to_string(kt) + "\n#define SKL_MO_HEAVY " + (kt > 1 ? "1" : "0") + "\n";
+         std::to_string(kt) + "\n#define SKL_MO_HEAVY " + (full ? "1" : "0") + "\n";
 }
 
 // Scratch buffer per (skeleton, device), grown on demand.
@@ -236,7 +238,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       s->mo_th = th;
       s->mo_kt = ctx->mo_kt > 0 ? ctx->mo_kt : 1;
       s->mo_defs = defs;  // rows and tiles per block go in last (mo_rows_defs): chosen after compiling
-      defs += mo_rows_defs(rh, th, s->mo_kt);
+      defs += mo_rows_defs(ctx, rh, th, s->mo_kt);
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;
@@ -270,7 +272,7 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       s->mo_th = s->mo_th / s->mo_rh * rh;
       s->mo_rh = rh;
       s->mo_kt = kt;
-      s->prog = compile(ctx, s->mo_defs + mo_rows_defs(rh, s->mo_th, kt) + program_source(ctx, body), &log);
+      s->prog = compile(ctx, s->mo_defs + mo_rows_defs(ctx, rh, s->mo_th, kt) + program_source(ctx, body), &log);
     };
     cudaFuncAttributes fa{};
     if (attrs(&fa)) {

@@ -142,6 +142,7 @@ struct Ctx {
   int mo_persist = 0;          // MapOverlap 2-D: persistent blocks, double-buffered tiles
   int mo_tma = 1;              // MapOverlap 2-D: one TMA copy stages a block's tile (skl_mo2d_t)
   int mo_kt = 0;               //   tiles per block (stacked vertically, copies issued up front; 0 = auto)
+  int mo_full = -1;            //   unguarded full-tile apply loop (-1 = auto: with 2+ tiles per block)
   int mo_ws = 0;               // MapOverlap 2-D: TMA producer warp + consumer warps (skl_mo2d_ws)
   int mo_ws_stages = 4;        //   shared-memory ring depth
   int mo_ws_minb = 0;          //   resident blocks per SM the registers must allow (0 = auto)
