@@ -144,15 +144,49 @@ def test_sobel_both_forms_full_image():
         c.finalize()
 
 
-@pytest.mark.parametrize("cw,rh,kt", [(16, 4, 2), (8, 8, 1), (4, 16, 1), (8, 4, 1), (16, 2, 2)])
-def test_sobel_tuned_geometries(cw, rh, kt):
-    """the tuned Sobel in the register-block geometries the bench sweeps, on a
-    ragged 1000 x 1500 image with every edge: bit-exact against the oracle"""
+@pytest.mark.parametrize("cw,rh,kt,full", [(16, 4, 2, -1), (8, 8, 1, -1), (4, 16, 1, -1), (8, 4, 1, -1),
+                                           (16, 2, 2, -1), (8, 16, 1, 1), (8, 32, 1, 1), (8, 8, 2, 0),
+                                           (16, 4, 1, 1)])
+def test_sobel_tuned_geometries(cw, rh, kt, full):
+    """the tuned Sobel in the register-block geometries the bench sweeps (with and
+    without the unguarded full-tile loop, option mo_full), on a ragged 1000 x
+    1500 image with every edge: bit-exact against the oracle"""
     c = tma_ctx()
     try:
-        for k, v in (("mo_cw", cw), ("mo_rh", rh), ("mo_kt", kt)):
+        for k, v in (("mo_cw", cw), ("mo_rh", rh), ("mo_kt", kt), ("mo_full", full)):
             c.set_option(k, v)
         img = I.image_u8(I.SEED_SOBEL + 11, 1000, 1500)
+        got = S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)(S.Matrix.from_numpy(c, img)).to_numpy()
+        assert np.array_equal(got, O.mapoverlap2d(O.OS_SOBEL, img, 1, O.OB_NEUTRAL, 0))
+    finally:
+        c.finalize()
+
+
+@pytest.mark.parametrize("full", [0, 1])
+@pytest.mark.parametrize("shape", [(37, 48), (65, 144), (513, 1008), (70, 1040)])
+def test_full_tile_loop_forced(shape, full):
+    """option mo_full forces the unguarded full-tile loop on (or off) whatever the
+    tiles per block: byte and float stencils on ragged shapes stay bit-exact (the
+    loop runs only for threads whose rows and packed stores are all in range)"""
+    c = tma_ctx(mo_full=full, mo_kt=1)
+    try:
+        x8 = I.image_u8(I.SEED_SOBEL + 3, *shape)
+        for src, kind in ((A.SOBEL, O.OS_SOBEL), (A.SOBEL_TUNED, O.OS_SOBEL), (A.IDENT2D_U8, O.OS_IDENT)):
+            got = S.MapOverlap(c, src, S.U8, S.U8, 1, S.NEUTRAL, 0)(S.Matrix.from_numpy(c, x8)).to_numpy()
+            assert np.array_equal(got, O.mapoverlap2d(kind, x8, 1, O.OB_NEUTRAL, 0)), (src, shape)
+        x32 = I.image_f32(I.SEED_GAUSS + 3, shape[0], shape[1] // 4 * 4)
+        got = S.MapOverlap(c, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)(S.Matrix.from_numpy(c, x32)).to_numpy()
+        assert np.array_equal(got, O.mapoverlap2d(O.OS_GAUSS5, x32, 2, O.OB_NEAREST, 0.0))
+    finally:
+        c.finalize()
+
+
+def test_sobel_tuned_bench_geometry_full_image():
+    """8192^2 in the bench's sobel_tuned configuration (16 x 8 register block, one
+    tile per block, the unguarded full-tile loop): the oracle's whole image"""
+    c = tma_ctx(mo_rh=16, mo_cw=8, mo_kt=1, mo_full=1)
+    try:
+        img = I.image_u8(I.SEED_SOBEL, 8192, 8192)
         got = S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)(S.Matrix.from_numpy(c, img)).to_numpy()
         assert np.array_equal(got, O.mapoverlap2d(O.OS_SOBEL, img, 1, O.OB_NEUTRAL, 0))
     finally:
