@@ -529,11 +529,12 @@ def try_capture(ctx, fn):
         return None
 
 
-# register block of 16 rows x 8 columns per thread, one tile per block, the
-# unguarded full-tile loop: the fastest swept geometry for apps.SOBEL_TUNED
-# (45.1 us; 8 x 8 with guards 49.2, the automatic 4 x 16 / 2 tiles 55 us;
-# profiles/sweeps/sweep_r02_sobel.log r7-r8).  Restored to the defaults after.
-SOBEL_TUNED_GEOMETRY = {"mo_rh": 16, "mo_cw": 8, "mo_kt": 1, "mo_full": 1}
+# register block of 8 rows x 8 columns per thread, one tile per block, the
+# unguarded full-tile loop: the fastest geometry for apps.SOBEL_TUNED in this
+# bench (47.2 us; with per-row guards 49.2, 16 x 8 51.1 - 3.5 waves of blocks -,
+# the automatic 4 x 16 / 2 tiles 55 us; profiles/sweeps/sweep_r02_sobel.log
+# r7-r9).  Restored to the defaults after.
+SOBEL_TUNED_GEOMETRY = {"mo_rh": 8, "mo_cw": 8, "mo_kt": 1, "mo_full": 1}
 MO_DEFAULTS = {"mo_rh": 0, "mo_cw": 0, "mo_kt": 0, "mo_full": -1}
 NCU_KEY = {"ident_u8": "ident_u8_stencil"}   # bench line -> profiles/ncu_traffic.json entry
 
@@ -987,11 +988,15 @@ def bench_skeletons(args, E: Env, P: dict, which):
                 # for speed with bit-identical results (apps.SOBEL_TUNED)
                 img = I.image_u8(I.SEED_SOBEL, R, Cc)
                 if name == "sobel_tuned":
-                    for k, v in SOBEL_TUNED_GEOMETRY.items():
+                    geo = dict(SOBEL_TUNED_GEOMETRY)
+                    # SKL_BENCH_SOBEL_GEOM="mo_rh=8,mo_cw=8,...": another geometry (sweeps)
+                    for kv in filter(None, os.environ.get("SKL_BENCH_SOBEL_GEOM", "").split(",")):
+                        geo[kv.split("=")[0]] = int(kv.split("=")[1])
+                    for k, v in geo.items():
                         ctx.set_option(k, v)
                 mo = S.MapOverlap(ctx, A.SOBEL if name == "sobel" else A.SOBEL_TUNED, S.U8, S.U8, 1,
                                   S.NEUTRAL, 0)
-                for k in SOBEL_TUNED_GEOMETRY:
+                for k in MO_DEFAULTS:
                     ctx.set_option(k, MO_DEFAULTS[k])
                 bpp, okind = 2, O.OS_SOBEL
             else:
@@ -1024,7 +1029,7 @@ def bench_skeletons(args, E: Env, P: dict, which):
             desc = {"ident_u8": "identity u8 d=1 NEUTRAL (the skeleton alone)",
                     "sobel": "Sobel u8 d=1 NEUTRAL (Listing 1.5 as printed)",
                     "sobel_tuned": "Sobel u8 d=1 NEUTRAL, Listing 1.5 rewritten for speed: difference "
-                                   "form and an exact sqrt.approx floor (apps.SOBEL_TUNED, bit-identical); 16 x 8 "
+                                   "form and an exact sqrt.approx floor (apps.SOBEL_TUNED, bit-identical); 8 x 8 "
                                    "outputs per thread, unguarded full-tile loop (mo_full)",
                     "gauss": "Gaussian 5x5 f32 d=2 NEAREST"}[name]
             res[name] = {"workload": f"{desc} MapOverlap {R}x{Cc}, overlap distribution",

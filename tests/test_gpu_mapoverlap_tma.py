@@ -182,9 +182,15 @@ def test_full_tile_loop_forced(shape, full):
 
 
 def test_sobel_tuned_bench_geometry_full_image():
-    """8192^2 in the bench's sobel_tuned configuration (16 x 8 register block, one
-    tile per block, the unguarded full-tile loop): the oracle's whole image"""
-    c = tma_ctx(mo_rh=16, mo_cw=8, mo_kt=1, mo_full=1)
+    """8192^2 in the bench's sobel_tuned configuration (8 x 8 register block, one
+    tile per block, the unguarded full-tile loop; also 16 x 8): the oracle's
+    whole image"""
+    for rh in (8, 16):
+        _sobel_tuned_full_image(rh)
+
+
+def _sobel_tuned_full_image(rh):
+    c = tma_ctx(mo_rh=rh, mo_cw=8, mo_kt=1, mo_full=1)
     try:
         img = I.image_u8(I.SEED_SOBEL, 8192, 8192)
         got = S.MapOverlap(c, A.SOBEL_TUNED, S.U8, S.U8, 1, S.NEUTRAL, 0)(S.Matrix.from_numpy(c, img)).to_numpy()
