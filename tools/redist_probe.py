@@ -1,5 +1,6 @@
 import sys, time, numpy as np, torch
-sys.path.insert(0, '/root/repo')
+import os
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 from paper_conf_pact_steuwerg13_b200 import skl as S, apps as A, inputs as I
 G, nvox = 4, 150**3
 c4 = S.Context(G, devices=[0]*G)
