@@ -102,6 +102,9 @@ skl_status skl_type_size(skl_ctx* ctx, skl_type t, size_t* size);
  *     already loaded in the process, if any - is loaded on first use; the id is
  *     an ncclUniqueId);
  *   "shm": a host shared-memory loopback (tests, several ranks on one GPU).
+ * With world == 1 the context is the one-process form unless SKL_DIST_FORCE=1,
+ * which keeps the multi-process code path and sets up the transport anyway
+ * (tests: NCCL's communicator setup, group calls and teardown on one GPU).
  * Every rank must issue the same sequence of calls (SPMD): host-visible results
  * and redistributions are collective.                                          */
 skl_status skl_init(int ndev, const int* devices, skl_ctx** out);
@@ -179,7 +182,8 @@ skl_status skl_set_option(skl_ctx* ctx, const char* key, long long value);
  * bytes), "halo_push_bytes" (halo bytes stored by MapOverlap kernels directly
  * into neighbour devices' memory), "disk_cache_hits" (cubins loaded from
  * SKL_CACHE_DIR instead of compiled), "tma_launches" (MapOverlap launches of
- * the TMA / warp-specialised kernel).                                          */
+ * the TMA / warp-specialised kernel), "nccl_groups" (NCCL send/recv groups of
+ * redistributions issued), "nccl_comm" (1 when an NCCL communicator exists). */
 skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value);
 const char* skl_last_error(void);
 

@@ -281,6 +281,8 @@ skl_status skl_get_counter(skl_ctx* ctx, const char* key, long long* value) {
     else if (k == "halo_push_bytes") *value = c->pushed;
     else if (k == "disk_cache_hits") *value = c->n_disk_hit;
     else if (k == "tma_launches") *value = c->n_tma;
+    else if (k == "nccl_groups") *value = c->n_nccl_group;           // NCCL send/recv groups issued
+    else if (k == "nccl_comm") *value = c->nccl_comm != nullptr;     // an NCCL communicator exists
     else fail(SKL_ERR_INVALID_ARG, "unknown counter " + k);
   });
 }

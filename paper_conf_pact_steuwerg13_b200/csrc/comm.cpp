@@ -319,6 +319,7 @@ void run_transfers(Ctx* ctx, const std::vector<Transfer>& tr, size_t unit_bytes,
     }
   }
   nccl_check(a->groupEnd(), "ncclGroupEnd");
+  ctx->n_nccl_group++;
   // errors of communication already in flight (peer failure, transport errors)
   if (a->asyncError) {
     ncclResult_t ar = ncclSuccess;

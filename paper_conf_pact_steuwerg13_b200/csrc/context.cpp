@@ -171,7 +171,11 @@ Ctx* ctx_create_dist(int rank, int world, int cuda_device, const void* nccl_id) 
   auto* c = new Ctx();
   init_types(c);
   c->G = world;
-  c->dist_mode = world > 1;
+  // SKL_DIST_FORCE=1: the multi-process code path and its transport even for
+  // one rank, so the transport's setup, group calls and teardown (NCCL's
+  // included, which refuses two ranks on one GPU) run on a one-GPU box
+  const char* force = std::getenv("SKL_DIST_FORCE");
+  c->dist_mode = world > 1 || (force && std::string(force) == "1");
   c->rank = rank;
   c->world = world;
   c->first_local = rank;
@@ -181,7 +185,7 @@ Ctx* ctx_create_dist(int rank, int world, int cuda_device, const void* nccl_id) 
   c->dev[0].phys = cuda_device;
   try {
     init_device(c, c->dev[0]);
-    if (world > 1) nccl_init(c, nccl_id);
+    if (c->dist_mode) nccl_init(c, nccl_id);
   } catch (...) {
     delete c;
     throw;

@@ -170,7 +170,7 @@ struct Ctx {
   // only: 3 / 4 / 6 without look-back (wrong results, the pipeline's ceiling)
   int scan_variant = 6;
   // counters
-  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0}, n_disk_hit{0}, n_tma{0};
+  std::atomic<long long> n_launch{0}, n_compile{0}, n_cache_hit{0}, h2d{0}, d2h{0}, p2p{0}, pushed{0}, n_disk_hit{0}, n_tma{0}, n_nccl_group{0};
   int composed_id = 0;  // names of composed Map chains (lazy fusion)
   // optional caller-provided device allocator (skl_set_allocator)
   void* (*user_alloc)(size_t, int, void*, void*) = nullptr;

@@ -31,6 +31,9 @@ def _worker(rank, world, nid, q, comm="shm"):
         from paper_conf_pact_steuwerg13_b200 import inputs as I
         from paper_conf_pact_steuwerg13_b200 import skl as S
         from paper_conf_pact_steuwerg13_b200.lmosem import ListModeOSEM
+        if comm == "nccl":   # as in the bench: torch (with its own NCCL) in the same process
+            import torch
+            torch.zeros(1, device="cuda")
 
         def rel(a, b):
             a, b = np.asarray(a, np.float64), np.asarray(b, np.float64)
@@ -67,7 +70,7 @@ def _worker(rank, world, nid, q, comm="shm"):
         g2 = gau(gau(S.Matrix.from_numpy(ctx, img)))
         r1 = O.mapoverlap2d(O.OS_GAUSS5, img, 2, O.OB_NEAREST, 0.0)
         assert np.array_equal(g2.to_numpy(), O.mapoverlap2d(O.OS_GAUSS5, r1, 2, O.OB_NEAREST, 0.0))
-        if comm == "ipc":   # the first stencil pushed its border rows into the neighbours' halos
+        if comm == "ipc" and world > 1:   # the first stencil pushed its border rows into the neighbours' halos
             assert ctx.counter("halo_push_bytes") > h0
         # iterated Sobel (ping-pong, halos pushed / exchanged every iteration)
         im8 = I.image_u8(I.SEED_SOBEL, 131, 80)
@@ -99,6 +102,10 @@ def _worker(rank, world, nid, q, comm="shm"):
         ap = S.Allpairs(ctx, A.MULT, S.F32, S.F32, reduce=A.ADD)
         assert np.array_equal(ap(S.Matrix.from_numpy(ctx, a), S.Matrix.from_numpy(ctx, b)).to_numpy(),
                               O.allpairs(O.AP_DOT, a, b))
+        if comm == "nccl":   # the NCCL transport is the one set up
+            assert ctx.counter("nccl_comm") == 1
+            if world == 1:     # no move leaves the rank: no send/recv group is issued
+                assert ctx.counter("nccl_groups") == 0
         ctx.finalize()
         q.put((rank, "ok"))
     except BaseException:   # noqa: BLE001 - reported to the parent
@@ -133,3 +140,33 @@ def test_ranks_on_one_gpu(world, comm):
             if p.is_alive():
                 p.kill()
     assert results == {r: "ok" for r in range(world)}, results
+
+
+@pytest.mark.parametrize("comm", ["nccl", "ipc", "shm"])
+def test_one_rank_forced_dist(comm):
+    """world size 1 with SKL_DIST_FORCE=1: the multi-process code path and its
+    transport on one GPU - for NCCL (which refuses two ranks on one device) the
+    library's libnccl load, ncclGetUniqueId, ncclCommInitRank and ncclCommDestroy
+    next to torch (and torch's NCCL) in the same process - with every oracle
+    check of the multi-rank worker"""
+    require_gpu()
+    sys.path.insert(0, ROOT)
+    from paper_conf_pact_steuwerg13_b200 import skl as S
+    os.environ["SKL_COMM"] = comm
+    os.environ["SKL_DIST_FORCE"] = "1"
+    try:
+        nid = S.Context.nccl_unique_id()
+        ctxm = mp.get_context("spawn")
+        q = ctxm.Queue()
+        p = ctxm.Process(target=_worker, args=(0, 1, nid, q, comm))
+        p.start()
+        try:
+            rank, msg = q.get(timeout=600)
+        finally:
+            p.join(timeout=60)
+            if p.is_alive():
+                p.kill()
+    finally:
+        os.environ.pop("SKL_COMM", None)
+        os.environ.pop("SKL_DIST_FORCE", None)
+    assert (rank, msg) == (0, "ok"), msg
