@@ -1004,7 +1004,15 @@ def bench_skeletons(args, E: Env, P: dict, which):
                 # 128-thread blocks (8 rows x 4 columns per thread, <= 128 registers):
                 # the fastest swept configuration (profiles/sweeps/sweep16-17)
                 ctx.set_option("block_threads", 128)
+                # SKL_BENCH_GAUSS_GEOM="mo_rh=16,mo_kt=1,...": another geometry (sweeps)
+                gkeys = []
+                for kv in filter(None, os.environ.get("SKL_BENCH_GAUSS_GEOM", "").split(",")):
+                    ctx.set_option(kv.split("=")[0], int(kv.split("=")[1]))
+                    gkeys.append(kv.split("=")[0])
                 mo = S.MapOverlap(ctx, A.gaussian5(), S.F32, S.F32, 2, S.NEAREST, 0.0)
+                for k in gkeys:
+                    if k in MO_DEFAULTS:
+                        ctx.set_option(k, MO_DEFAULTS[k])
                 ctx.set_option("block_threads", 256)
                 bpp, okind = 8, O.OS_GAUSS5
             mi = S.Matrix.from_numpy(ctx, img)
