@@ -529,12 +529,12 @@ def try_capture(ctx, fn):
         return None
 
 
-# register block of 8 rows x 8 columns per thread, one tile per block, the
-# unguarded full-tile loop: the fastest geometry for apps.SOBEL_TUNED in this
-# bench (47.2 us; with per-row guards 49.2, 16 x 8 51.1 - 3.5 waves of blocks -,
-# the automatic 4 x 16 / 2 tiles 55 us; profiles/sweeps/sweep_r02_sobel.log
-# r7-r9).  Restored to the defaults after.
-SOBEL_TUNED_GEOMETRY = {"mo_rh": 8, "mo_cw": 8, "mo_kt": 1, "mo_full": 1}
+# apps.SOBEL_TUNED runs in the library's automatic geometry, which for a heavy
+# function on a byte image is 8 x 8 outputs per thread, one tile per block and
+# the unguarded full-tile loop (47.1 us; 16 x 8: 51.1 - 3.5 waves of blocks -,
+# the earlier automatic 4 x 16 / 2 tiles 51.2; profiles/sweeps/sweep_r02_sobel.log
+# r7-r10).  SKL_BENCH_SOBEL_GEOM overrides it for sweeps.
+SOBEL_TUNED_GEOMETRY = {}
 MO_DEFAULTS = {"mo_rh": 0, "mo_cw": 0, "mo_kt": 0, "mo_full": -1}
 NCU_KEY = {"ident_u8": "ident_u8_stencil"}   # bench line -> profiles/ncu_traffic.json entry
 
@@ -987,6 +987,10 @@ def bench_skeletons(args, E: Env, P: dict, which):
                 # Listing 1.5 as printed, and the same operator rewritten by a user
                 # for speed with bit-identical results (apps.SOBEL_TUNED)
                 img = I.image_u8(I.SEED_SOBEL, R, Cc)
+                if name == "sobel":
+                    # SKL_BENCH_SOBEL_PAPER_GEOM="mo_rh=8,...": a geometry for Listing 1.5 (sweeps)
+                    for kv in filter(None, os.environ.get("SKL_BENCH_SOBEL_PAPER_GEOM", "").split(",")):
+                        ctx.set_option(kv.split("=")[0], int(kv.split("=")[1]))
                 if name == "sobel_tuned":
                     geo = dict(SOBEL_TUNED_GEOMETRY)
                     # SKL_BENCH_SOBEL_GEOM="mo_rh=8,mo_cw=8,...": another geometry (sweeps)
@@ -1037,8 +1041,8 @@ def bench_skeletons(args, E: Env, P: dict, which):
             desc = {"ident_u8": "identity u8 d=1 NEUTRAL (the skeleton alone)",
                     "sobel": "Sobel u8 d=1 NEUTRAL (Listing 1.5 as printed)",
                     "sobel_tuned": "Sobel u8 d=1 NEUTRAL, Listing 1.5 rewritten for speed: difference "
-                                   "form and an exact sqrt.approx floor (apps.SOBEL_TUNED, bit-identical); 8 x 8 "
-                                   "outputs per thread, unguarded full-tile loop (mo_full)",
+                                   "form and an exact sqrt.approx floor (apps.SOBEL_TUNED, bit-identical), the "
+                                   "library's automatic geometry",
                     "gauss": "Gaussian 5x5 f32 d=2 NEAREST"}[name]
             res[name] = {"workload": f"{desc} MapOverlap {R}x{Cc}, overlap distribution",
                          **ms_fields(st), "elements_per_s": R * Cc / (ms / 1e3),

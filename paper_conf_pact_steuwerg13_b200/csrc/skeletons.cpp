@@ -12,6 +12,7 @@
 //   Reduce        ordered fold of the G device partials
 //   Scan          device totals -> carry-in of the later devices
 //   MapOverlap    overlap halo refresh before the stencil
+#include <functional>
 #include <algorithm>
 #include <cstdio>
 #include <numeric>
@@ -59,8 +60,8 @@ std::string tname(Ctx* ctx, int t) { return ctx->type(t).name; }
 // rows per thread, tile rows, tiles per block; a block of 2+ tiles marks a heavy
 // function (>= 64 registers), which also gets the unguarded full-tile path
 // (option mo_full: 1 / 0 forces it on / off)
-std::string mo_rows_defs(Ctx* ctx, int rh, int th, int kt) {
-  const bool full = ctx->mo_full >= 0 ? ctx->mo_full == 1 : kt > 1;
+std::string mo_rows_defs(Ctx* ctx, int rh, int th, int kt, int force_full = -1) {
+  const bool full = force_full >= 0 ? force_full == 1 : ctx->mo_full >= 0 ? ctx->mo_full == 1 : kt > 1;
   return "#define SKL_RH " + std::to_string(rh) + "\n#define SKL_TH " + std::to_string(th) + "\n#define SKL_MO_KT " +
          std::to_string(kt) + "\n#define SKL_MO_HEAVY " + (full ? "1" : "0") + "\n";
 }
@@ -87,6 +88,8 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
                   int tout, const int* extra, int nextra, int d, int boundary, const void* neutral) {
   if (!src) fail(SKL_ERR_INVALID_ARG, "customising function source is NULL");
   auto s = std::make_unique<Skel>();
+  std::function<std::string(int, int)> mo_geo;  // MapOverlap: register-block defines
+  std::string mo_tail;                          // MapOverlap: defines after the geometry
   s->ctx = ctx;
   s->kind = kind;
   s->user_src = src;
@@ -203,27 +206,39 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       if (ctx->mo_cw > 0) cw = ctx->mo_cw;  // register block per thread (tuning knobs)
       if (ctx->mo_rh > 0) rh = ctx->mo_rh;
       s->mo_auto_rh = ctx->mo_rh == 0 && si == 1;
-      if ((cw * (int)si) % 16 != 0 && (16 % (cw * (int)si)) != 0)
-        fail(SKL_ERR_INVALID_ARG, "mo_cw x element size must divide or be a multiple of 16 bytes");
+      // byte images, geometry fully automatic: a heavy function gets the 8 x 8
+      // register block below (chosen after compiling)
+      s->mo_auto_byte = si == 1 && ctx->mo_rh == 0 && ctx->mo_cw == 0 && ctx->mo_kt == 0 && ctx->mo_full < 0;
       const int nthr = ctx->block_threads;
-      const int tw = 32 * cw;
-      const int rows_thr = nthr / 32;
-      int th = rows_thr * rh;
-      while (rh > 1 && (size_t)(th + 2 * d) * (size_t)(tw + 2 * A) * si > 44 * 1024) {
-        rh /= 2;
-        th = rows_thr * rh;
-      }
-      s->mo_tw = tw;
-      s->mo_a = A;
-      s->mo_pitch = tw + 2 * A;
-      s->mo_cw = cw;
-      defs += "#define SKL_TIN " + tname(ctx, tin) + "\n#define SKL_TOUT " + tname(ctx, tout) + "\n";
-      defs += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(boundary) + "\n";
-      defs += "#define SKL_A " + std::to_string(A) + "\n";
-      defs += "#define SKL_PITCH " + std::to_string(tw + 2 * A) + "\n";
-      defs += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_CW " + std::to_string(cw) + "\n";
-      defs += "#define SKL_OUTB " + std::to_string((size_t)cw * so) + "\n#define SKL_SO " + std::to_string(so) + "\n";
-      defs += "#define SKL_MO1D 0\n";
+      const std::string pre = defs;
+      // the register-block geometry's defines (and the skeleton's copy of it)
+      mo_geo = [&, pre, nthr, A, si, so, tin, tout, d, boundary](int cw_, int rh_) {
+        if ((cw_ * (int)si) % 16 != 0 && (16 % (cw_ * (int)si)) != 0)
+          fail(SKL_ERR_INVALID_ARG, "mo_cw x element size must divide or be a multiple of 16 bytes");
+        const int tw = 32 * cw_;
+        const int rows_thr = nthr / 32;
+        int th = rows_thr * rh_;
+        while (rh_ > 1 && (size_t)(th + 2 * d) * (size_t)(tw + 2 * A) * si > 44 * 1024) {
+          rh_ /= 2;
+          th = rows_thr * rh_;
+        }
+        s->mo_tw = tw;
+        s->mo_a = A;
+        s->mo_pitch = tw + 2 * A;
+        s->mo_cw = cw_;
+        s->mo_rh = rh_;
+        s->mo_th = th;
+        std::string g = pre;
+        g += "#define SKL_TIN " + tname(ctx, tin) + "\n#define SKL_TOUT " + tname(ctx, tout) + "\n";
+        g += "#define SKL_D " + std::to_string(d) + "\n#define SKL_BOUNDARY " + std::to_string(boundary) + "\n";
+        g += "#define SKL_A " + std::to_string(A) + "\n";
+        g += "#define SKL_PITCH " + std::to_string(tw + 2 * A) + "\n";
+        g += "#define SKL_TW " + std::to_string(tw) + "\n#define SKL_CW " + std::to_string(cw_) + "\n";
+        g += "#define SKL_OUTB " + std::to_string((size_t)cw_ * so) + "\n#define SKL_SO " + std::to_string(so) + "\n";
+        g += "#define SKL_MO1D 0\n";
+        return g;
+      };
+      defs = mo_geo(cw, rh);
       // resident blocks per SM the register allocation must allow (default: 64
       // registers per thread for byte images - 87 registers halved the Sobel
       // occupancy and cost 30 % - and 128 for wider elements)
@@ -234,11 +249,10 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       const int wsminb =
           ctx->mo_ws_minb > 0 ? ctx->mo_ws_minb : std::max(1, 65536 / ((nthr + 32) * (si >= 4 ? 128 : 64)));
       defs += "#define SKL_WS_MINB " + std::to_string(wsminb) + "\n";
-      s->mo_rh = rh;
-      s->mo_th = th;
+      mo_tail = "#define SKL_MO_MINB " + std::to_string(minb) + "\n#define SKL_WS_MINB " + std::to_string(wsminb) + "\n";
       s->mo_kt = ctx->mo_kt > 0 ? ctx->mo_kt : 1;
       s->mo_defs = defs;  // rows and tiles per block go in last (mo_rows_defs): chosen after compiling
-      defs += mo_rows_defs(ctx, rh, th, s->mo_kt);
+      defs += mo_rows_defs(ctx, s->mo_rh, s->mo_th, s->mo_kt);
       body = user + kernel_template("common.cuh") + kernel_template("mapoverlap.cuh");
       // 1-D variant (vector containers), compiled lazily in run_mapoverlap
       break;
@@ -275,7 +289,16 @@ Skel* skel_create(Ctx* ctx, int kind, const char* src, const char* entry, int ti
       s->prog = compile(ctx, s->mo_defs + mo_rows_defs(ctx, rh, s->mo_th, kt) + program_source(ctx, body), &log);
     };
     cudaFuncAttributes fa{};
-    if (attrs(&fa)) {
+    if (attrs(&fa) && s->mo_auto_byte && fa.numRegs >= 64) {
+      //  * byte images with a heavy function (every option automatic): 8 x 8
+      //    outputs per thread, one tile per block, the unguarded full-tile loop
+      //    (bench context, 8192^2: Listing 1.5 67.6 -> 65.6 us, the tuned Sobel
+      //    51.2 -> 47.1 us; profiles/sweeps/sweep_r02_sobel.log r10)
+      s->mo_defs = mo_geo(8, 8) + mo_tail;
+      s->mo_kt = 1;
+      s->prog = compile(ctx, s->mo_defs + mo_rows_defs(ctx, s->mo_rh, s->mo_th, 1, 1) + program_source(ctx, body),
+                        &log);
+    } else if (attrs(&fa)) {
       const bool heavy = fa.numRegs >= 64;
       if (ctx->mo_kt == 0 && heavy) {
         recompile(s->mo_rh, 2);

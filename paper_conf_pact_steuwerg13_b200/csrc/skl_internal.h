@@ -340,6 +340,7 @@ struct Skel {
   int mo_tw = 0, mo_th = 0, mo_pitch = 0, mo_a = 0, mo_rh = 0, mo_cw = 0;
   int mo_kt = 1;            // TMA tile kernel: tiles per block (SKL_MO_KT)
   bool mo_auto_rh = false;  // byte images: row count chosen after compiling (spill check)
+  bool mo_auto_byte = false;  // byte images, geometry automatic: 8 x 8 block for heavy functions
   std::string mo_defs;      // program defines without the row count
   bool mo_1d = false;
   int scan_ch = 0;   // Scan: 16-byte chunks per thread (0 = generic path)
