@@ -32,6 +32,12 @@ median over steps (mean and min reported too); max over ranks.  nvidia-smi
 clocks are sampled during the timed region.  Exit status is non-zero when a
 parity check fails or a section raises or times out (the line is printed first).
 
+Sweep hooks (unset in a normal run): SKL_BENCH_SOBEL_PAPER_GEOM /
+SKL_BENCH_SOBEL_GEOM / SKL_BENCH_GAUSS_GEOM="key=value,..." set library options
+(register-block geometry) for the Listing 1.5 / tuned Sobel / Gaussian lines;
+every line runs in the library's automatic geometry otherwise (the Gaussian at
+128-thread blocks).
+
 --impl reference: the CPU oracle (oracle/, plain single-threaded C++) timed on
 this host on a bounded sample of the same workload (the paper's method has no
 reference code to install: DESIGN.md §7 "Reference arm").
